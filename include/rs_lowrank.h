@@ -1,0 +1,144 @@
+/*
+ * rs_lowrank.h -- C ABI of the B200 (sm_100a) random-sampling rank-k approximation
+ *
+ *     A P ~= Q R,   A: m x n,  Q: m x k (orthonormal columns),  R: k x n,  P: column permutation
+ *
+ * following Mary, Yamazaki, Kurzak, Luszczek, Tomov, Dongarra, "Performance of random sampling
+ * for computing low-rank approximations of a dense matrix on GPUs", SC15 (PAPER.md, cited as
+ * P:L<lines>).  Eq. (1); the algorithm is Fig. 2:
+ *
+ *   Step 1  sample        B := Omega A,  Omega l x m Gaussian, l = k + p
+ *           power_iterate q x { B := QR(B); C := B A^T; C := QR(C); B := C A }  (Fig. 2(a))
+ *   Step 2  pivot         [Q^, R^, P] := truncated QRCP(B), T := R^_{1:k}^{-1} R^_{k+1:n}
+ *   Step 3  factor        [Q, Rbar] := QR(A P_{1:k}),  R := Rbar [I_k T]
+ *
+ * QR(.) of the short-wide B (l x n) and C (l x m) and of the tall A P_{1:k} is CholQR with one
+ * full re-orthogonalisation ("CholQR2").  Omega is generated on the
+ * device by Philox4x32-10 + the RS-BM32 Gaussian transform inside the GEMM tile
+ * loader and is never stored.
+ *
+ * CONVENTIONS
+ *  - All matrices are FP64, column-major (LAPACK/MAGMA convention), 0-based indices.
+ *  - All matrix pointers passed to sample/power_iterate/pivot/factor are DEVICE pointers on the
+ *    device that was current at rs_lowrank_create; they must be 16-byte aligned and every
+ *    leading dimension must be even (TMA: 16-byte row pitch).
+ *  - Multi-GPU (1-D block-row distribution): rank r passes its row block A(r)
+ *    (m_local rows starting at global row row_offset).  Omega is keyed by GLOBAL row index, so
+ *    the result does not depend on the partition (up to summation order).  B and R are
+ *    replicated on every rank, Q is row-distributed like A.
+ *  - Every call enqueues work on the handle's CUDA stream.  sample and power_iterate do not
+ *    synchronise; pivot and factor synchronise the stream before returning so that device-side
+ *    failures (Cholesky breakdown, zero pivot norm) can be reported (cuSOLVER devInfo style).
+ *  - Ownership: the caller owns A, Q, R, perm and the workspace (allocate them with any device
+ *    allocator); the library never frees them.  A must stay unmodified from sample through
+ *    factor (it is re-read by power_iterate and factor).  The handle owns only host state.
+ *  - Call order: create -> sample -> power_iterate? -> pivot -> factor -> destroy.  sample may
+ *    be called again at any time (fresh pipeline).  Out-of-order calls return RS_ERR_BAD_STATE.
+ *  - No exceptions cross the ABI; rs_lowrank_last_error returns a static per-handle message.
+ */
+#ifndef RS_LOWRANK_H_
+#define RS_LOWRANK_H_
+
+#include <stddef.h>
+#include <stdint.h>
+
+#if defined(__GNUC__)
+#define RS_API __attribute__((visibility("default")))
+#else
+#define RS_API
+#endif
+
+#ifdef __cplusplus
+extern "C" {
+#endif
+
+typedef struct rs_lowrank_s* rs_lowrank_t;
+
+typedef enum {
+  RS_OK = 0,
+  RS_ERR_INVALID_ARG = 1,    /* bad size / pointer alignment / leading dimension */
+  RS_ERR_BAD_STATE = 2,      /* call out of order */
+  RS_ERR_CUDA = 3,           /* CUDA runtime error (message in last_error) */
+  RS_ERR_NCCL = 4,           /* NCCL error */
+  RS_ERR_NOT_SPD = 5,        /* CholQR breakdown: Gram matrix not numerically SPD (see get_info) */
+  RS_ERR_RANK_DEFICIENT = 6, /* QRCP found a zero residual norm before k steps (see get_info) */
+  RS_ERR_WORKSPACE = 7,      /* workspace too small */
+  RS_ERR_UNSUPPORTED = 8     /* device is not sm_100 / size outside the supported range */
+} rs_status_t;
+
+/* Bytes of device workspace rs_lowrank_create needs for these sizes (no device access). */
+RS_API size_t rs_lowrank_workspace_bytes(int64_t m_local, int64_t n, int32_t k, int32_t p, int32_t nranks);
+
+/* Create a handle.
+ *  m_global, m_local, row_offset : global rows, this rank's rows, first global row of this rank
+ *  n, k, p                       : columns, target rank, oversampling (l = k + p);
+ *                                  require 1 <= k <= l <= min(m_global, n), l <= 512
+ *  seed                          : Philox key (64 bit) of Omega
+ *  workspace, workspace_bytes    : device buffer of at least rs_lowrank_workspace_bytes(...)
+ *  cuda_stream                   : cudaStream_t (NULL = legacy default stream)
+ *  nccl_comm                     : ncclComm_t spanning all ranks, or NULL for a single GPU     */
+RS_API rs_status_t rs_lowrank_create(rs_lowrank_t* h, int64_t m_global, int64_t m_local, int64_t row_offset, int64_t n,
+                              int32_t k, int32_t p, uint64_t seed, void* workspace, size_t workspace_bytes,
+                              void* cuda_stream, void* nccl_comm);
+
+/* Step 1: B := Omega A  (l x n, summed over ranks; Fig. 2(b) lines 2-3).  A: m_local x n, lda. */
+RS_API rs_status_t rs_lowrank_sample(rs_lowrank_t h, const double* A, int64_t lda);
+
+/* q passes of the power method with CholQR2 re-orthonormalisation of B and C (Fig. 2(a)).
+ * q = 0 is a no-op.  No orthonormalisation after the last B := C A.                         */
+RS_API rs_status_t rs_lowrank_power_iterate(rs_lowrank_t h, const double* A, int64_t lda, int32_t q);
+
+/* Step 2: truncated QRCP of B (k steps, largest residual column norm, ties -> lowest index)
+ * and T := R^_{1:k}^{-1} R^_{k+1:n}.  perm (device int64[n], may be NULL) receives P:
+ * perm[0..k) are the pivot columns, perm[k..n) the rest in LAPACK swap order.  Synchronises. */
+RS_API rs_status_t rs_lowrank_pivot(rs_lowrank_t h, int64_t* perm);
+
+/* Step 3: Q := orth(A(:, P_{1:k})) by CholQR2 (Q: m_local x k, ldq >= m_local, even) and
+ * R := Rbar [I_k T] (k x n, ldr >= k, even, columns in pivot order; replicated).  Synchronises. */
+RS_API rs_status_t rs_lowrank_factor(rs_lowrank_t h, const double* A, int64_t lda, double* Q, int64_t ldq, double* R,
+                              int64_t ldr);
+
+/* End-to-end call with HOST buffers: copies A (m_local x n, lda, host) to the device buffer
+ * A_dev (ld_dev), runs sample -> power_iterate(q) -> pivot -> factor, and copies perm (int64[n]),
+ * Q (m_local x k, ldq) and R (k x n, ldr) back to host memory.  Host buffers should be pinned
+ * for full PCIe bandwidth.  Q_dev (m_local x k, even ld_qdev) and R_dev (k x n, even ld_rdev)
+ * are device scratch for the outputs.  Synchronises.                                          */
+RS_API rs_status_t rs_lowrank_run_host(rs_lowrank_t h, const double* A_host, int64_t lda, double* A_dev, int64_t ld_dev,
+                                int32_t q, int64_t* perm_host, double* Q_host, int64_t ldq, double* R_host,
+                                int64_t ldr, double* Q_dev, int64_t ld_qdev, double* R_dev, int64_t ld_rdev);
+
+RS_API rs_status_t rs_lowrank_destroy(rs_lowrank_t h);
+
+/* ---- accessors (tests / bench) ---- */
+/* B (l x n, device, column-major, ldb >= l) after sample / power_iterate.                   */
+RS_API rs_status_t rs_lowrank_get_sample(rs_lowrank_t h, double* B, int64_t ldb);
+/* Replace B (l x n, device) -- e.g. the Omega = I special case (B := A, l = m).             */
+RS_API rs_status_t rs_lowrank_set_sample(rs_lowrank_t h, const double* B, int64_t ldb);
+/* After pivot: T (k x (n-k), ldt >= k) and R^ (k x n in pivot order, ldrh >= k), device;
+ * gaps (host double[k], may be NULL): per-step relative gap (best - second)/best of norms.    */
+RS_API rs_status_t rs_lowrank_get_pivot_data(rs_lowrank_t h, double* T, int64_t ldt, double* Rhat, int64_t ldrh,
+                                      double* gaps_host);
+/* Materialise Omega[0:l, j0:j0+ncols) (global columns) into out (device, l x ncols, ldo >= l):
+ * the exact values the fused sampling GEMM generates.                                        */
+RS_API rs_status_t rs_lowrank_omega(rs_lowrank_t h, int64_t j0, int64_t ncols, double* out, int64_t ldo);
+/* info[0] = status code of the first device-detected failure (0 if none), info[1] = 1-based
+ * failing Cholesky column / QRCP step.  Synchronises.                                        */
+RS_API rs_status_t rs_lowrank_get_info(rs_lowrank_t h, int64_t* info);
+/* Per-kernel-class device time (ms, CUDA events on the handle's stream) accumulated while
+ * profiling is enabled.  names: "gemm_sample", "gemm_power_c", "gemm_power_b", "gram",
+ * "apply", "chol", "qrcp", "factor", "reduce", "comm", "other".                              */
+RS_API rs_status_t rs_lowrank_set_profiling(rs_lowrank_t h, int32_t enable);
+RS_API rs_status_t rs_lowrank_get_profile(rs_lowrank_t h, const char* name, double* ms, int64_t* launches,
+                                   double* flops);
+RS_API rs_status_t rs_lowrank_reset_profile(rs_lowrank_t h);
+RS_API const char* rs_lowrank_last_error(rs_lowrank_t h);
+
+/* ---- NCCL plumbing (the harness exchanges the id with torch.distributed) ---- */
+RS_API rs_status_t rs_comm_get_unique_id(char id_out[128]);
+RS_API rs_status_t rs_comm_init(void** comm, int32_t nranks, const char id[128], int32_t rank);
+RS_API rs_status_t rs_comm_destroy(void* comm);
+
+#ifdef __cplusplus
+}
+#endif
+#endif /* RS_LOWRANK_H_ */

@@ -1,0 +1,178 @@
+// Host launchers for the FP64 DMMA GEMM families (tensor-map encoding, tile/split choice).
+#include <cstdio>
+#include <mutex>
+
+#include "gemm_f64.cuh"
+#include "internal.h"
+
+namespace rs {
+
+namespace {
+
+using EncodeTiledFn = CUresult (*)(CUtensorMap*, CUtensorMapDataType, cuuint32_t, void*, const cuuint64_t*,
+                                   const cuuint64_t*, const cuuint32_t*, const cuuint32_t*, CUtensorMapInterleave,
+                                   CUtensorMapSwizzle, CUtensorMapL2promotion, CUtensorMapFloatOOBfill);
+
+EncodeTiledFn get_encode() {
+  static EncodeTiledFn fn = nullptr;
+  static std::once_flag once;
+  std::call_once(once, [] {
+    void* p = nullptr;
+    cudaDriverEntryPointQueryResult q;
+    if (cudaGetDriverEntryPoint("cuTensorMapEncodeTiled", &p, cudaEnableDefault, &q) == cudaSuccess &&
+        q == cudaDriverEntryPointSuccess)
+      fn = reinterpret_cast<EncodeTiledFn>(p);
+  });
+  return fn;
+}
+
+// 2-D FP64 tensor map, 128B swizzle, OOB -> zero.  box0 must be 16 (128 bytes).
+bool make_tmap(CUtensorMap* m, const View2D& v, uint32_t box0, uint32_t box1) {
+  EncodeTiledFn enc = get_encode();
+  if (!enc) return false;
+  cuuint64_t dims[2] = {static_cast<cuuint64_t>(v.dim0), static_cast<cuuint64_t>(v.dim1)};
+  cuuint64_t strides[1] = {static_cast<cuuint64_t>(v.ld) * 8};
+  cuuint32_t box[2] = {box0, box1};
+  cuuint32_t estr[2] = {1, 1};
+  CUresult r = enc(m, CU_TENSOR_MAP_DATA_TYPE_FLOAT64, 2, const_cast<double*>(v.base), dims, strides, box, estr,
+                   CU_TENSOR_MAP_INTERLEAVE_NONE, CU_TENSOR_MAP_SWIZZLE_128B, CU_TENSOR_MAP_L2_PROMOTION_L2_256B,
+                   CU_TENSOR_MAP_FLOAT_OOB_FILL_NONE);
+  return r == CUDA_SUCCESS;
+}
+
+template <int MFW, bool PHILOX>
+cudaError_t launch_kc_t(cudaStream_t st, dim3 grid, const CUtensorMap& tR, const CUtensorMap& tL, const GemmArgs& a) {
+  constexpr int smem = KCSmem<MFW, PHILOX>::TOTAL;
+  static bool attr_set = false;  // per-instantiation; races are benign (idempotent)
+  if (!attr_set) {
+    cudaError_t e = cudaFuncSetAttribute(kc_gemm_kernel<MFW, PHILOX>, cudaFuncAttributeMaxDynamicSharedMemorySize, smem);
+    if (e != cudaSuccess) return e;
+    attr_set = true;
+  }
+  kc_gemm_kernel<MFW, PHILOX><<<grid, GEMM_THREADS, smem, st>>>(tR, tL, a);
+  return cudaGetLastError();
+}
+
+template <int MFW>
+cudaError_t launch_mc_t(cudaStream_t st, dim3 grid, const CUtensorMap& tL, const CUtensorMap& tR, const GemmArgs& a) {
+  constexpr int smem = MCSmem<MFW>::TOTAL;
+  static bool attr_set = false;
+  if (!attr_set) {
+    cudaError_t e = cudaFuncSetAttribute(mc_gemm_kernel<MFW>, cudaFuncAttributeMaxDynamicSharedMemorySize, smem);
+    if (e != cudaSuccess) return e;
+    attr_set = true;
+  }
+  mc_gemm_kernel<MFW><<<grid, GEMM_THREADS, smem, st>>>(tL, tR, a);
+  return cudaGetLastError();
+}
+
+}  // namespace
+
+int gemm_mtile(int M) {
+  if (M <= 128) return 16 * ((M + 15) / 16);
+  const int mt = (M + 127) / 128;
+  return 16 * ((M + 16 * mt - 1) / (16 * mt));
+}
+
+int gemm_choose_splits(int M, int N, long long K, int max_splits, int num_sms) {
+  const long long mtiles = (M + gemm_mtile(M) - 1) / gemm_mtile(M);
+  const long long tiles = mtiles * ((N + NT - 1) / NT);
+  if (tiles >= 2LL * num_sms || max_splits <= 1) return 1;
+  int best = 1;
+  double best_score = -1.0;
+  for (int s = 1; s <= max_splits; ++s) {
+    const long long chunk = ((K + s - 1) / s + KT - 1) / KT * KT;
+    if (chunk < 8 * KT && s > 1) break;
+    const long long real_s = (K + chunk - 1) / chunk;
+    const long long ctas = tiles * real_s;
+    const long long waves = (ctas + num_sms - 1) / num_sms;
+    const double eff = static_cast<double>(ctas) / static_cast<double>(waves * num_sms);
+    const double score = eff - 0.002 * static_cast<double>(waves);
+    if (score > best_score + 1e-12) {
+      best_score = score;
+      best = static_cast<int>(real_s);
+    }
+  }
+  return best;
+}
+
+int gemm_nsplit(long long K, int splits) {
+  const int s = splits < 1 ? 1 : splits;
+  long long chunk = ((K + s - 1) / s + KT - 1) / KT * KT;
+  if (chunk < KT) chunk = KT;
+  const long long ns = (K + chunk - 1) / chunk;
+  return ns < 1 ? 1 : static_cast<int>(ns);
+}
+
+static GemmArgs make_args(int M, int N, long long K, int splits, const GemmOutDesc& out) {
+  GemmArgs a{};
+  a.M = M;
+  a.N = N;
+  a.K = K;
+  const int s = splits < 1 ? 1 : splits;
+  a.k_chunk = ((K + s - 1) / s + KT - 1) / KT * KT;
+  if (a.k_chunk < KT) a.k_chunk = KT;
+  a.out.ptr = out.ptr;
+  a.out.ld_m = out.ld_m;
+  a.out.ld_n = out.ld_n;
+  a.out.split_stride = out.split_stride;
+  a.out.m_store = out.m_store;
+  a.out.n_store = out.n_store;
+  return a;
+}
+
+cudaError_t gemm_kc(cudaStream_t st, int M, int N, long long K, const View2D& Lv, const View2D& Rv,
+                    const PhiloxDesc& phx, const GemmOutDesc& out, int splits) {
+  const int MT = gemm_mtile(M);
+  const int mfw = MT / 16;
+  GemmArgs a = make_args(M, N, K, splits, out);
+  const long long nsplit = (K + a.k_chunk - 1) / a.k_chunk;
+  if (phx.enabled) {
+    a.key.k0 = static_cast<uint32_t>(phx.seed);
+    a.key.k1 = static_cast<uint32_t>(phx.seed >> 32);
+    a.tag = phx.tag;
+    a.row_offset = phx.row_offset;
+    a.ell = phx.ell;
+  }
+  CUtensorMap tR, tL;
+  if (!make_tmap(&tR, Rv, 16, NT)) return cudaErrorInvalidValue;
+  if (phx.enabled) {
+    tL = tR;
+  } else if (!make_tmap(&tL, Lv, 16, MT)) {
+    return cudaErrorInvalidValue;
+  }
+  dim3 grid((N + NT - 1) / NT, (M + MT - 1) / MT, static_cast<unsigned>(nsplit < 1 ? 1 : nsplit));
+#define RS_KC(W)                                                              \
+  case W:                                                                     \
+    return phx.enabled ? launch_kc_t<W, true>(st, grid, tR, tL, a)            \
+                       : launch_kc_t<W, false>(st, grid, tR, tL, a);
+  switch (mfw) {
+    RS_KC(1) RS_KC(2) RS_KC(3) RS_KC(4) RS_KC(5) RS_KC(6) RS_KC(7) RS_KC(8)
+    default:
+      return cudaErrorInvalidConfiguration;
+  }
+#undef RS_KC
+}
+
+cudaError_t gemm_mc(cudaStream_t st, int M, int N, long long K, const View2D& Lv, const View2D& Rv,
+                    const GemmOutDesc& out, int splits) {
+  const int MT = gemm_mtile(M);
+  const int mfw = MT / 16;
+  GemmArgs a = make_args(M, N, K, splits, out);
+  const long long nsplit = (K + a.k_chunk - 1) / a.k_chunk;
+  CUtensorMap tL, tR;
+  if (!make_tmap(&tL, Lv, 16, 16)) return cudaErrorInvalidValue;
+  if (!make_tmap(&tR, Rv, 16, 16)) return cudaErrorInvalidValue;
+  dim3 grid((N + NT - 1) / NT, (M + MT - 1) / MT, static_cast<unsigned>(nsplit < 1 ? 1 : nsplit));
+#define RS_MC(W) \
+  case W:        \
+    return launch_mc_t<W>(st, grid, tL, tR, a);
+  switch (mfw) {
+    RS_MC(1) RS_MC(2) RS_MC(3) RS_MC(4) RS_MC(5) RS_MC(6) RS_MC(7) RS_MC(8)
+    default:
+      return cudaErrorInvalidConfiguration;
+  }
+#undef RS_MC
+}
+
+}  // namespace rs

@@ -1,0 +1,342 @@
+// FP64 tensor-core GEMM tiles for the sampling / power-iteration contractions
+// (Fig. 2(a) lines 7 and 12, Fig. 2(b) line 3) and the CholQR Gram products
+// (P:L476).  sm_100a has no FP64 tcgen05 (no kind::f64), so the FP64 tensor path is the
+// warp-level mma.sync.m8n8k4.f64 -> SASS DMMA.8x8x4 (measured 37.1 TF/s = 99.8 % of
+// 148 SM x 64 FMA/clk x 2 x 1.965 GHz, profiles/r01_probe_fp64_peak.jsonl).  Operands are
+// streamed by TMA (cp.async.bulk.tensor, 128B swizzle) through an NSTAGE mbarrier ring; 8 MMA
+// warps (2 along M x 4 along N) hold the FP64 accumulators in registers, and one elected thread
+// issues the TMA loads NSTAGE-1 stages ahead.  (A dedicated producer warp would put 3 warps on
+// one SM sub-partition and cap registers at 168/thread, which spills the 56-double accumulator
+// tile; 8 warps keep 255 available.)
+//
+// Two operand-layout families:
+//  KC  "K-contiguous":  Out[MxN] = L[MxK] * R[KxN], R given as a column-major matrix whose
+//      columns run along K (A itself for B = Omega A and B = C A); L either generated on the
+//      fly (Philox, Omega never touches HBM) or a row-major matrix (rows along K).  Fragments
+//      read 8 rows/cols that are 2 apart ({2r+f}) so that 128B-swizzled rows hit distinct banks.
+//  MC  "M/N-contiguous": L column-major (M contiguous), R stored with N contiguous (e.g. A for
+//      C = B A^T, C for Linv*C).  Fragments read the K rows {2*kk + s} for the same reason.
+// Both support split-K (blockIdx.z = split, partial tiles reduced in a fixed order later).
+#pragma once
+#include "common.cuh"
+#include "philox.cuh"
+
+namespace rs {
+
+constexpr int KT = 16;             // K per pipeline stage (one 128-byte swizzle row of FP64)
+constexpr int NT = 128;            // N per CTA
+constexpr int NSTAGE = 4;          // TMA ring depth
+constexpr int NCONS = 8;           // MMA warps: 2 (M) x 4 (N); lane 0 of warp 0 also issues TMA
+constexpr int GEMM_THREADS = NCONS * 32;  // 2 warps per SM sub-partition -> up to 255 regs/thread
+constexpr int PHX_LA = 2;          // Philox look-ahead (stages generated ahead of use)
+constexpr int PHX_LD = KT + 4;     // padded Omega tile row (doubles): conflict-free A fragments
+
+struct GemmOut {
+  double* ptr;
+  long long ld_m, ld_n;       // element (m, n) at ptr[m*ld_m + n*ld_n]
+  long long split_stride;     // + blockIdx.z * split_stride
+  int m_store, n_store;       // store only m < m_store, n < n_store
+};
+
+struct GemmArgs {
+  int M, N;                   // rows / cols covered by the grid
+  long long K;                // total K
+  long long k_chunk;          // K per split (multiple of KT)
+  GemmOut out;
+  // Philox Omega (KC with generated L): Omega[i, row_offset + k] for i < ell, else 0
+  PhiloxKey key;
+  uint32_t tag;
+  long long row_offset;
+  int ell;
+};
+
+template <int MFW, bool PHILOX>
+struct KCSmem {
+  static constexpr int MT = 16 * MFW;
+  static constexpr int R_BYTES = NT * KT * 8;
+  static constexpr int L_BYTES_TMA = MT * KT * 8;
+  static constexpr int L_BYTES_RAW = PHILOX ? MT * PHX_LD * 8 : L_BYTES_TMA;
+  static constexpr int L_BYTES = (L_BYTES_RAW + 1023) / 1024 * 1024;
+  static constexpr int TOTAL = 1024 + NSTAGE * (R_BYTES + L_BYTES) + 2 * NSTAGE * 8;
+};
+
+template <int MFW>
+struct MCSmem {
+  static constexpr int MT = 16 * MFW;
+  static constexpr int R_BYTES = NT * KT * 8;
+  static constexpr int L_BYTES = MT * KT * 8;
+  static constexpr int TOTAL = 1024 + NSTAGE * (R_BYTES + L_BYTES) + 2 * NSTAGE * 8;
+};
+
+RS_DEVINL unsigned char* align1024(unsigned char* p) {
+  return reinterpret_cast<unsigned char*>((reinterpret_cast<uintptr_t>(p) + 1023) & ~uintptr_t(1023));
+}
+
+// ------------------------------------------------------------------------------------------
+// KC family.  tmR: A-type tensor, dims {K (contiguous), N}, box {16, 128}.
+//             tmL: dims {K (contiguous), M}, box {16, MT} (unused when PHILOX).
+// ------------------------------------------------------------------------------------------
+template <int MFW, bool PHILOX>
+__global__ void __launch_bounds__(GEMM_THREADS, 1)
+    kc_gemm_kernel(const __grid_constant__ CUtensorMap tmR, const __grid_constant__ CUtensorMap tmL,
+                   const GemmArgs a) {
+  using SM = KCSmem<MFW, PHILOX>;
+  constexpr int MT = SM::MT;
+  extern __shared__ unsigned char smem_raw[];
+  unsigned char* smem = align1024(smem_raw);
+  unsigned char* sR = smem;
+  unsigned char* sL = sR + NSTAGE * SM::R_BYTES;
+  uint64_t* full = reinterpret_cast<uint64_t*>(sL + NSTAGE * SM::L_BYTES);
+  uint64_t* empty = full + NSTAGE;
+
+  const int warp = threadIdx.x >> 5, lane = threadIdx.x & 31;
+  const int n0 = blockIdx.x * NT, m0 = blockIdx.y * MT;
+  const long long kb = static_cast<long long>(blockIdx.z) * a.k_chunk;
+  const long long ke = min(a.K, kb + a.k_chunk);
+  const int nk = kb < ke ? static_cast<int>((ke - kb + KT - 1) / KT) : 0;
+
+  if (threadIdx.x == 0) {
+#pragma unroll
+    for (int s = 0; s < NSTAGE; ++s) {
+      mbar_init(&full[s], 1);
+      mbar_init(&empty[s], NCONS);
+    }
+    fence_mbar_init();
+  }
+  __syncthreads();
+
+  auto issue = [&](int it) {  // one thread: fill stage `it`
+    const int s = it % NSTAGE;
+    if (it >= NSTAGE) mbar_wait(&empty[s], ((it / NSTAGE) - 1) & 1);
+    mbar_arrive_expect_tx(&full[s], SM::R_BYTES + (PHILOX ? 0 : SM::L_BYTES_TMA));
+    const int kc = static_cast<int>(kb + static_cast<long long>(it) * KT);
+    tma_load_2d(sR + s * SM::R_BYTES, &tmR, &full[s], kc, n0);
+    if (!PHILOX) tma_load_2d(sL + s * SM::L_BYTES, &tmL, &full[s], kc, m0);
+  };
+  if (threadIdx.x == 0) {
+    tma_prefetch_desc(&tmR);
+    if (!PHILOX) tma_prefetch_desc(&tmL);
+    for (int it = 0; it < NSTAGE - 1 && it < nk; ++it) issue(it);
+  }
+
+  // ---------------- consumers ----------------
+  const int wm = warp >> 2, wn = warp & 3;
+  const int r = lane >> 2, kk = lane & 3;
+
+  // Omega generator: stage `it` -> smem slot, rows [m0, m0+MT) x local k [kb+it*KT, +KT)
+  auto generate = [&](int it, int slot) {
+    double* L = reinterpret_cast<double*>(sL + slot * SM::L_BYTES);
+    const long long kbase = kb + static_cast<long long>(it) * KT;
+    for (int c = threadIdx.x; c < MT * 4; c += NCONS * 32) {
+      const int i = c >> 2, q = c & 3;
+      const int gi = m0 + i;
+      double v[4] = {0.0, 0.0, 0.0, 0.0};
+      if (gi < a.ell) {
+        const long long j = a.row_offset + kbase + 4 * q;
+        const int o = static_cast<int>(j & 3);
+        if (o == 0) {
+          omega_block4(static_cast<uint32_t>(gi), static_cast<uint64_t>(j >> 2), a.tag, a.key, v);
+        } else {
+          double v0[4], v1[4];
+          omega_block4(static_cast<uint32_t>(gi), static_cast<uint64_t>(j >> 2), a.tag, a.key, v0);
+          omega_block4(static_cast<uint32_t>(gi), static_cast<uint64_t>(j >> 2) + 1, a.tag, a.key, v1);
+#pragma unroll
+          for (int e = 0; e < 4; ++e) v[e] = (o + e < 4) ? v0[o + e] : v1[o + e - 4];
+        }
+      }
+      double2* dst = reinterpret_cast<double2*>(L + i * PHX_LD + 4 * q);
+      dst[0] = make_double2(v[0], v[1]);
+      dst[1] = make_double2(v[2], v[3]);
+    }
+  };
+
+  double acc[MFW][4][2];
+#pragma unroll
+  for (int mf = 0; mf < MFW; ++mf)
+#pragma unroll
+    for (int nf = 0; nf < 4; ++nf) acc[mf][nf][0] = acc[mf][nf][1] = 0.0;
+
+  // per-fragment smem row indices
+  int lrow[MFW];
+#pragma unroll
+  for (int mf = 0; mf < MFW; ++mf) {
+    const int mg = wm * MFW + mf;
+    lrow[mf] = PHILOX ? (8 * mg + r) : (16 * (mg >> 1) + 2 * r + (mg & 1));
+  }
+  int rrow[4];
+#pragma unroll
+  for (int nf = 0; nf < 4; ++nf) {
+    const int ng = wn * 4 + nf;
+    rrow[nf] = 16 * (ng >> 1) + 2 * r + (ng & 1);
+  }
+
+  if (PHILOX) {
+    for (int it = 0; it < PHX_LA && it < nk; ++it) generate(it, it % NSTAGE);
+    __syncthreads();
+  }
+
+  for (int it = 0; it < nk; ++it) {
+    const int s = it % NSTAGE;
+    if (threadIdx.x == 0 && it + NSTAGE - 1 < nk) issue(it + NSTAGE - 1);
+    if (PHILOX && it + PHX_LA < nk) generate(it + PHX_LA, (it + PHX_LA) % NSTAGE);
+    mbar_wait(&full[s], (it / NSTAGE) & 1);
+    const unsigned char* Ls = sL + s * SM::L_BYTES;
+    const unsigned char* Rs = sR + s * SM::R_BYTES;
+#pragma unroll
+    for (int ks = 0; ks < KT / 4; ++ks) {
+      const int k = 4 * ks + kk;
+      double af[MFW], bf[4];
+#pragma unroll
+      for (int mf = 0; mf < MFW; ++mf) {
+        if (PHILOX)
+          af[mf] = reinterpret_cast<const double*>(Ls)[lrow[mf] * PHX_LD + k];
+        else
+          af[mf] = *reinterpret_cast<const double*>(Ls + swz128_off(lrow[mf], k));
+      }
+#pragma unroll
+      for (int nf = 0; nf < 4; ++nf) bf[nf] = *reinterpret_cast<const double*>(Rs + swz128_off(rrow[nf], k));
+#pragma unroll
+      for (int mf = 0; mf < MFW; ++mf)
+#pragma unroll
+        for (int nf = 0; nf < 4; ++nf) dmma_8x8x4(acc[mf][nf][0], acc[mf][nf][1], af[mf], bf[nf]);
+    }
+    __syncwarp();
+    if (lane == 0) mbar_arrive(&empty[s]);
+    if (PHILOX) __syncthreads();
+  }
+
+  // ---------------- epilogue ----------------
+  const GemmOut& o = a.out;
+  double* base = o.ptr + static_cast<long long>(blockIdx.z) * o.split_stride;
+#pragma unroll
+  for (int mf = 0; mf < MFW; ++mf) {
+    const int gm = m0 + lrow[mf];
+    if (gm >= o.m_store) continue;
+#pragma unroll
+    for (int nf = 0; nf < 4; ++nf) {
+      const int ng = wn * 4 + nf;
+#pragma unroll
+      for (int e = 0; e < 2; ++e) {
+        const int gn = n0 + 16 * (ng >> 1) + 2 * (2 * kk + e) + (ng & 1);
+        if (gn < o.n_store) base[gm * o.ld_m + gn * o.ld_n] = acc[mf][nf][e];
+      }
+    }
+  }
+}
+
+// ------------------------------------------------------------------------------------------
+// MC family.  tmL: dims {M (contiguous), K}, box {16, 16};  tmR: dims {N (contiguous), K},
+// box {16, 16}.  One 2 KB box per 16 rows of M (or N) per stage.
+// ------------------------------------------------------------------------------------------
+template <int MFW>
+__global__ void __launch_bounds__(GEMM_THREADS, 1)
+    mc_gemm_kernel(const __grid_constant__ CUtensorMap tmL, const __grid_constant__ CUtensorMap tmR,
+                   const GemmArgs a) {
+  using SM = MCSmem<MFW>;
+  constexpr int MT = SM::MT;
+  extern __shared__ unsigned char smem_raw[];
+  unsigned char* smem = align1024(smem_raw);
+  unsigned char* sR = smem;
+  unsigned char* sL = sR + NSTAGE * SM::R_BYTES;
+  uint64_t* full = reinterpret_cast<uint64_t*>(sL + NSTAGE * SM::L_BYTES);
+  uint64_t* empty = full + NSTAGE;
+
+  const int warp = threadIdx.x >> 5, lane = threadIdx.x & 31;
+  const int n0 = blockIdx.x * NT, m0 = blockIdx.y * MT;
+  const long long kb = static_cast<long long>(blockIdx.z) * a.k_chunk;
+  const long long ke = min(a.K, kb + a.k_chunk);
+  const int nk = kb < ke ? static_cast<int>((ke - kb + KT - 1) / KT) : 0;
+
+  if (threadIdx.x == 0) {
+#pragma unroll
+    for (int s = 0; s < NSTAGE; ++s) {
+      mbar_init(&full[s], 1);
+      mbar_init(&empty[s], NCONS);
+    }
+    fence_mbar_init();
+  }
+  __syncthreads();
+
+  auto issue = [&](int it) {
+    const int s = it % NSTAGE;
+    if (it >= NSTAGE) mbar_wait(&empty[s], ((it / NSTAGE) - 1) & 1);
+    mbar_arrive_expect_tx(&full[s], SM::R_BYTES + SM::L_BYTES);
+    const int kc = static_cast<int>(kb + static_cast<long long>(it) * KT);
+#pragma unroll 1
+    for (int b = 0; b < MT / 16; ++b) tma_load_2d(sL + s * SM::L_BYTES + b * 2048, &tmL, &full[s], m0 + 16 * b, kc);
+#pragma unroll 1
+    for (int b = 0; b < NT / 16; ++b) tma_load_2d(sR + s * SM::R_BYTES + b * 2048, &tmR, &full[s], n0 + 16 * b, kc);
+  };
+  if (threadIdx.x == 0) {
+    tma_prefetch_desc(&tmL);
+    tma_prefetch_desc(&tmR);
+    for (int it = 0; it < NSTAGE - 1 && it < nk; ++it) issue(it);
+  }
+
+  const int wm = warp >> 2, wn = warp & 3;
+  const int r = lane >> 2, kk = lane & 3;
+  double acc[MFW][4][2];
+#pragma unroll
+  for (int mf = 0; mf < MFW; ++mf)
+#pragma unroll
+    for (int nf = 0; nf < 4; ++nf) acc[mf][nf][0] = acc[mf][nf][1] = 0.0;
+
+  uint32_t loff[MFW], roff[4];
+#pragma unroll
+  for (int mf = 0; mf < MFW; ++mf) {
+    const int m = 8 * (wm * MFW + mf) + r;
+    loff[mf] = (m >> 4) * 2048;
+  }
+#pragma unroll
+  for (int nf = 0; nf < 4; ++nf) {
+    const int n = 8 * (wn * 4 + nf) + r;
+    roff[nf] = (n >> 4) * 2048;
+  }
+
+  for (int it = 0; it < nk; ++it) {
+    const int s = it % NSTAGE;
+    if (threadIdx.x == 0 && it + NSTAGE - 1 < nk) issue(it + NSTAGE - 1);
+    mbar_wait(&full[s], (it / NSTAGE) & 1);
+    const unsigned char* Ls = sL + s * SM::L_BYTES;
+    const unsigned char* Rs = sR + s * SM::R_BYTES;
+#pragma unroll
+    for (int ks = 0; ks < KT / 4; ++ks) {
+      const uint32_t krow = 8 * (ks >> 1) + 2 * kk + (ks & 1);
+      double af[MFW], bf[4];
+#pragma unroll
+      for (int mf = 0; mf < MFW; ++mf) {
+        const uint32_t mm = (8 * (wm * MFW + mf) + r) & 15;
+        af[mf] = *reinterpret_cast<const double*>(Ls + loff[mf] + swz128_off(krow, mm));
+      }
+#pragma unroll
+      for (int nf = 0; nf < 4; ++nf) {
+        const uint32_t nn = (8 * (wn * 4 + nf) + r) & 15;
+        bf[nf] = *reinterpret_cast<const double*>(Rs + roff[nf] + swz128_off(krow, nn));
+      }
+#pragma unroll
+      for (int mf = 0; mf < MFW; ++mf)
+#pragma unroll
+        for (int nf = 0; nf < 4; ++nf) dmma_8x8x4(acc[mf][nf][0], acc[mf][nf][1], af[mf], bf[nf]);
+    }
+    __syncwarp();
+    if (lane == 0) mbar_arrive(&empty[s]);
+  }
+
+  const GemmOut& o = a.out;
+  double* base = o.ptr + static_cast<long long>(blockIdx.z) * o.split_stride;
+#pragma unroll
+  for (int mf = 0; mf < MFW; ++mf) {
+    const long long gm = m0 + 8 * (wm * MFW + mf) + r;
+    if (gm >= o.m_store) continue;
+#pragma unroll
+    for (int nf = 0; nf < 4; ++nf) {
+#pragma unroll
+      for (int e = 0; e < 2; ++e) {
+        const long long gn = n0 + 8 * (wn * 4 + nf) + 2 * kk + e;
+        if (gn < o.n_store) base[gm * o.ld_m + gn * o.ld_n] = acc[mf][nf][e];
+      }
+    }
+  }
+}
+
+}  // namespace rs

@@ -1,0 +1,69 @@
+// Internal host-side interfaces between the C-ABI orchestration and the kernel launchers.
+#pragma once
+#include <cstdint>
+#include <cuda.h>
+#include <cuda_runtime.h>
+
+namespace rs {
+
+// A 2-D FP64 view: element (i, j) at base[i + j*ld]  (i runs along the contiguous dim0).
+struct View2D {
+  const double* base;
+  long long dim0, dim1, ld;
+};
+
+// Operand descriptions for the two GEMM families (see gemm_f64.cuh).
+struct GemmOutDesc {
+  double* ptr;
+  long long ld_m, ld_n, split_stride;
+  int m_store, n_store;
+};
+
+struct PhiloxDesc {
+  bool enabled;
+  uint64_t seed;
+  uint32_t tag;
+  long long row_offset;
+  int ell;
+};
+
+// Out[M x N] (+split partials) = L[M x K] * R[K x N]
+//   KC: R = Rv with dim0 = K (contiguous), dim1 = N;  L = Lv with dim0 = K, dim1 = M  (or Philox)
+//   MC: L = Lv with dim0 = M (contiguous), dim1 = K;  R = Rv with dim0 = N, dim1 = K
+// splits: number of K splits (>= 1); out.split_stride must be set when splits > 1.
+// `ns_kernel` (optional) receives the kernel's device time when events != nullptr.
+cudaError_t gemm_kc(cudaStream_t st, int M, int N, long long K, const View2D& Lv, const View2D& Rv,
+                    const PhiloxDesc& phx, const GemmOutDesc& out, int splits);
+cudaError_t gemm_mc(cudaStream_t st, int M, int N, long long K, const View2D& Lv, const View2D& Rv,
+                    const GemmOutDesc& out, int splits);
+int gemm_choose_splits(int M, int N, long long K, int max_splits, int num_sms);
+int gemm_nsplit(long long K, int splits);   // splits actually launched for a requested count
+int gemm_mtile(int M);   // rows per CTA tile used for M
+
+// small kernels (small.cu)
+cudaError_t splitk_reduce(cudaStream_t st, double* out, const double* parts, int nsplit, long long count,
+                          long long stride);
+// n x n factor of G; R and Linv are written (zero-padded) as npad x npad.
+cudaError_t chol_inv(cudaStream_t st, const double* G, int ldg, int n, int npad, double* R, int ldr, double* Linv,
+                     int ldl, double* gwork, int* info, int info_code);
+// C[M x N] = A[M x K] * B[K x N] (+ C if accumulate); element strides (row, col) for each.
+cudaError_t small_gemm(cudaStream_t st, int M, int N, int K, const double* A, long long a_rs, long long a_cs,
+                       const double* B, long long b_rs, long long b_cs, double* C, long long c_rs, long long c_cs,
+                       bool accumulate);
+cudaError_t gather_cols(cudaStream_t st, const double* A, long long lda, long long m, const int64_t* perm, int k,
+                        double* Q, long long ldq);
+cudaError_t permute_cols(cudaStream_t st, const double* Rorig, int ldro, int k, long long n, const int64_t* perm,
+                         double* Rp, int ldrp);
+cudaError_t trsm_upper_cols(cudaStream_t st, const double* U, int ldu, int k, const double* Y, long long ldy,
+                            long long ncols, double* X, long long ldx);
+cudaError_t copy_2d(cudaStream_t st, const double* src, long long lds, double* dst, long long ldd, long long rows,
+                    long long cols);
+cudaError_t omega_materialize(cudaStream_t st, uint64_t seed, uint32_t tag, int ell, long long j0, long long ncols,
+                              double* out, long long ldo);
+
+// truncated QRCP (qrcp.cu)
+size_t qrcp_workspace_bytes(int ell, long long n);
+cudaError_t qrcp_truncated(cudaStream_t st, const double* B, int ldb, int ell, long long n, int k, void* work,
+                           int64_t* perm, double* Rhat_orig, int ldr, double* gaps, int* info, int num_sms);
+
+}  // namespace rs

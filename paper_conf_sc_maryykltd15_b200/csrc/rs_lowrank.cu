@@ -1,0 +1,680 @@
+// C-ABI and host orchestration of the random-sampling pipeline (Fig. 2) on one
+// B200 per process, with NCCL over NVLink for the reductions of the 1-D block-row distribution
+// (P:L535-575).  See include/rs_lowrank.h for the contract and DESIGN.md for the design.
+#include <nccl.h>
+
+#include <algorithm>
+#include <cstdarg>
+#include <cstdio>
+#include <cstring>
+#include <map>
+#include <string>
+#include <vector>
+
+#include "internal.h"
+#include "rs_lowrank.h"
+
+using namespace rs;
+
+namespace {
+
+enum State { ST_CREATED = 0, ST_SAMPLED = 1, ST_PIVOTED = 2, ST_FACTORED = 3 };
+
+inline long long round_up(long long x, long long a) { return (x + a - 1) / a * a; }
+
+struct ProfEntry {
+  double ms = 0.0;
+  long long launches = 0;
+  double flops = 0.0;
+};
+
+struct Pending {
+  std::string name;
+  cudaEvent_t e0, e1;
+  double flops;
+};
+
+// Workspace layout (byte offsets), shared by rs_lowrank_workspace_bytes and create.
+struct Layout {
+  int ell, lp, kp, lmax;
+  long long ldc, ldq1;
+  int smax;          // max split-K partial tiles of an l x n product
+  long long part_elems;
+  size_t off_B, off_Bt, off_B1, off_C, off_C1, off_part, off_G, off_Rf, off_Linv, off_cholw, off_Rho, off_Rhat,
+      off_T, off_Q1, off_R1, off_R2, off_Rbar, off_perm, off_info, off_qr, off_gaps;
+  size_t total;
+};
+
+Layout plan(long long m_local, long long n, int k, int p) {
+  Layout L{};
+  L.ell = k + p;
+  L.lp = static_cast<int>(round_up(L.ell, 8));
+  L.kp = static_cast<int>(round_up(k, 8));
+  L.lmax = std::max(L.lp, L.kp);
+  L.ldc = round_up(std::max<long long>(m_local, 1), 16);
+  L.ldq1 = L.ldc;
+  const long long lxn = static_cast<long long>(L.lp) * n;
+  const long long cap = (1LL << 30) / 8;  // <= 1 GiB of partial tiles
+  L.smax = static_cast<int>(std::max<long long>(8, std::min<long long>(64, cap / std::max<long long>(lxn, 1))));
+  L.part_elems = std::max<long long>(static_cast<long long>(L.smax) * lxn,
+                                     1024LL * L.lmax * L.lmax);  // Gram partials: up to 1024 splits
+  size_t off = 0;
+  auto take = [&](size_t bytes) {
+    const size_t o = off;
+    off = (off + bytes + 255) / 256 * 256;
+    return o;
+  };
+  L.off_B = take(lxn * 8);
+  L.off_Bt = take(lxn * 8);
+  L.off_B1 = take(lxn * 8);
+  L.off_C = take(static_cast<size_t>(L.lp) * L.ldc * 8);
+  L.off_C1 = take(static_cast<size_t>(L.lp) * L.ldc * 8);
+  L.off_part = take(static_cast<size_t>(L.part_elems) * 8);
+  const size_t sq = static_cast<size_t>(L.lmax) * L.lmax * 8;
+  L.off_G = take(sq);
+  L.off_Rf = take(sq);
+  L.off_Linv = take(sq);
+  L.off_cholw = take(sq);
+  L.off_Rho = take(static_cast<size_t>(L.kp) * n * 8);
+  L.off_Rhat = take(static_cast<size_t>(L.kp) * n * 8);
+  L.off_T = take(static_cast<size_t>(L.kp) * std::max<long long>(n - k, 1) * 8);
+  L.off_Q1 = take(static_cast<size_t>(L.ldq1) * std::max(k, 1) * 8);
+  L.off_R1 = take(static_cast<size_t>(L.kp) * L.kp * 8);
+  L.off_R2 = take(static_cast<size_t>(L.kp) * L.kp * 8);
+  L.off_Rbar = take(static_cast<size_t>(L.kp) * L.kp * 8);
+  L.off_perm = take(static_cast<size_t>(n) * 8);
+  L.off_info = take(64);
+  L.off_qr = take(qrcp_workspace_bytes(L.ell, n));
+  L.off_gaps = take(static_cast<size_t>(std::max(k, 1)) * 8);
+  L.total = off + 1024;
+  return L;
+}
+
+}  // namespace
+
+struct rs_lowrank_s {
+  long long m_global, m_local, row_offset, n;
+  int k, p, ell;
+  uint64_t seed;
+  cudaStream_t st;
+  ncclComm_t comm;
+  int nranks, rank, sms;
+  Layout L;
+  char* ws;
+  double *B, *Bt, *B1, *C, *C1, *part, *G, *Rf, *Linv, *cholw, *Rho, *Rhat, *T, *Q1, *R1, *R2, *Rbar, *gaps;
+  int64_t* perm;
+  int* info;
+  void* qr;
+  int state;
+  int powers;
+  std::string err;
+  bool prof = false;
+  std::map<std::string, ProfEntry> profile;
+  std::vector<Pending> pending;
+  std::vector<cudaEvent_t> event_pool;
+  std::vector<double> gaps_host;
+};
+
+namespace {
+
+rs_status_t fail(rs_lowrank_t h, rs_status_t code, const char* fmt, ...) {
+  if (h) {
+    char buf[512];
+    va_list ap;
+    va_start(ap, fmt);
+    vsnprintf(buf, sizeof(buf), fmt, ap);
+    va_end(ap);
+    h->err = buf;
+  }
+  return code;
+}
+
+#define RS_CUDA(h, call)                                                                      \
+  do {                                                                                        \
+    cudaError_t e_ = (call);                                                                  \
+    if (e_ != cudaSuccess) return fail(h, RS_ERR_CUDA, "%s: %s (%s:%d)", #call, cudaGetErrorString(e_), __FILE__, __LINE__); \
+  } while (0)
+
+#define RS_NCCL(h, call)                                                                      \
+  do {                                                                                        \
+    ncclResult_t r_ = (call);                                                                 \
+    if (r_ != ncclSuccess) return fail(h, RS_ERR_NCCL, "%s: %s", #call, ncclGetErrorString(r_)); \
+  } while (0)
+
+cudaEvent_t get_event(rs_lowrank_t h) {
+  if (!h->event_pool.empty()) {
+    cudaEvent_t e = h->event_pool.back();
+    h->event_pool.pop_back();
+    return e;
+  }
+  cudaEvent_t e;
+  cudaEventCreate(&e);
+  return e;
+}
+
+// Times the enclosed launches on the handle's stream when profiling is on.
+struct Scope {
+  rs_lowrank_t h;
+  const char* name;
+  double flops;
+  cudaEvent_t e0{};
+  Scope(rs_lowrank_t hh, const char* nm, double fl) : h(hh), name(nm), flops(fl) {
+    if (h->prof) {
+      e0 = get_event(h);
+      cudaEventRecord(e0, h->st);
+    }
+  }
+  ~Scope() {
+    if (h->prof) {
+      cudaEvent_t e1 = get_event(h);
+      cudaEventRecord(e1, h->st);
+      h->pending.push_back(Pending{name, e0, e1, flops});
+    }
+  }
+};
+
+void drain_profile(rs_lowrank_t h) {
+  for (auto& p : h->pending) {
+    cudaEventSynchronize(p.e1);
+    float ms = 0.f;
+    cudaEventElapsedTime(&ms, p.e0, p.e1);
+    auto& e = h->profile[p.name];
+    e.ms += ms;
+    e.launches += 1;
+    e.flops += p.flops;
+    h->event_pool.push_back(p.e0);
+    h->event_pool.push_back(p.e1);
+  }
+  h->pending.clear();
+}
+
+rs_status_t allreduce(rs_lowrank_t h, double* buf, long long count) {
+  if (!h->comm || h->nranks <= 1 || count <= 0) return RS_OK;
+  Scope sc(h, "comm", 0.0);
+  RS_NCCL(h, ncclAllReduce(buf, buf, static_cast<size_t>(count), ncclDouble, ncclSum, h->comm, h->st));
+  return RS_OK;
+}
+
+int max_splits_for(rs_lowrank_t h, long long tile_elems) {
+  const long long s = h->L.part_elems / std::max<long long>(tile_elems, 1);
+  return static_cast<int>(std::max<long long>(1, std::min<long long>(s, 1024)));
+}
+
+// Gram of the rows of a row-major X (lp x ldx, K = m_local along the rows): G = X X^T  (KC)
+rs_status_t gram_rows_kc(rs_lowrank_t h, const double* X, long long ldx, long long K, int rows, int ld_g) {
+  const int splits = gemm_choose_splits(rows, rows, K, max_splits_for(h, static_cast<long long>(ld_g) * ld_g), h->sms);
+  const int ns = gemm_nsplit(K, splits);
+  {
+    Scope sc(h, "gram", 2.0 * rows * rows * static_cast<double>(K));
+    if (K > 0) {
+      View2D Xv{X, K, rows, ldx};
+      GemmOutDesc out{h->part, 1, ld_g, static_cast<long long>(ld_g) * ld_g, ld_g, ld_g};
+      PhiloxDesc nophx{false, 0, 0, 0, 0};
+      RS_CUDA(h, gemm_kc(h->st, rows, rows, K, Xv, Xv, nophx, out, splits));
+    } else {
+      RS_CUDA(h, cudaMemsetAsync(h->part, 0, static_cast<size_t>(ld_g) * ld_g * 8, h->st));
+    }
+  }
+  {
+    Scope sc(h, "reduce", 0.0);
+    RS_CUDA(h, splitk_reduce(h->st, h->G, h->part, K > 0 ? ns : 1, static_cast<long long>(ld_g) * ld_g,
+                             static_cast<long long>(ld_g) * ld_g));
+  }
+  return RS_OK;
+}
+
+// CholQR2 of the replicated short-wide X (lp x n, column-major, ld lp) into Y:
+// G = X X^T, R^T R = G, Y = R^{-T} X, twice.
+rs_status_t cholqr2_rows_small(rs_lowrank_t h, const double* X, double* Y) {
+  const Layout& L = h->L;
+  const double* src = X;
+  for (int pass = 0; pass < 2; ++pass) {
+    double* dst = pass == 0 ? h->B1 : Y;
+    const int splits = gemm_choose_splits(L.lp, L.lp, h->n, max_splits_for(h, static_cast<long long>(L.lp) * L.lp), h->sms);
+    const int ns = gemm_nsplit(h->n, splits);
+    {
+      Scope sc(h, "gram", 2.0 * L.lp * L.lp * static_cast<double>(h->n));
+      View2D Xv{src, L.lp, h->n, L.lp};
+      GemmOutDesc out{h->part, 1, L.lp, static_cast<long long>(L.lp) * L.lp, L.lp, L.lp};
+      RS_CUDA(h, gemm_mc(h->st, L.lp, L.lp, h->n, Xv, Xv, out, splits));
+    }
+    {
+      Scope sc(h, "reduce", 0.0);
+      RS_CUDA(h, splitk_reduce(h->st, h->G, h->part, ns, static_cast<long long>(L.lp) * L.lp,
+                               static_cast<long long>(L.lp) * L.lp));
+    }
+    {
+      Scope sc(h, "chol", L.ell * static_cast<double>(L.ell) * L.ell / 3.0);
+      RS_CUDA(h, chol_inv(h->st, h->G, L.lp, L.ell, L.lp, h->Rf, L.lp, h->Linv, L.lp, h->cholw, h->info, RS_ERR_NOT_SPD));
+    }
+    {
+      Scope sc(h, "apply", 2.0 * L.ell * L.ell * static_cast<double>(h->n));
+      RS_CUDA(h, small_gemm(h->st, L.lp, static_cast<int>(h->n), L.lp, h->Linv, 1, L.lp, src, 1, L.lp, dst, 1, L.lp, false));
+    }
+    src = dst;
+  }
+  return RS_OK;
+}
+
+rs_status_t check_matrix(rs_lowrank_t h, const void* p, long long ld, long long rows, const char* name) {
+  if (!p) return fail(h, RS_ERR_INVALID_ARG, "%s is NULL", name);
+  if (reinterpret_cast<uintptr_t>(p) % 16 != 0) return fail(h, RS_ERR_INVALID_ARG, "%s not 16-byte aligned", name);
+  if (ld < rows || ld % 2 != 0) return fail(h, RS_ERR_INVALID_ARG, "%s leading dimension %lld invalid (rows %lld, must be even)", name, ld, rows);
+  return RS_OK;
+}
+
+rs_status_t sync_and_check(rs_lowrank_t h) {
+  RS_CUDA(h, cudaStreamSynchronize(h->st));
+  int info[2] = {0, 0};
+  RS_CUDA(h, cudaMemcpy(info, h->info, sizeof(info), cudaMemcpyDeviceToHost));
+  if (info[0] == RS_ERR_NOT_SPD)
+    return fail(h, RS_ERR_NOT_SPD, "CholQR breakdown: Gram matrix not positive definite at column %d", info[1]);
+  if (info[0] == RS_ERR_RANK_DEFICIENT)
+    return fail(h, RS_ERR_RANK_DEFICIENT, "QRCP: zero residual norm at step %d (rank < k)", info[1]);
+  return RS_OK;
+}
+
+}  // namespace
+
+extern "C" {
+
+size_t rs_lowrank_workspace_bytes(int64_t m_local, int64_t n, int32_t k, int32_t p, int32_t nranks) {
+  (void)nranks;
+  if (m_local < 0 || n < 1 || k < 1 || p < 0) return 0;
+  return plan(m_local, n, k, p).total;
+}
+
+rs_status_t rs_lowrank_create(rs_lowrank_t* out, int64_t m_global, int64_t m_local, int64_t row_offset, int64_t n,
+                              int32_t k, int32_t p, uint64_t seed, void* workspace, size_t workspace_bytes,
+                              void* cuda_stream, void* nccl_comm) {
+  if (!out) return RS_ERR_INVALID_ARG;
+  *out = nullptr;
+  const long long ell = static_cast<long long>(k) + p;
+  if (k < 1 || p < 0 || ell > 512 || ell > m_global || ell > n || m_local < 0 || row_offset < 0 ||
+      row_offset + m_local > m_global || m_global >= (1LL << 31) || n >= (1LL << 31))
+    return RS_ERR_INVALID_ARG;
+  int dev = 0, major = 0, sms = 0;
+  if (cudaGetDevice(&dev) != cudaSuccess) return RS_ERR_CUDA;
+  cudaDeviceGetAttribute(&major, cudaDevAttrComputeCapabilityMajor, dev);
+  cudaDeviceGetAttribute(&sms, cudaDevAttrMultiProcessorCount, dev);
+  if (major != 10) return RS_ERR_UNSUPPORTED;
+  Layout L = plan(m_local, n, k, p);
+  if (!workspace || workspace_bytes < L.total) return RS_ERR_WORKSPACE;
+  auto* h = new rs_lowrank_s();
+  h->m_global = m_global;
+  h->m_local = m_local;
+  h->row_offset = row_offset;
+  h->n = n;
+  h->k = k;
+  h->p = p;
+  h->ell = static_cast<int>(ell);
+  h->seed = seed;
+  h->st = static_cast<cudaStream_t>(cuda_stream);
+  h->comm = static_cast<ncclComm_t>(nccl_comm);
+  h->nranks = 1;
+  h->rank = 0;
+  h->sms = sms;
+  if (h->comm) {
+    if (ncclCommCount(h->comm, &h->nranks) != ncclSuccess || ncclCommUserRank(h->comm, &h->rank) != ncclSuccess) {
+      delete h;
+      return RS_ERR_NCCL;
+    }
+  }
+  h->L = L;
+  char* base = reinterpret_cast<char*>((reinterpret_cast<uintptr_t>(workspace) + 255) & ~uintptr_t(255));
+  h->ws = base;
+  auto D = [&](size_t off) { return reinterpret_cast<double*>(base + off); };
+  h->B = D(L.off_B);
+  h->Bt = D(L.off_Bt);
+  h->B1 = D(L.off_B1);
+  h->C = D(L.off_C);
+  h->C1 = D(L.off_C1);
+  h->part = D(L.off_part);
+  h->G = D(L.off_G);
+  h->Rf = D(L.off_Rf);
+  h->Linv = D(L.off_Linv);
+  h->cholw = D(L.off_cholw);
+  h->Rho = D(L.off_Rho);
+  h->Rhat = D(L.off_Rhat);
+  h->T = D(L.off_T);
+  h->Q1 = D(L.off_Q1);
+  h->R1 = D(L.off_R1);
+  h->R2 = D(L.off_R2);
+  h->Rbar = D(L.off_Rbar);
+  h->gaps = D(L.off_gaps);
+  h->perm = reinterpret_cast<int64_t*>(base + L.off_perm);
+  h->info = reinterpret_cast<int*>(base + L.off_info);
+  h->qr = base + L.off_qr;
+  h->state = ST_CREATED;
+  h->powers = 0;
+  // zero everything once: padding rows/columns of B, C, Linv, R stay zero forever
+  if (cudaMemsetAsync(workspace, 0, L.total, h->st) != cudaSuccess) {
+    delete h;
+    return RS_ERR_CUDA;
+  }
+  *out = h;
+  return RS_OK;
+}
+
+rs_status_t rs_lowrank_sample(rs_lowrank_t h, const double* A, int64_t lda) {
+  if (!h) return RS_ERR_INVALID_ARG;
+  const Layout& L = h->L;
+  if (h->m_local > 0) {
+    rs_status_t s = check_matrix(h, A, lda, h->m_local, "A");
+    if (s != RS_OK) return s;
+  }
+  RS_CUDA(h, cudaMemsetAsync(h->info, 0, 16, h->st));
+  const long long lxn = static_cast<long long>(L.lp) * h->n;
+  if (h->m_local > 0) {
+    const int splits = gemm_choose_splits(L.lp, static_cast<int>(h->n), h->m_local, max_splits_for(h, lxn), h->sms);
+    const int ns = gemm_nsplit(h->m_local, splits);
+    {
+      Scope sc(h, "gemm_sample", 2.0 * h->ell * static_cast<double>(h->m_local) * h->n);
+      View2D Av{A, h->m_local, h->n, lda};
+      GemmOutDesc out{h->part, 1, L.lp, lxn, L.lp, static_cast<int>(h->n)};
+      PhiloxDesc phx{true, h->seed, 0u, h->row_offset, h->ell};
+      RS_CUDA(h, gemm_kc(h->st, L.lp, static_cast<int>(h->n), h->m_local, Av, Av, phx, out, splits));
+    }
+    {
+      Scope sc(h, "reduce", 0.0);
+      RS_CUDA(h, splitk_reduce(h->st, h->B, h->part, ns, lxn, lxn));
+    }
+  } else {
+    RS_CUDA(h, cudaMemsetAsync(h->B, 0, lxn * 8, h->st));
+  }
+  rs_status_t s = allreduce(h, h->B, lxn);
+  if (s != RS_OK) return s;
+  h->state = ST_SAMPLED;
+  h->powers = 0;
+  return RS_OK;
+}
+
+rs_status_t rs_lowrank_power_iterate(rs_lowrank_t h, const double* A, int64_t lda, int32_t q) {
+  if (!h) return RS_ERR_INVALID_ARG;
+  if (h->state != ST_SAMPLED) return fail(h, RS_ERR_BAD_STATE, "power_iterate needs a fresh sample");
+  if (q < 0) return fail(h, RS_ERR_INVALID_ARG, "q < 0");
+  if (q == 0) return RS_OK;
+  const Layout& L = h->L;
+  if (h->m_local > 0) {
+    rs_status_t s = check_matrix(h, A, lda, h->m_local, "A");
+    if (s != RS_OK) return s;
+  }
+  const long long ml = h->m_local, n = h->n;
+  const long long lxn = static_cast<long long>(L.lp) * n;
+  for (int it = 0; it < q; ++it) {
+    // line 5: B := QR(B)  (replicated CholQR2)
+    rs_status_t s = cholqr2_rows_small(h, h->B, h->Bt);
+    if (s != RS_OK) return s;
+    // line 7: C := B A^T   (C row-major lp x ldc: C[i, j] at i*ldc + j)
+    if (ml > 0) {
+      Scope sc(h, "gemm_power_c", 2.0 * h->ell * static_cast<double>(ml) * n);
+      View2D Bv{h->Bt, L.lp, n, L.lp};
+      View2D Av{A, ml, n, lda};
+      GemmOutDesc out{h->C, L.ldc, 1, 0, L.lp, static_cast<int>(ml)};
+      RS_CUDA(h, gemm_mc(h->st, L.lp, static_cast<int>(ml), n, Bv, Av, out, 1));
+    }
+    // line 10: C := QR(C)  (distributed CholQR2; the second R^{-T} is applied to B below)
+    s = gram_rows_kc(h, h->C, L.ldc, ml, L.lp, L.lp);
+    if (s != RS_OK) return s;
+    s = allreduce(h, h->G, static_cast<long long>(L.lp) * L.lp);
+    if (s != RS_OK) return s;
+    {
+      Scope sc(h, "chol", L.ell * static_cast<double>(L.ell) * L.ell / 3.0);
+      RS_CUDA(h, chol_inv(h->st, h->G, L.lp, L.ell, L.lp, h->Rf, L.lp, h->Linv, L.lp, h->cholw, h->info, RS_ERR_NOT_SPD));
+    }
+    if (ml > 0) {
+      Scope sc(h, "apply", 2.0 * L.ell * static_cast<double>(L.ell) * ml);
+      View2D Lv{h->Linv, L.lp, L.lp, L.lp};
+      View2D Cv{h->C, ml, L.lp, L.ldc};
+      GemmOutDesc out{h->C1, L.ldc, 1, 0, L.lp, static_cast<int>(ml)};
+      RS_CUDA(h, gemm_mc(h->st, L.lp, static_cast<int>(ml), L.lp, Lv, Cv, out, 1));
+    }
+    s = gram_rows_kc(h, h->C1, L.ldc, ml, L.lp, L.lp);
+    if (s != RS_OK) return s;
+    s = allreduce(h, h->G, static_cast<long long>(L.lp) * L.lp);
+    if (s != RS_OK) return s;
+    {
+      Scope sc(h, "chol", L.ell * static_cast<double>(L.ell) * L.ell / 3.0);
+      RS_CUDA(h, chol_inv(h->st, h->G, L.lp, L.ell, L.lp, h->Rf, L.lp, h->Linv, L.lp, h->cholw, h->info, RS_ERR_NOT_SPD));
+    }
+    // line 12: B := C A   (B1 = C1 A summed over ranks; then B = R2^{-T} B1, exact re-association)
+    if (ml > 0) {
+      const int splits = gemm_choose_splits(L.lp, static_cast<int>(n), ml, max_splits_for(h, lxn), h->sms);
+      const int ns = gemm_nsplit(ml, splits);
+      {
+        Scope sc(h, "gemm_power_b", 2.0 * h->ell * static_cast<double>(ml) * n);
+        View2D Cv{h->C1, ml, L.lp, L.ldc};
+        View2D Av{A, ml, n, lda};
+        GemmOutDesc out{h->part, 1, L.lp, lxn, L.lp, static_cast<int>(n)};
+        PhiloxDesc nophx{false, 0, 0, 0, 0};
+        RS_CUDA(h, gemm_kc(h->st, L.lp, static_cast<int>(n), ml, Cv, Av, nophx, out, splits));
+      }
+      Scope sc(h, "reduce", 0.0);
+      RS_CUDA(h, splitk_reduce(h->st, h->B1, h->part, ns, lxn, lxn));
+    } else {
+      RS_CUDA(h, cudaMemsetAsync(h->B1, 0, lxn * 8, h->st));
+    }
+    s = allreduce(h, h->B1, lxn);
+    if (s != RS_OK) return s;
+    {
+      Scope sc(h, "apply", 2.0 * L.ell * static_cast<double>(L.ell) * n);
+      RS_CUDA(h, small_gemm(h->st, L.lp, static_cast<int>(n), L.lp, h->Linv, 1, L.lp, h->B1, 1, L.lp, h->B, 1, L.lp, false));
+    }
+    h->powers++;
+  }
+  return RS_OK;
+}
+
+rs_status_t rs_lowrank_pivot(rs_lowrank_t h, int64_t* perm) {
+  if (!h) return RS_ERR_INVALID_ARG;
+  if (h->state != ST_SAMPLED) return fail(h, RS_ERR_BAD_STATE, "pivot needs a sample");
+  const Layout& L = h->L;
+  {
+    Scope sc(h, "qrcp", 0.0);
+    RS_CUDA(h, qrcp_truncated(h->st, h->B, L.lp, L.ell, h->n, h->k, h->qr, h->perm, h->Rho, L.kp, h->gaps, h->info,
+                              h->sms));
+  }
+  {
+    Scope sc(h, "other", static_cast<double>(h->k) * h->k * (h->n - h->k));
+    RS_CUDA(h, permute_cols(h->st, h->Rho, L.kp, h->k, h->n, h->perm, h->Rhat, L.kp));
+    RS_CUDA(h, trsm_upper_cols(h->st, h->Rhat, L.kp, h->k, h->Rhat + static_cast<long long>(h->k) * L.kp, L.kp,
+                               h->n - h->k, h->T, L.kp));
+  }
+  if (perm) RS_CUDA(h, cudaMemcpyAsync(perm, h->perm, h->n * 8, cudaMemcpyDeviceToDevice, h->st));
+  rs_status_t s = sync_and_check(h);
+  if (s != RS_OK) return s;
+  h->gaps_host.assign(h->k, 0.0);
+  RS_CUDA(h, cudaMemcpy(h->gaps_host.data(), h->gaps, h->k * 8, cudaMemcpyDeviceToHost));
+  h->state = ST_PIVOTED;
+  return RS_OK;
+}
+
+rs_status_t rs_lowrank_factor(rs_lowrank_t h, const double* A, int64_t lda, double* Q, int64_t ldq, double* R,
+                              int64_t ldr) {
+  if (!h) return RS_ERR_INVALID_ARG;
+  if (h->state != ST_PIVOTED && h->state != ST_FACTORED) return fail(h, RS_ERR_BAD_STATE, "factor needs pivot");
+  const Layout& L = h->L;
+  const long long ml = h->m_local, n = h->n;
+  const int k = h->k;
+  rs_status_t s;
+  if (ml > 0) {
+    if ((s = check_matrix(h, A, lda, ml, "A")) != RS_OK) return s;
+    if ((s = check_matrix(h, Q, ldq, ml, "Q")) != RS_OK) return s;
+  }
+  if ((s = check_matrix(h, R, ldr, k, "R")) != RS_OK) return s;
+  // Q := A(:, P_{1:k})
+  if (ml > 0) {
+    Scope sc(h, "factor", 0.0);
+    RS_CUDA(h, gather_cols(h->st, A, lda, ml, h->perm, k, Q, ldq));
+  }
+  const double* src = Q;
+  long long ld_src = ldq;
+  for (int pass = 0; pass < 2; ++pass) {
+    double* dst = pass == 0 ? h->Q1 : Q;
+    const long long ld_dst = pass == 0 ? L.ldq1 : ldq;
+    // Gram G = X^T X (k x k) of the tall X = src (m_local x k column-major)
+    s = gram_rows_kc(h, src, ld_src, ml, k, L.kp);
+    if (s != RS_OK) return s;
+    s = allreduce(h, h->G, static_cast<long long>(L.kp) * L.kp);
+    if (s != RS_OK) return s;
+    double* Rk = pass == 0 ? h->R1 : h->R2;
+    {
+      Scope sc(h, "chol", k * static_cast<double>(k) * k / 3.0);
+      RS_CUDA(h, chol_inv(h->st, h->G, L.kp, k, L.kp, Rk, L.kp, h->Linv, L.kp, h->cholw, h->info, RS_ERR_NOT_SPD));
+    }
+    // dst = src * Rk^{-1}  (Rk^{-1}[kk, c] = Linv[c + kk*kp]: N-contiguous operand)
+    if (ml > 0) {
+      Scope sc(h, "factor", 2.0 * k * static_cast<double>(k) * ml);
+      View2D Xv{src, ml, k, ld_src};
+      View2D Wv{h->Linv, k, k, L.kp};
+      GemmOutDesc out{dst, 1, ld_dst, 0, static_cast<int>(ml), k};
+      RS_CUDA(h, gemm_mc(h->st, static_cast<int>(ml), k, k, Xv, Wv, out, 1));
+    }
+    src = dst;
+    ld_src = ld_dst;
+  }
+  {
+    Scope sc(h, "other", 2.0 * k * static_cast<double>(k) * n);
+    // Rbar = R2 R1 ; R = Rbar [I_k T]
+    RS_CUDA(h, small_gemm(h->st, k, k, k, h->R2, 1, L.kp, h->R1, 1, L.kp, h->Rbar, 1, L.kp, false));
+    RS_CUDA(h, copy_2d(h->st, h->Rbar, L.kp, R, ldr, k, k));
+    if (n > k)
+      RS_CUDA(h, small_gemm(h->st, k, static_cast<int>(n - k), k, h->Rbar, 1, L.kp, h->T, 1, L.kp,
+                            R + static_cast<long long>(k) * ldr, 1, ldr, false));
+  }
+  s = sync_and_check(h);
+  if (s != RS_OK) return s;
+  h->state = ST_FACTORED;
+  return RS_OK;
+}
+
+rs_status_t rs_lowrank_run_host(rs_lowrank_t h, const double* A_host, int64_t lda, double* A_dev, int64_t ld_dev,
+                                int32_t q, int64_t* perm_host, double* Q_host, int64_t ldq, double* R_host,
+                                int64_t ldr, double* Q_dev, int64_t ld_qdev, double* R_dev, int64_t ld_rdev) {
+  if (!h || !A_host || lda < h->m_local) return RS_ERR_INVALID_ARG;
+  const long long ml = h->m_local, n = h->n;
+  if (ml > 0)
+    RS_CUDA(h, cudaMemcpy2DAsync(A_dev, ld_dev * 8, A_host, lda * 8, ml * 8, n, cudaMemcpyHostToDevice, h->st));
+  rs_status_t s = rs_lowrank_sample(h, A_dev, ld_dev);
+  if (s != RS_OK) return s;
+  if ((s = rs_lowrank_power_iterate(h, A_dev, ld_dev, q)) != RS_OK) return s;
+  if ((s = rs_lowrank_pivot(h, nullptr)) != RS_OK) return s;
+  if ((s = rs_lowrank_factor(h, A_dev, ld_dev, Q_dev, ld_qdev, R_dev, ld_rdev)) != RS_OK) return s;
+  if (perm_host) RS_CUDA(h, cudaMemcpyAsync(perm_host, h->perm, n * 8, cudaMemcpyDeviceToHost, h->st));
+  if (Q_host && ml > 0)
+    RS_CUDA(h, cudaMemcpy2DAsync(Q_host, ldq * 8, Q_dev, ld_qdev * 8, ml * 8, h->k, cudaMemcpyDeviceToHost, h->st));
+  if (R_host)
+    RS_CUDA(h, cudaMemcpy2DAsync(R_host, ldr * 8, R_dev, ld_rdev * 8, static_cast<size_t>(h->k) * 8, n,
+                                 cudaMemcpyDeviceToHost, h->st));
+  RS_CUDA(h, cudaStreamSynchronize(h->st));
+  return RS_OK;
+}
+
+rs_status_t rs_lowrank_destroy(rs_lowrank_t h) {
+  if (!h) return RS_ERR_INVALID_ARG;
+  for (auto& p : h->pending) {
+    cudaEventDestroy(p.e0);
+    cudaEventDestroy(p.e1);
+  }
+  for (auto e : h->event_pool) cudaEventDestroy(e);
+  delete h;
+  return RS_OK;
+}
+
+rs_status_t rs_lowrank_get_sample(rs_lowrank_t h, double* B, int64_t ldb) {
+  if (!h || !B || ldb < h->ell) return RS_ERR_INVALID_ARG;
+  RS_CUDA(h, cudaMemcpy2DAsync(B, ldb * 8, h->B, h->L.lp * 8, h->ell * 8, h->n, cudaMemcpyDeviceToDevice, h->st));
+  RS_CUDA(h, cudaStreamSynchronize(h->st));
+  return RS_OK;
+}
+
+rs_status_t rs_lowrank_set_sample(rs_lowrank_t h, const double* B, int64_t ldb) {
+  if (!h || !B || ldb < h->ell) return RS_ERR_INVALID_ARG;
+  RS_CUDA(h, cudaMemcpy2DAsync(h->B, h->L.lp * 8, B, ldb * 8, h->ell * 8, h->n, cudaMemcpyDeviceToDevice, h->st));
+  RS_CUDA(h, cudaMemsetAsync(h->info, 0, 16, h->st));
+  h->state = ST_SAMPLED;
+  h->powers = 0;
+  return RS_OK;
+}
+
+rs_status_t rs_lowrank_get_pivot_data(rs_lowrank_t h, double* T, int64_t ldt, double* Rhat, int64_t ldrh,
+                                      double* gaps_host) {
+  if (!h) return RS_ERR_INVALID_ARG;
+  if (h->state < ST_PIVOTED) return fail(h, RS_ERR_BAD_STATE, "no pivot data yet");
+  const int k = h->k;
+  if (T && h->n > k)
+    RS_CUDA(h, cudaMemcpy2DAsync(T, ldt * 8, h->T, h->L.kp * 8, k * 8, h->n - k, cudaMemcpyDeviceToDevice, h->st));
+  if (Rhat)
+    RS_CUDA(h, cudaMemcpy2DAsync(Rhat, ldrh * 8, h->Rhat, h->L.kp * 8, k * 8, h->n, cudaMemcpyDeviceToDevice, h->st));
+  RS_CUDA(h, cudaStreamSynchronize(h->st));
+  if (gaps_host) std::copy(h->gaps_host.begin(), h->gaps_host.end(), gaps_host);
+  return RS_OK;
+}
+
+rs_status_t rs_lowrank_omega(rs_lowrank_t h, int64_t j0, int64_t ncols, double* out, int64_t ldo) {
+  if (!h || !out || ldo < h->ell || j0 < 0 || ncols < 0) return RS_ERR_INVALID_ARG;
+  RS_CUDA(h, omega_materialize(h->st, h->seed, 0u, h->ell, j0, ncols, out, ldo));
+  RS_CUDA(h, cudaStreamSynchronize(h->st));
+  return RS_OK;
+}
+
+rs_status_t rs_lowrank_get_info(rs_lowrank_t h, int64_t* info) {
+  if (!h || !info) return RS_ERR_INVALID_ARG;
+  RS_CUDA(h, cudaStreamSynchronize(h->st));
+  int v[2];
+  RS_CUDA(h, cudaMemcpy(v, h->info, sizeof(v), cudaMemcpyDeviceToHost));
+  info[0] = v[0];
+  info[1] = v[1];
+  return RS_OK;
+}
+
+rs_status_t rs_lowrank_set_profiling(rs_lowrank_t h, int32_t enable) {
+  if (!h) return RS_ERR_INVALID_ARG;
+  h->prof = enable != 0;
+  return RS_OK;
+}
+
+rs_status_t rs_lowrank_get_profile(rs_lowrank_t h, const char* name, double* ms, int64_t* launches, double* flops) {
+  if (!h || !name) return RS_ERR_INVALID_ARG;
+  drain_profile(h);
+  auto it = h->profile.find(name);
+  const ProfEntry e = it == h->profile.end() ? ProfEntry{} : it->second;
+  if (ms) *ms = e.ms;
+  if (launches) *launches = e.launches;
+  if (flops) *flops = e.flops;
+  return RS_OK;
+}
+
+rs_status_t rs_lowrank_reset_profile(rs_lowrank_t h) {
+  if (!h) return RS_ERR_INVALID_ARG;
+  drain_profile(h);
+  h->profile.clear();
+  return RS_OK;
+}
+
+const char* rs_lowrank_last_error(rs_lowrank_t h) { return h ? h->err.c_str() : "null handle"; }
+
+rs_status_t rs_comm_get_unique_id(char id_out[128]) {
+  ncclUniqueId id;
+  if (ncclGetUniqueId(&id) != ncclSuccess) return RS_ERR_NCCL;
+  static_assert(sizeof(ncclUniqueId) == 128, "ncclUniqueId size");
+  std::memcpy(id_out, &id, 128);
+  return RS_OK;
+}
+
+rs_status_t rs_comm_init(void** comm, int32_t nranks, const char id[128], int32_t rank) {
+  if (!comm) return RS_ERR_INVALID_ARG;
+  ncclUniqueId uid;
+  std::memcpy(&uid, id, 128);
+  ncclComm_t c;
+  if (ncclCommInitRank(&c, nranks, uid, rank) != ncclSuccess) return RS_ERR_NCCL;
+  *comm = c;
+  return RS_OK;
+}
+
+rs_status_t rs_comm_destroy(void* comm) {
+  if (!comm) return RS_OK;
+  return ncclCommDestroy(static_cast<ncclComm_t>(comm)) == ncclSuccess ? RS_OK : RS_ERR_NCCL;
+}
+
+}  // extern "C"

@@ -1,0 +1,294 @@
+"""Thin Python binding of the C ABI in ``include/rs_lowrank.h`` (argument marshalling only).
+
+Every step of the path runs in the CUDA library ``lib/librs_lowrank.so``; this module only
+converts torch tensors to (pointer, leading dimension) pairs, checks layouts and maps status codes
+to exceptions.  There is no CPU fallback: if the library is missing, importing a function that
+needs it raises.
+
+Matrices are column-major: an m x n matrix is a torch tensor of shape (m, n) with strides
+(1, ld), ld >= m and even (use :func:`empty_colmajor`).
+"""
+
+from __future__ import annotations
+
+import ctypes
+import os
+from dataclasses import dataclass
+
+import torch
+
+_PKG = os.path.dirname(os.path.abspath(__file__))
+LIB_PATH = os.path.join(_PKG, "lib", "librs_lowrank.so")
+
+STATUS = {0: "RS_OK", 1: "RS_ERR_INVALID_ARG", 2: "RS_ERR_BAD_STATE", 3: "RS_ERR_CUDA", 4: "RS_ERR_NCCL",
+          5: "RS_ERR_NOT_SPD", 6: "RS_ERR_RANK_DEFICIENT", 7: "RS_ERR_WORKSPACE", 8: "RS_ERR_UNSUPPORTED"}
+
+ABI_FUNCTIONS = (
+    "rs_lowrank_workspace_bytes", "rs_lowrank_create", "rs_lowrank_sample", "rs_lowrank_power_iterate",
+    "rs_lowrank_pivot", "rs_lowrank_factor", "rs_lowrank_run_host", "rs_lowrank_destroy",
+    "rs_lowrank_get_sample", "rs_lowrank_set_sample", "rs_lowrank_get_pivot_data", "rs_lowrank_omega",
+    "rs_lowrank_get_info", "rs_lowrank_set_profiling", "rs_lowrank_get_profile", "rs_lowrank_reset_profile",
+    "rs_lowrank_last_error", "rs_comm_get_unique_id", "rs_comm_init", "rs_comm_destroy",
+)
+
+
+class RSError(RuntimeError):
+    def __init__(self, code: int, msg: str):
+        super().__init__(f"{STATUS.get(code, code)}: {msg}")
+        self.code = code
+        self.name = STATUS.get(code, str(code))
+
+
+_lib = None
+
+
+def load_library(path: str = LIB_PATH):
+    """Load (once) the CUDA library; raises if it is missing -- no fallback."""
+    global _lib
+    if _lib is not None:
+        return _lib
+    if not os.path.exists(path):
+        raise RuntimeError(f"CUDA library {path} is missing: run `python -m paper_conf_sc_maryykltd15_b200.build` "
+                           "(or __graft_entry__.build()); there is no CPU fallback")
+    lib = ctypes.CDLL(path)
+    P, I64, I32, U64, SZ = ctypes.c_void_p, ctypes.c_int64, ctypes.c_int32, ctypes.c_uint64, ctypes.c_size_t
+    D = ctypes.POINTER(ctypes.c_double)
+    sig = {
+        "rs_lowrank_workspace_bytes": (SZ, [I64, I64, I32, I32, I32]),
+        "rs_lowrank_create": (ctypes.c_int, [ctypes.POINTER(P), I64, I64, I64, I64, I32, I32, U64, P, SZ, P, P]),
+        "rs_lowrank_sample": (ctypes.c_int, [P, P, I64]),
+        "rs_lowrank_power_iterate": (ctypes.c_int, [P, P, I64, I32]),
+        "rs_lowrank_pivot": (ctypes.c_int, [P, P]),
+        "rs_lowrank_factor": (ctypes.c_int, [P, P, I64, P, I64, P, I64]),
+        "rs_lowrank_run_host": (ctypes.c_int, [P, P, I64, P, I64, I32, P, P, I64, P, I64, P, I64, P, I64]),
+        "rs_lowrank_destroy": (ctypes.c_int, [P]),
+        "rs_lowrank_get_sample": (ctypes.c_int, [P, P, I64]),
+        "rs_lowrank_set_sample": (ctypes.c_int, [P, P, I64]),
+        "rs_lowrank_get_pivot_data": (ctypes.c_int, [P, P, I64, P, I64, D]),
+        "rs_lowrank_omega": (ctypes.c_int, [P, I64, I64, P, I64]),
+        "rs_lowrank_get_info": (ctypes.c_int, [P, ctypes.POINTER(I64)]),
+        "rs_lowrank_set_profiling": (ctypes.c_int, [P, I32]),
+        "rs_lowrank_get_profile": (ctypes.c_int, [P, ctypes.c_char_p, D, ctypes.POINTER(I64), D]),
+        "rs_lowrank_reset_profile": (ctypes.c_int, [P]),
+        "rs_lowrank_last_error": (ctypes.c_char_p, [P]),
+        "rs_comm_get_unique_id": (ctypes.c_int, [ctypes.c_char_p]),
+        "rs_comm_init": (ctypes.c_int, [ctypes.POINTER(P), I32, ctypes.c_char_p, I32]),
+        "rs_comm_destroy": (ctypes.c_int, [P]),
+    }
+    for name, (res, args) in sig.items():
+        fn = getattr(lib, name)
+        fn.restype = res
+        fn.argtypes = args
+    _lib = lib
+    return lib
+
+
+# ---------------------------------------------------------------------------------------------
+# layout helpers
+# ---------------------------------------------------------------------------------------------
+def empty_colmajor(m: int, n: int, device="cuda", dtype=torch.float64, ld: int | None = None, pin: bool = False):
+    """Uninitialised m x n column-major tensor (strides (1, ld)), ld >= m rounded up to even."""
+    ld = max(m, 1) if ld is None else ld
+    ld += ld & 1
+    if device == "cpu" or (isinstance(device, torch.device) and device.type == "cpu"):
+        store = torch.empty((n, ld), dtype=dtype, pin_memory=pin)
+    else:
+        store = torch.empty((n, ld), dtype=dtype, device=device)
+    return store[:, :m].t()
+
+
+def colmajor_ld(t: torch.Tensor, name: str = "matrix") -> int:
+    if t.dim() != 2:
+        raise ValueError(f"{name} must be 2-D")
+    if t.dtype != torch.float64:
+        raise ValueError(f"{name} must be float64 (the paper's precision, P:L666-667)")
+    m, n = t.shape
+    if n > 1 and t.stride(0) != 1:
+        raise ValueError(f"{name} must be column-major (stride(0) == 1), got strides {t.stride()}")
+    ld = t.stride(1) if n > 1 else max(m, 1)
+    return ld
+
+
+def _check(code: int, h=None):
+    if code != 0:
+        msg = load_library().rs_lowrank_last_error(h).decode() if h else ""
+        raise RSError(code, msg)
+
+
+def _stream_ptr(stream) -> int:
+    if stream is None:
+        stream = torch.cuda.current_stream()
+    return stream.cuda_stream
+
+
+# ---------------------------------------------------------------------------------------------
+# ABI-named functions
+# ---------------------------------------------------------------------------------------------
+def workspace_bytes(m_local: int, n: int, k: int, p: int, nranks: int = 1) -> int:
+    return int(load_library().rs_lowrank_workspace_bytes(m_local, n, k, p, nranks))
+
+
+@dataclass
+class Handle:
+    ptr: ctypes.c_void_p
+    workspace: torch.Tensor
+    m_global: int
+    m_local: int
+    row_offset: int
+    n: int
+    k: int
+    p: int
+    seed: int
+    stream: torch.cuda.Stream
+
+    @property
+    def ell(self) -> int:
+        return self.k + self.p
+
+
+def create(m_global: int, m_local: int, row_offset: int, n: int, k: int, p: int, seed: int = 0x5C15, *,
+           device=None, stream=None, nccl_comm=None) -> Handle:
+    lib = load_library()
+    device = torch.device("cuda", torch.cuda.current_device()) if device is None else torch.device(device)
+    nbytes = workspace_bytes(m_local, n, k, p)
+    if nbytes == 0:
+        raise RSError(1, "invalid sizes")
+    ws = torch.empty(nbytes, dtype=torch.uint8, device=device)
+    stream = torch.cuda.current_stream(device) if stream is None else stream
+    h = ctypes.c_void_p()
+    code = lib.rs_lowrank_create(ctypes.byref(h), m_global, m_local, row_offset, n, k, p, seed & (2**64 - 1),
+                                 ws.data_ptr(), nbytes, stream.cuda_stream, nccl_comm)
+    _check(code)
+    return Handle(h, ws, m_global, m_local, row_offset, n, k, p, seed, stream)
+
+
+def sample(h: Handle, A: torch.Tensor):
+    _check(load_library().rs_lowrank_sample(h.ptr, A.data_ptr(), colmajor_ld(A, "A")), h.ptr)
+
+
+def power_iterate(h: Handle, A: torch.Tensor, q: int):
+    _check(load_library().rs_lowrank_power_iterate(h.ptr, A.data_ptr(), colmajor_ld(A, "A"), q), h.ptr)
+
+
+def pivot(h: Handle, perm: torch.Tensor | None = None):
+    if perm is not None and (perm.dtype != torch.int64 or not perm.is_cuda):
+        raise ValueError("perm must be a CUDA int64 tensor")
+    _check(load_library().rs_lowrank_pivot(h.ptr, perm.data_ptr() if perm is not None else None), h.ptr)
+
+
+def factor(h: Handle, A: torch.Tensor, Q: torch.Tensor, R: torch.Tensor):
+    _check(load_library().rs_lowrank_factor(h.ptr, A.data_ptr(), colmajor_ld(A, "A"), Q.data_ptr(),
+                                            colmajor_ld(Q, "Q"), R.data_ptr(), colmajor_ld(R, "R")), h.ptr)
+
+
+def run_host(h: Handle, A_host: torch.Tensor, A_dev: torch.Tensor, q: int, perm_host: torch.Tensor,
+             Q_host: torch.Tensor, R_host: torch.Tensor, Q_dev: torch.Tensor, R_dev: torch.Tensor):
+    _check(load_library().rs_lowrank_run_host(
+        h.ptr, A_host.data_ptr(), colmajor_ld(A_host, "A_host"), A_dev.data_ptr(), colmajor_ld(A_dev, "A_dev"), q,
+        perm_host.data_ptr(), Q_host.data_ptr(), colmajor_ld(Q_host, "Q_host"), R_host.data_ptr(),
+        colmajor_ld(R_host, "R_host"), Q_dev.data_ptr(), colmajor_ld(Q_dev, "Q_dev"), R_dev.data_ptr(),
+        colmajor_ld(R_dev, "R_dev")), h.ptr)
+
+
+def destroy(h: Handle):
+    if h.ptr:
+        _check(load_library().rs_lowrank_destroy(h.ptr))
+        h.ptr = ctypes.c_void_p()
+
+
+def get_sample(h: Handle) -> torch.Tensor:
+    B = empty_colmajor(h.ell, h.n, device=h.workspace.device)
+    _check(load_library().rs_lowrank_get_sample(h.ptr, B.data_ptr(), colmajor_ld(B)), h.ptr)
+    return B
+
+
+def set_sample(h: Handle, B: torch.Tensor):
+    _check(load_library().rs_lowrank_set_sample(h.ptr, B.data_ptr(), colmajor_ld(B, "B")), h.ptr)
+
+
+def get_pivot_data(h: Handle):
+    """(T k x (n-k), R̂ k x n in pivot order, gaps[k]) after pivot."""
+    dev = h.workspace.device
+    T = empty_colmajor(h.k, max(h.n - h.k, 1), device=dev)
+    Rh = empty_colmajor(h.k, h.n, device=dev)
+    gaps = (ctypes.c_double * h.k)()
+    _check(load_library().rs_lowrank_get_pivot_data(h.ptr, T.data_ptr(), colmajor_ld(T), Rh.data_ptr(),
+                                                    colmajor_ld(Rh), gaps), h.ptr)
+    return T[:, : h.n - h.k], Rh, list(gaps)
+
+
+def omega(h: Handle, j0: int, ncols: int) -> torch.Tensor:
+    out = empty_colmajor(h.ell, max(ncols, 1), device=h.workspace.device)
+    _check(load_library().rs_lowrank_omega(h.ptr, j0, ncols, out.data_ptr(), colmajor_ld(out)), h.ptr)
+    return out[:, :ncols]
+
+
+def get_info(h: Handle):
+    arr = (ctypes.c_int64 * 2)()
+    _check(load_library().rs_lowrank_get_info(h.ptr, arr), h.ptr)
+    return int(arr[0]), int(arr[1])
+
+
+def set_profiling(h: Handle, enable: bool = True):
+    _check(load_library().rs_lowrank_set_profiling(h.ptr, 1 if enable else 0), h.ptr)
+
+
+PROFILE_NAMES = ("gemm_sample", "gemm_power_c", "gemm_power_b", "gram", "apply", "chol", "qrcp", "factor",
+                 "reduce", "comm", "other")
+
+
+def get_profile(h: Handle) -> dict:
+    lib = load_library()
+    out = {}
+    for nm in PROFILE_NAMES:
+        ms, fl = ctypes.c_double(), ctypes.c_double()
+        nl = ctypes.c_int64()
+        _check(lib.rs_lowrank_get_profile(h.ptr, nm.encode(), ctypes.byref(ms), ctypes.byref(nl), ctypes.byref(fl)),
+               h.ptr)
+        out[nm] = {"ms": ms.value, "launches": int(nl.value), "flops": fl.value}
+    return out
+
+
+def reset_profile(h: Handle):
+    _check(load_library().rs_lowrank_reset_profile(h.ptr), h.ptr)
+
+
+def last_error(h: Handle) -> str:
+    return load_library().rs_lowrank_last_error(h.ptr).decode()
+
+
+def comm_get_unique_id() -> bytes:
+    buf = ctypes.create_string_buffer(128)
+    _check(load_library().rs_comm_get_unique_id(buf))
+    return buf.raw
+
+
+def comm_init(nranks: int, uid: bytes, rank: int) -> int:
+    c = ctypes.c_void_p()
+    _check(load_library().rs_comm_init(ctypes.byref(c), nranks, uid, rank))
+    return c.value
+
+
+def comm_destroy(comm: int):
+    _check(load_library().rs_comm_destroy(comm))
+
+
+# ---------------------------------------------------------------------------------------------
+# convenience: the whole Fig. 2(b) on one rank's block
+# ---------------------------------------------------------------------------------------------
+def rs_lowrank(A: torch.Tensor, k: int, p: int, q: int, seed: int = 0x5C15, *, m_global: int | None = None,
+               row_offset: int = 0, nccl_comm=None, h: Handle | None = None):
+    """Run sample -> power_iterate(q) -> pivot -> factor.  Returns (perm, Q, R, handle)."""
+    m_local, n = A.shape
+    m_global = m_local if m_global is None else m_global
+    own = h is None
+    if own:
+        h = create(m_global, m_local, row_offset, n, k, p, seed, device=A.device, nccl_comm=nccl_comm)
+    perm = torch.empty(n, dtype=torch.int64, device=A.device)
+    Q = empty_colmajor(m_local, k, device=A.device)
+    R = empty_colmajor(k, n, device=A.device)
+    sample(h, A)
+    power_iterate(h, A, q)
+    pivot(h, perm)
+    factor(h, A, Q, R)
+    return perm, Q, R, h

@@ -1,0 +1,253 @@
+"""GPU parity: the CUDA path (through the C ABI) against the CPU oracle, element by element.
+
+Tolerances (BASELINE.json north_star): Omega bit-exact; B, R, T normwise relative
+<= 1e-11; Q <= 1e-11 (kappa-scaled above kappa(Rbar) = 2e5); pivots identical where every step's
+oracle gap >= 1e-10; |e_gpu - e_oracle| <= 1e-12 on the normalised error."""
+
+import numpy as np
+import pytest
+import torch
+
+from tests.gpu_helpers import pivots_comparable, q_tolerance, rel, to_dev, to_np
+
+pytestmark = pytest.mark.gpu
+
+cuda = pytest.importorskip("torch").cuda
+if not cuda.is_available():  # pragma: no cover
+    pytest.skip("needs a GPU", allow_module_level=True)
+
+import paper_conf_sc_maryykltd15_b200 as rs  # noqa: E402
+from oracle import philox as OP  # noqa: E402
+from oracle import pipeline as OPL  # noqa: E402
+from synth.matrices import make_matrix  # noqa: E402
+
+SEED = 0x5C15
+
+
+@pytest.fixture(scope="module", autouse=True)
+def _built():
+    from paper_conf_sc_maryykltd15_b200 import build
+
+    build.build()
+    rs.load_library()
+
+
+# ------------------------------------------------------------------------------------------
+# Omega: bit-exact against the oracle's Philox + RS-BM32
+# ------------------------------------------------------------------------------------------
+@pytest.mark.parametrize("j0,ncols", [(0, 64), (3, 1001), (123457, 517), (2**33 + 5, 40)])
+def test_omega_bit_exact(j0, ncols):
+    ell = 37
+    h = rs.create(64, 64, 0, 64, 30, 7, SEED)
+    try:
+        got = to_np(rs.omega(h, j0, ncols))
+        want = OP.omega(ell, j0, j0 + ncols, SEED)
+        assert got.shape == want.shape
+        np.testing.assert_array_equal(got, want)
+    finally:
+        rs.destroy(h)
+
+
+# ------------------------------------------------------------------------------------------
+# Step 1: B = Omega A (fused Philox GEMM + split-K)
+# ------------------------------------------------------------------------------------------
+@pytest.mark.parametrize("m,n,k,p", [(500, 200, 20, 10), (1237, 301, 13, 6), (20000, 1000, 50, 10), (64, 130, 8, 0)])
+def test_sample_parity(m, n, k, p):
+    A, _ = make_matrix(m, n, "exp-k", k, seed=m + n)
+    Ad = to_dev(A)
+    h = rs.create(m, m, 0, n, k, p, SEED)
+    try:
+        rs.sample(h, Ad)
+        B = to_np(rs.get_sample(h))
+    finally:
+        rs.destroy(h)
+    Bo = OPL.sample(A, k + p, SEED)
+    assert rel(B, Bo) <= 1e-13
+
+
+def test_sample_row_offset_partition_sums_to_whole():
+    """Two row blocks (offset not a multiple of 4) computed by two handles sum to the 1-rank B."""
+    m, n, k, p = 3001, 257, 16, 8
+    A, _ = make_matrix(m, n, "exp-k", k, seed=7)
+    parts = [(0, 1499), (1499, m)]
+    Bs = []
+    for r0, r1 in parts:
+        h = rs.create(m, r1 - r0, r0, n, k, p, SEED)
+        try:
+            rs.sample(h, to_dev(np.asfortranarray(A[r0:r1])))
+            Bs.append(to_np(rs.get_sample(h)))
+        finally:
+            rs.destroy(h)
+    Bo = OPL.sample(A, k + p, SEED)
+    assert rel(Bs[0] + Bs[1], Bo) <= 1e-13
+    assert rel(Bs[0], OPL.sample(np.asfortranarray(A[:1499]), k + p, SEED)) <= 1e-13
+
+
+def test_sample_with_padded_leading_dimension():
+    m, n, k, p = 777, 150, 10, 5
+    A, _ = make_matrix(m, n, "exp-k", k, seed=3)
+    Ad = to_dev(A, ld=800)
+    assert Ad.stride(1) == 800
+    h = rs.create(m, m, 0, n, k, p, SEED)
+    try:
+        rs.sample(h, Ad)
+        assert rel(to_np(rs.get_sample(h)), OPL.sample(A, k + p, SEED)) <= 1e-13
+    finally:
+        rs.destroy(h)
+
+
+# ------------------------------------------------------------------------------------------
+# The whole pipeline
+# ------------------------------------------------------------------------------------------
+def _run_gpu(A, k, p, q, seed=SEED):
+    Ad = to_dev(A)
+    perm, Q, R, h = rs.rs_lowrank.rs_lowrank(Ad, k, p, q, seed)
+    try:
+        B = to_np(rs.get_sample(h))
+        T, Rhat, gaps = rs.get_pivot_data(h)
+        out = dict(B=B, perm=perm.cpu().numpy(), Q=to_np(Q), R=to_np(R), T=to_np(T), Rhat=to_np(Rhat),
+                   gaps=np.array(gaps))
+    finally:
+        rs.destroy(h)
+    return out
+
+
+def _compare(A, k, p, q, seed=SEED, *, law=None):
+    g = _run_gpu(A, k, p, q, seed)
+    o = OPL.rs_lowrank(A, k, p, q, seed)
+    # B after POWER (what QRCP sees)
+    assert rel(g["B"], o.B) <= 1e-11, ("B", rel(g["B"], o.B))
+    kc = pivots_comparable(o.gaps, k)
+    assert list(g["perm"][:kc]) == list(o.perm[:kc])
+    if kc == k:
+        assert list(g["perm"]) == list(o.perm)
+        assert rel(g["T"], o.T) <= 1e-11, ("T", rel(g["T"], o.T))
+        assert rel(np.abs(g["Rhat"]), np.abs(o.Rhat)) <= 1e-11
+        assert rel(g["R"], o.R) <= 1e-11, ("R", rel(g["R"], o.R))
+        tolq = q_tolerance(o.Rbar)
+        assert rel(g["Q"], o.Q) <= tolq, ("Q", rel(g["Q"], o.Q), tolq)
+        # same evaluator for both factorizations
+        eg = OPL.approx_error(A, g["perm"], g["Q"], g["R"])
+        assert abs(eg - o.err) <= 1e-12, (eg, o.err)
+    Qg = g["Q"]
+    assert np.abs(Qg.T @ Qg - np.eye(k)).max() <= 1e-13
+    return g, o
+
+
+@pytest.mark.parametrize("q", [0, 1, 2])
+def test_pipeline_cfg1(q):
+    """BASELINE configs[0]: m=500, n=200, k=20, p=10, exp-paper decay (plus q = 1, 2)."""
+    A, _ = make_matrix(500, 200, "exp-paper", 20, seed=2015)
+    _compare(A, 20, 10, q)
+
+
+@pytest.mark.parametrize("m,n,k,p,q,law", [
+    (1237, 301, 13, 6, 1, "exp-k"),       # ragged: l = 19 (pads to 24), m, n not tile multiples
+    (3000, 600, 40, 10, 2, "power"),
+    (20000, 1000, 50, 10, 1, "exp-k"),    # several N tiles, split-K
+    (2000, 400, 120, 8, 1, "exp-k"),      # l = 128: full M tile
+    (4000, 500, 150, 10, 0, "exp-k"),     # l = 160 > 128: two M tiles, k > 128
+])
+def test_pipeline_ragged_and_multitile(m, n, k, p, q, law):
+    A, _ = make_matrix(m, n, law, k, seed=m + 3 * n)
+    _compare(A, k, p, q)
+
+
+def test_pipeline_is_bitwise_deterministic():
+    A, _ = make_matrix(5000, 400, "exp-k", 30, seed=5)
+    g1 = _run_gpu(A, 30, 10, 1)
+    g2 = _run_gpu(A, 30, 10, 1)
+    for key in ("B", "Q", "R", "T"):
+        np.testing.assert_array_equal(g1[key], g2[key])
+    np.testing.assert_array_equal(g1["perm"], g2["perm"])
+
+
+def test_omega_identity_special_case_is_truncated_qp3():
+    """set_sample(B := A) with l = m, q = 0: pivots = LAPACK dgeqp3's; |R| rows = QP3's."""
+    import scipy.linalg as sla
+
+    rng = np.random.default_rng(8)
+    A = np.asfortranarray(rng.standard_normal((24, 60)) @ np.diag(np.exp(-np.linspace(0, 4, 60))))
+    k = 8
+    Ad = to_dev(A)
+    h = rs.create(24, 24, 0, 60, k, 16, SEED)
+    try:
+        rs.set_sample(h, Ad)
+        perm = torch.empty(60, dtype=torch.int64, device="cuda")
+        rs.pivot(h, perm)
+        Q = rs.empty_colmajor(24, k)
+        R = rs.empty_colmajor(k, 60)
+        rs.factor(h, Ad, Q, R)
+        perm = perm.cpu().numpy()
+        R = to_np(R)
+    finally:
+        rs.destroy(h)
+    _, Rl, pl = sla.qr(A, pivoting=True, mode="economic")
+    assert list(perm[:k]) == list(pl[:k])
+    R_orig = np.empty_like(R)
+    R_orig[:, perm] = R
+    Rl_orig = np.empty((k, 60))
+    Rl_orig[:, pl] = Rl[:k]
+    np.testing.assert_allclose(np.abs(R_orig), np.abs(Rl_orig), atol=1e-12)
+
+
+def test_exact_recovery_rank_k():
+    A, _ = make_matrix(3000, 300, "rank-k", 12, seed=4)
+    g = _run_gpu(A, 12, 6, 0)
+    e = OPL.approx_error(A, g["perm"], g["Q"], g["R"])
+    assert e <= 1e-13
+
+
+# ------------------------------------------------------------------------------------------
+# errors and state machine
+# ------------------------------------------------------------------------------------------
+def test_rank_deficient_power_iteration_reports_not_spd():
+    """rank(A) = k < l with q >= 1: Gram(C) is singular -> RS_ERR_NOT_SPD."""
+    A, _ = make_matrix(2000, 200, "rank-k", 10, seed=9)
+    Ad = to_dev(A)
+    h = rs.create(2000, 2000, 0, 200, 10, 8, SEED)
+    try:
+        rs.sample(h, Ad)
+        rs.power_iterate(h, Ad, 1)
+        with pytest.raises(rs.RSError) as ei:
+            rs.pivot(h, None)
+        assert ei.value.name == "RS_ERR_NOT_SPD"
+        assert rs.get_info(h)[0] == 5
+    finally:
+        rs.destroy(h)
+
+
+def test_zero_matrix_reports_rank_deficient():
+    A = np.zeros((300, 100), order="F")
+    Ad = to_dev(A)
+    h = rs.create(300, 300, 0, 100, 5, 3, SEED)
+    try:
+        rs.sample(h, Ad)
+        with pytest.raises(rs.RSError) as ei:
+            rs.pivot(h, None)
+        assert ei.value.name == "RS_ERR_RANK_DEFICIENT"
+    finally:
+        rs.destroy(h)
+
+
+def test_state_machine_and_argument_checks():
+    A, _ = make_matrix(300, 100, "exp-k", 5, seed=1)
+    Ad = to_dev(A)
+    h = rs.create(300, 300, 0, 100, 5, 3, SEED)
+    try:
+        with pytest.raises(rs.RSError) as ei:
+            rs.pivot(h, None)
+        assert ei.value.name == "RS_ERR_BAD_STATE"
+        with pytest.raises(rs.RSError):
+            rs.factor(h, Ad, rs.empty_colmajor(300, 5), rs.empty_colmajor(5, 100))
+        odd = torch.empty((100, 301), dtype=torch.float64, device="cuda")[:, :300].t()
+        with pytest.raises(rs.RSError) as ei:
+            rs.sample(h, odd)   # ld = 301 is odd
+        assert ei.value.name == "RS_ERR_INVALID_ARG"
+        rs.sample(h, Ad)
+        rs.pivot(h, None)
+        with pytest.raises(rs.RSError) as ei:
+            rs.power_iterate(h, Ad, 1)
+        assert ei.value.name == "RS_ERR_BAD_STATE"
+    finally:
+        rs.destroy(h)
