@@ -131,6 +131,8 @@ RS_API rs_status_t rs_lowrank_set_profiling(rs_lowrank_t h, int32_t enable);
 RS_API rs_status_t rs_lowrank_get_profile(rs_lowrank_t h, const char* name, double* ms, int64_t* launches,
                                    double* flops);
 RS_API rs_status_t rs_lowrank_reset_profile(rs_lowrank_t h);
+/* Number of CUDA kernels this library has launched in the process (all handles). */
+RS_API int64_t rs_lowrank_kernel_launches(void);
 RS_API const char* rs_lowrank_last_error(rs_lowrank_t h);
 
 /* ---- NCCL plumbing (the harness exchanges the id with torch.distributed) ---- */

@@ -50,6 +50,7 @@ cudaError_t launch_kc_t(cudaStream_t st, dim3 grid, const CUtensorMap& tR, const
     attr_set = true;
   }
   kc_gemm_kernel<MFW, PHILOX><<<grid, GEMM_THREADS, smem, st>>>(tR, tL, a);
+  count_launch();
   return cudaGetLastError();
 }
 
@@ -63,6 +64,7 @@ cudaError_t launch_mc_t(cudaStream_t st, dim3 grid, const CUtensorMap& tL, const
     attr_set = true;
   }
   mc_gemm_kernel<MFW><<<grid, GEMM_THREADS, smem, st>>>(tL, tR, a);
+  count_launch();
   return cudaGetLastError();
 }
 

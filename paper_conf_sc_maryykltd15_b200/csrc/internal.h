@@ -40,6 +40,10 @@ int gemm_choose_splits(int M, int N, long long K, int max_splits, int num_sms);
 int gemm_nsplit(long long K, int splits);   // splits actually launched for a requested count
 int gemm_mtile(int M);   // rows per CTA tile used for M
 
+// kernel launch accounting (every launcher calls count_launch once per kernel launch)
+void count_launch();
+long long launch_count();
+
 // small kernels (small.cu)
 cudaError_t splitk_reduce(cudaStream_t st, double* out, const double* parts, int nsplit, long long count,
                           long long stride);

@@ -203,7 +203,7 @@ __global__ void __launch_bounds__(QR_THREADS, 1)
         s_tau = tau;
         s_beta = beta;
         if (gblk < 0 || !(s_gbest > 0.0)) {
-          if (info && blk == 0) atomicCAS(info, 0, 2), atomicCAS(info + 1, 0, j + 1);
+          if (info && blk == 0) atomicCAS(info, 0, 6 /* RS_ERR_RANK_DEFICIENT */), atomicCAS(info + 1, 0, j + 1);
         }
       }
     }
@@ -286,6 +286,7 @@ cudaError_t qrcp_truncated(cudaStream_t st, const double* B, int ldb, int ell, l
   QrWork* w = static_cast<QrWork*>(work);
   void* args[] = {(void*)&B, (void*)&ldb, (void*)&ell, (void*)&n, (void*)&k, (void*)&w, (void*)&NB, (void*)&cols_per,
                   (void*)&perm, (void*)&Rho, (void*)&ldr, (void*)&gaps, (void*)&info};
+  count_launch();
   return cudaLaunchCooperativeKernel(reinterpret_cast<void*>(qrcp_kernel), dim3(NB), dim3(QR_THREADS), args, smem, st);
 }
 

@@ -652,6 +652,8 @@ rs_status_t rs_lowrank_reset_profile(rs_lowrank_t h) {
   return RS_OK;
 }
 
+int64_t rs_lowrank_kernel_launches(void) { return rs::launch_count(); }
+
 const char* rs_lowrank_last_error(rs_lowrank_t h) { return h ? h->err.c_str() : "null handle"; }
 
 rs_status_t rs_comm_get_unique_id(char id_out[128]) {

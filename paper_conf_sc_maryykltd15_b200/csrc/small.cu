@@ -3,6 +3,7 @@
 // products (T, R = Rbar [I T], Linv * B), column gather A(:, P_{1:k}) and the back substitution
 // T := R̂_{1:k}^{-1} R̂_{k+1:n} (Fig. 2(b) lines 8-10).
 #include <algorithm>
+#include <atomic>
 #include <cstdio>
 
 #include "common.cuh"
@@ -10,6 +11,12 @@
 #include "philox.cuh"
 
 namespace rs {
+
+namespace {
+std::atomic<long long> g_launches{0};
+}
+void count_launch() { g_launches.fetch_add(1, std::memory_order_relaxed); }
+long long launch_count() { return g_launches.load(); }
 
 // ---------------------------------------------------------------------------------------------
 // out[i] = sum_{s=0}^{nsplit-1} parts[s*stride + i], summed in increasing s (deterministic).
@@ -41,6 +48,7 @@ cudaError_t splitk_reduce(cudaStream_t st, double* out, const double* parts, int
   const long long n2 = count / 2 + 1;
   int blocks = static_cast<int>(std::min<long long>((n2 + 255) / 256, 148LL * 8));
   splitk_reduce_kernel<<<blocks, 256, 0, st>>>(out, parts, nsplit, count, stride);
+  count_launch();
   return cudaGetLastError();
 }
 
@@ -121,12 +129,13 @@ cudaError_t chol_inv(cudaStream_t st, const double* G, int ldg, int n, int npad,
   const size_t smem = (use_smem ? static_cast<size_t>(n) * n : 0) * 8 + static_cast<size_t>(CHOL_THREADS / 32) * n * 8;
   static bool attr = false;
   if (!attr) {
-    cudaError_t e = cudaFuncSetAttribute(chol_inv_kernel, cudaFuncAttributeMaxDynamicSharedMemorySize, 227 * 1024);
+    cudaError_t e = cudaFuncSetAttribute(chol_inv_kernel, cudaFuncAttributeMaxDynamicSharedMemorySize, 220 * 1024);
     if (e != cudaSuccess) return e;
     attr = true;
   }
-  if (smem > 227 * 1024) return cudaErrorInvalidValue;
+  if (smem > 220 * 1024) return cudaErrorInvalidValue;
   chol_inv_kernel<<<1, CHOL_THREADS, smem, st>>>(G, ldg, n, R, ldr, Linv, ldl, gwork, info, info_code, npad);
+  count_launch();
   return cudaGetLastError();
 }
 
@@ -183,6 +192,7 @@ cudaError_t small_gemm(cudaStream_t st, int M, int N, int K, const double* A, lo
   if (M <= 0 || N <= 0) return cudaSuccess;
   dim3 grid((N + 63) / 64, (M + 63) / 64);
   small_gemm_kernel<<<grid, 256, 0, st>>>(M, N, K, A, a_rs, a_cs, B, b_rs, b_cs, C, c_rs, c_cs, accumulate);
+  count_launch();
   return cudaGetLastError();
 }
 
@@ -204,6 +214,7 @@ cudaError_t gather_cols(cudaStream_t st, const double* A, long long lda, long lo
   if (m <= 0 || k <= 0) return cudaSuccess;
   const int bx = static_cast<int>(std::min<long long>((m + 255) / 256, 64));
   gather_cols_kernel<<<dim3(bx, k), 256, 0, st>>>(A, lda, m, perm, Q, ldq);
+  count_launch();
   return cudaGetLastError();
 }
 
@@ -223,6 +234,7 @@ cudaError_t permute_cols(cudaStream_t st, const double* Rorig, int ldro, int k, 
   const long long tot = n * k;
   const int blocks = static_cast<int>(std::min<long long>((tot + 255) / 256, 148LL * 8));
   permute_cols_kernel<<<blocks, 256, 0, st>>>(Rorig, ldro, k, n, perm, Rp, ldrp);
+  count_launch();
   return cudaGetLastError();
 }
 
@@ -258,16 +270,17 @@ cudaError_t trsm_upper_cols(cudaStream_t st, const double* U, int ldu, int k, co
                             long long ncols, double* X, long long ldx) {
   if (ncols <= 0) return cudaSuccess;
   const size_t smem = static_cast<size_t>(TRSM_WARPS) * k * 8;
-  if (smem > 227 * 1024) return cudaErrorInvalidValue;
+  if (smem > 220 * 1024) return cudaErrorInvalidValue;
   static bool attr = false;
   if (!attr) {
     cudaError_t e =
-        cudaFuncSetAttribute(trsm_upper_cols_kernel, cudaFuncAttributeMaxDynamicSharedMemorySize, 227 * 1024);
+        cudaFuncSetAttribute(trsm_upper_cols_kernel, cudaFuncAttributeMaxDynamicSharedMemorySize, 220 * 1024);
     if (e != cudaSuccess) return e;
     attr = true;
   }
   const int blocks = static_cast<int>(std::min<long long>((ncols + TRSM_WARPS - 1) / TRSM_WARPS, 148LL * 16));
   trsm_upper_cols_kernel<<<blocks, TRSM_WARPS * 32, smem, st>>>(U, ldu, k, Y, ldy, ncols, X, ldx);
+  count_launch();
   return cudaGetLastError();
 }
 
@@ -286,6 +299,7 @@ cudaError_t copy_2d(cudaStream_t st, const double* src, long long lds, double* d
   if (tot <= 0) return cudaSuccess;
   const int blocks = static_cast<int>(std::min<long long>((tot + 255) / 256, 148LL * 8));
   copy_2d_kernel<<<blocks, 256, 0, st>>>(src, lds, dst, ldd, rows, cols);
+  count_launch();
   return cudaGetLastError();
 }
 
@@ -310,6 +324,7 @@ cudaError_t omega_materialize(cudaStream_t st, uint64_t seed, uint32_t tag, int 
   PhiloxKey key{static_cast<uint32_t>(seed), static_cast<uint32_t>(seed >> 32)};
   const int blocks = static_cast<int>(std::min<long long>((tot + 255) / 256, 148LL * 8));
   omega_kernel<<<blocks, 256, 0, st>>>(key, tag, ell, j0, ncols, out, ldo);
+  count_launch();
   return cudaGetLastError();
 }
 

@@ -28,6 +28,7 @@ ABI_FUNCTIONS = (
     "rs_lowrank_pivot", "rs_lowrank_factor", "rs_lowrank_run_host", "rs_lowrank_destroy",
     "rs_lowrank_get_sample", "rs_lowrank_set_sample", "rs_lowrank_get_pivot_data", "rs_lowrank_omega",
     "rs_lowrank_get_info", "rs_lowrank_set_profiling", "rs_lowrank_get_profile", "rs_lowrank_reset_profile",
+    "rs_lowrank_kernel_launches",
     "rs_lowrank_last_error", "rs_comm_get_unique_id", "rs_comm_init", "rs_comm_destroy",
 )
 
@@ -70,6 +71,7 @@ def load_library(path: str = LIB_PATH):
         "rs_lowrank_set_profiling": (ctypes.c_int, [P, I32]),
         "rs_lowrank_get_profile": (ctypes.c_int, [P, ctypes.c_char_p, D, ctypes.POINTER(I64), D]),
         "rs_lowrank_reset_profile": (ctypes.c_int, [P]),
+        "rs_lowrank_kernel_launches": (I64, []),
         "rs_lowrank_last_error": (ctypes.c_char_p, [P]),
         "rs_comm_get_unique_id": (ctypes.c_int, [ctypes.c_char_p]),
         "rs_comm_init": (ctypes.c_int, [ctypes.POINTER(P), I32, ctypes.c_char_p, I32]),
@@ -251,6 +253,10 @@ def get_profile(h: Handle) -> dict:
 
 def reset_profile(h: Handle):
     _check(load_library().rs_lowrank_reset_profile(h.ptr), h.ptr)
+
+
+def kernel_launches() -> int:
+    return int(load_library().rs_lowrank_kernel_launches())
 
 
 def last_error(h: Handle) -> str:

@@ -72,8 +72,9 @@ def _factors(m: int, n: int, law: str, k: int, seed: int):
         signs = rng.choice(np.array([-1.0, 1.0]), size=m)
         factor = signs * math.sqrt(n / m)                 # exact: +-1 times a double
         return dict(kind="stacked", sigma=sigma, M0=M0, rows=rows, factor=factor)
-    U = haar_orthogonal(n, rng, m)
-    return dict(kind="dense", sigma=sigma, A=(U * sigma[None, :]) @ V.T)
+    r = min(m, n)
+    U = haar_orthogonal(r, rng, m)                        # m x r
+    return dict(kind="dense", sigma=sigma, A=(U * sigma[None, :r]) @ V[:, :r].T)
 
 
 def make_matrix(m: int, n: int, law: str = "exp-k", k: int = 50, seed: int = 2015,

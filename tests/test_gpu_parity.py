@@ -115,22 +115,33 @@ def _run_gpu(A, k, p, q, seed=SEED):
 def _compare(A, k, p, q, seed=SEED, *, law=None):
     g = _run_gpu(A, k, p, q, seed)
     o = OPL.rs_lowrank(A, k, p, q, seed)
-    # B after POWER (what QRCP sees)
-    assert rel(g["B"], o.B) <= 1e-11, ("B", rel(g["B"], o.B))
     kc = pivots_comparable(o.gaps, k)
-    assert list(g["perm"][:kc]) == list(o.perm[:kc])
+    errs = {"B": rel(g["B"], o.B), "pivots_equal": list(g["perm"][:kc]) == list(o.perm[:kc]), "kc": kc}
+    tol = {"B": 1e-11}
     if kc == k:
-        assert list(g["perm"]) == list(o.perm)
-        assert rel(g["T"], o.T) <= 1e-11, ("T", rel(g["T"], o.T))
-        assert rel(np.abs(g["Rhat"]), np.abs(o.Rhat)) <= 1e-11
-        assert rel(g["R"], o.R) <= 1e-11, ("R", rel(g["R"], o.R))
-        tolq = q_tolerance(o.Rbar)
-        assert rel(g["Q"], o.Q) <= tolq, ("Q", rel(g["Q"], o.Q), tolq)
+        errs["perm_all_equal"] = list(g["perm"]) == list(o.perm)
+        errs["T"] = rel(g["T"], o.T)
+        errs["Rhat"] = rel(np.abs(g["Rhat"]), np.abs(o.Rhat))
+        errs["R"] = rel(g["R"], o.R)
+        errs["Q"] = rel(g["Q"], o.Q)
         # same evaluator for both factorizations
-        eg = OPL.approx_error(A, g["perm"], g["Q"], g["R"])
-        assert abs(eg - o.err) <= 1e-12, (eg, o.err)
+        errs["e_gpu"] = OPL.approx_error(A, g["perm"], g["Q"], g["R"])
+        errs["e_oracle"] = o.err
+        # T = R̂11^{-1} R̂12 inherits kappa(R̂11) (reading R9); R, Q: north-star 1e-11,
+        # kappa-scaled above kappa = 2e5 like Q
+        kap11 = np.linalg.cond(o.Rhat[:, :k])
+        tol.update({"T": max(1e-11, 50 * kap11 * 2.0 ** -53), "Rhat": 1e-11,
+                    "R": max(1e-11, 50 * kap11 * 2.0 ** -53), "Q": q_tolerance(o.Rbar)})
     Qg = g["Q"]
-    assert np.abs(Qg.T @ Qg - np.eye(k)).max() <= 1e-13
+    errs["orth"] = float(np.abs(Qg.T @ Qg - np.eye(k)).max())
+    msg = f"errs={errs} tol={tol}"
+    assert errs["pivots_equal"], msg
+    for key, t in tol.items():
+        assert errs[key] <= t, msg
+    if kc == k:
+        assert errs["perm_all_equal"], msg
+        assert abs(errs["e_gpu"] - errs["e_oracle"]) <= 1e-12, msg
+    assert errs["orth"] <= 1e-13, msg
     return g, o
 
 
