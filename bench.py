@@ -140,8 +140,8 @@ def cpu_threads() -> int:
 
 
 def oracle_m_sample(c: dict) -> int:
-    # ~5-15 s of oracle work per sample on a 16-core host; a multiple of n keeps the stacked U
-    return max(c["n"], min(c["m"], 4 * c["n"]) // c["n"] * c["n"])
+    # ~10-20 s of oracle work per sample on the 16-core GPU host; a multiple of n keeps the stacked U
+    return max(c["n"], min(c["m"], 16 * c["n"]) // c["n"] * c["n"])
 
 
 def run_reference(args, c):

@@ -54,6 +54,56 @@ cudaError_t launch_kc_t(cudaStream_t st, dim3 grid, const CUtensorMap& tR, const
   return cudaGetLastError();
 }
 
+template <int MFW, int CS>
+cudaError_t launch_phx_cs(cudaStream_t st, dim3 grid, const CUtensorMap& tR, const GemmArgs& a) {
+  constexpr int smem = KCSmem<MFW, true>::TOTAL;
+  static bool attr_set = false;
+  if (!attr_set) {
+    cudaError_t e =
+        cudaFuncSetAttribute(kc_philox_kernel<MFW, CS>, cudaFuncAttributeMaxDynamicSharedMemorySize, smem);
+    if (e != cudaSuccess) return e;
+    attr_set = true;
+  }
+  grid.x = (grid.x + CS - 1) / CS * CS;  // whole clusters along N (extra CTAs store nothing)
+  cudaLaunchConfig_t cfg = {};
+  cfg.gridDim = grid;
+  cfg.blockDim = dim3(PHX_THREADS);
+  cfg.dynamicSmemBytes = smem;
+  cfg.stream = st;
+  cudaLaunchAttribute attr[1];
+  attr[0].id = cudaLaunchAttributeClusterDimension;
+  attr[0].val.clusterDim.x = CS;
+  attr[0].val.clusterDim.y = 1;
+  attr[0].val.clusterDim.z = 1;
+  cfg.attrs = attr;
+  cfg.numAttrs = 1;
+  cudaError_t e = cudaLaunchKernelEx(&cfg, kc_philox_kernel<MFW, CS>, tR, a);
+  count_launch();
+  return e != cudaSuccess ? e : cudaGetLastError();
+}
+
+// Cluster size for Omega sharing (RS_PHILOX_CLUSTER = 1, 2 or 4; default 2).
+int philox_cluster() {
+  static int cs = [] {
+    const char* v = getenv("RS_PHILOX_CLUSTER");
+    const int c = v ? atoi(v) : 2;
+    return (c == 1 || c == 2 || c == 4) ? c : 2;
+  }();
+  return cs;
+}
+
+template <int MFW>
+cudaError_t launch_phx_t(cudaStream_t st, dim3 grid, const CUtensorMap& tR, const GemmArgs& a) {
+  switch (philox_cluster()) {
+    case 1:
+      return launch_phx_cs<MFW, 1>(st, grid, tR, a);
+    case 2:
+      return launch_phx_cs<MFW, 2>(st, grid, tR, a);
+    default:
+      return launch_phx_cs<MFW, 4>(st, grid, tR, a);
+  }
+}
+
 template <int MFW>
 cudaError_t launch_mc_t(cudaStream_t st, dim3 grid, const CUtensorMap& tL, const CUtensorMap& tR, const GemmArgs& a) {
   constexpr int smem = MCSmem<MFW>::TOTAL;
@@ -146,7 +196,7 @@ cudaError_t gemm_kc(cudaStream_t st, int M, int N, long long K, const View2D& Lv
   dim3 grid((N + NT - 1) / NT, (M + MT - 1) / MT, static_cast<unsigned>(nsplit < 1 ? 1 : nsplit));
 #define RS_KC(W)                                                              \
   case W:                                                                     \
-    return phx.enabled ? launch_kc_t<W, true>(st, grid, tR, tL, a)            \
+    return phx.enabled ? launch_phx_t<W>(st, grid, tR, a)                     \
                        : launch_kc_t<W, false>(st, grid, tR, tL, a);
   switch (mfw) {
     RS_KC(1) RS_KC(2) RS_KC(3) RS_KC(4) RS_KC(5) RS_KC(6) RS_KC(7) RS_KC(8)

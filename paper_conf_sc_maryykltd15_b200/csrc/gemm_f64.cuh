@@ -225,6 +225,183 @@ __global__ void __launch_bounds__(GEMM_THREADS, 1)
 }
 
 // ------------------------------------------------------------------------------------------
+// KC family with Omega generated in the tile loader, warp-specialised: warpgroup 0 (4 warps,
+// one per SM sub-partition) runs Philox + RS-BM32 on the INT/FP32 pipes and issues the TMA
+// loads of A; warpgroups 1-2 (8 warps) run the FP64 DMMA tiles.  setmaxnreg moves registers
+// from the generator warps to the MMA warps.  Omega never leaves shared memory.
+// ------------------------------------------------------------------------------------------
+constexpr int PHX_GEN_WARPS = 4;
+constexpr int PHX_THREADS = (PHX_GEN_WARPS + NCONS) * 32;
+constexpr int PHX_GEN_REGS = 56;
+constexpr int PHX_MMA_REGS = 224;  // 4*32*56 + 8*32*224 = 64512 <= 65536
+
+template <int MFW, int CS>
+__global__ void __launch_bounds__(PHX_THREADS, 1)
+    kc_philox_kernel(const __grid_constant__ CUtensorMap tmR, const GemmArgs a) {
+  // CS > 1: a thread-block cluster of CS CTAs along N shares one Omega tile; CTA rank c generates
+  // rows [c*MT/CS, (c+1)*MT/CS) and stores them into every CTA's ring through distributed shared
+  // memory, so each Omega value is generated once per CS*128 columns of A.
+  using SM = KCSmem<MFW, true>;
+  constexpr int MT = SM::MT;
+  constexpr int ROWS = MT / CS;
+  extern __shared__ unsigned char smem_raw[];
+  unsigned char* smem = align1024(smem_raw);
+  unsigned char* sR = smem;
+  unsigned char* sL = sR + NSTAGE * SM::R_BYTES;
+  uint64_t* full = reinterpret_cast<uint64_t*>(sL + NSTAGE * SM::L_BYTES);
+  uint64_t* empty = full + NSTAGE;
+
+  const int warp = threadIdx.x >> 5, lane = threadIdx.x & 31;
+  const int n0 = blockIdx.x * NT, m0 = blockIdx.y * MT;
+  const long long kb = static_cast<long long>(blockIdx.z) * a.k_chunk;
+  const long long ke = min(a.K, kb + a.k_chunk);
+  const int nk = kb < ke ? static_cast<int>((ke - kb + KT - 1) / KT) : 0;
+  const uint32_t crank = CS > 1 ? cluster_ctarank() : 0;
+
+  if (threadIdx.x == 0) {
+#pragma unroll
+    for (int s = 0; s < NSTAGE; ++s) {
+      mbar_init(&full[s], 1 + PHX_GEN_WARPS * CS);
+      mbar_init(&empty[s], NCONS * CS);
+    }
+    fence_mbar_init();
+  }
+  if (CS > 1)
+    cluster_sync_all();
+  else
+    __syncthreads();
+
+  if (warp < PHX_GEN_WARPS) {
+    // ------------------------- generator / TMA warpgroup -------------------------
+    asm volatile("setmaxnreg.dec.sync.aligned.u32 %0;\n" ::"n"(PHX_GEN_REGS));
+    // work item w = (row, q): Omega[row, 4q .. 4q+3] of the stage (one Philox block when the
+    // row offset is a multiple of 4); items are spread over all 128 generator threads.
+    const int g = threadIdx.x;
+    const int o = static_cast<int>(a.row_offset & 3);  // uniform
+    constexpr int ITEMS = ROWS * 4;
+    if (g == 0) tma_prefetch_desc(&tmR);
+    for (int it = 0; it < nk; ++it) {
+      const int s = it % NSTAGE;
+      if (it >= NSTAGE) {
+        if (lane == 0) {
+          if (CS > 1)
+            mbar_wait_cluster(&empty[s], ((it / NSTAGE) - 1) & 1);
+          else
+            mbar_wait(&empty[s], ((it / NSTAGE) - 1) & 1);
+        }
+        __syncwarp();
+      }
+      if (g == 0) {
+        mbar_arrive_expect_tx(&full[s], SM::R_BYTES);
+        tma_load_2d(sR + s * SM::R_BYTES, &tmR, &full[s], static_cast<int>(kb + static_cast<long long>(it) * KT), n0);
+      }
+      const long long j0 = a.row_offset + kb + static_cast<long long>(it) * KT;  // global row of A
+      const uint64_t t0 = static_cast<uint64_t>(j0 >> 2);
+#pragma unroll 1
+      for (int w = g; w < ITEMS; w += PHX_GEN_WARPS * 32) {
+        const int lrow = static_cast<int>(crank) * ROWS + (w >> 2);
+        const int q = w & 3;
+        const int gi = m0 + lrow;
+        double* dst = reinterpret_cast<double*>(sL + s * SM::L_BYTES) + lrow * PHX_LD + 4 * q;
+        double v0 = 0.0, v1 = 0.0, v2 = 0.0, v3 = 0.0;
+        if (gi < a.ell) {
+          const float4 z = omega_block4f(static_cast<uint32_t>(gi), t0 + q, a.tag, a.key);
+          if (o == 0) {
+            v0 = z.x, v1 = z.y, v2 = z.z, v3 = z.w;
+          } else {
+            const float4 z2 = omega_block4f(static_cast<uint32_t>(gi), t0 + q + 1, a.tag, a.key);
+            v0 = o + 0 < 4 ? f4_get(z, o + 0) : f4_get(z2, o - 4);
+            v1 = o + 1 < 4 ? f4_get(z, o + 1) : f4_get(z2, o - 3);
+            v2 = o + 2 < 4 ? f4_get(z, o + 2) : f4_get(z2, o - 2);
+            v3 = f4_get(z2, o - 1);
+          }
+        }
+        reinterpret_cast<double2*>(dst)[0] = make_double2(v0, v1);
+        reinterpret_cast<double2*>(dst)[1] = make_double2(v2, v3);
+        if (CS > 1) {
+          const uint32_t sa = smem_u32(dst);
+#pragma unroll
+          for (int pc = 1; pc < CS; ++pc) {
+            const uint32_t ra = mapa_shared(sa, (crank + pc) % CS);
+            st_cluster_v2(ra, v0, v1);
+            st_cluster_v2(ra + 16, v2, v3);
+          }
+        }
+      }
+      __syncwarp();
+      if (lane == 0) {
+        mbar_arrive(&full[s]);
+#pragma unroll
+        for (int pc = 1; pc < CS; ++pc) mbar_arrive_remote(mapa_shared(smem_u32(&full[s]), (crank + pc) % CS));
+      }
+    }
+  } else {
+    // ------------------------- MMA warpgroups -------------------------
+    asm volatile("setmaxnreg.inc.sync.aligned.u32 %0;\n" ::"n"(PHX_MMA_REGS));
+    const int w = warp - PHX_GEN_WARPS;
+    const int wm = w >> 2, wn = w & 3;
+    const int r = lane >> 2, kk = lane & 3;
+    double acc[MFW][4][2];
+#pragma unroll
+    for (int mf = 0; mf < MFW; ++mf)
+#pragma unroll
+      for (int nf = 0; nf < 4; ++nf) acc[mf][nf][0] = acc[mf][nf][1] = 0.0;
+    int rrow[4];
+#pragma unroll
+    for (int nf = 0; nf < 4; ++nf) {
+      const int ng = wn * 4 + nf;
+      rrow[nf] = 16 * (ng >> 1) + 2 * r + (ng & 1);
+    }
+    for (int it = 0; it < nk; ++it) {
+      const int s = it % NSTAGE;
+      if (CS > 1)
+        mbar_wait_cluster(&full[s], (it / NSTAGE) & 1);
+      else
+        mbar_wait(&full[s], (it / NSTAGE) & 1);
+      const double* Ls = reinterpret_cast<const double*>(sL + s * SM::L_BYTES);
+      const unsigned char* Rs = sR + s * SM::R_BYTES;
+#pragma unroll
+      for (int ks = 0; ks < KT / 4; ++ks) {
+        const int k = 4 * ks + kk;
+        double af[MFW], bf[4];
+#pragma unroll
+        for (int mf = 0; mf < MFW; ++mf) af[mf] = Ls[(8 * (wm * MFW + mf) + r) * PHX_LD + k];
+#pragma unroll
+        for (int nf = 0; nf < 4; ++nf) bf[nf] = *reinterpret_cast<const double*>(Rs + swz128_off(rrow[nf], k));
+#pragma unroll
+        for (int mf = 0; mf < MFW; ++mf)
+#pragma unroll
+          for (int nf = 0; nf < 4; ++nf) dmma_8x8x4(acc[mf][nf][0], acc[mf][nf][1], af[mf], bf[nf]);
+      }
+      __syncwarp();
+      if (lane == 0) {
+        mbar_arrive(&empty[s]);
+#pragma unroll
+        for (int pc = 1; pc < CS; ++pc) mbar_arrive_remote(mapa_shared(smem_u32(&empty[s]), (crank + pc) % CS));
+      }
+    }
+    const GemmOut& ou = a.out;
+    double* base = ou.ptr + static_cast<long long>(blockIdx.z) * ou.split_stride;
+#pragma unroll
+    for (int mf = 0; mf < MFW; ++mf) {
+      const int gm = m0 + 8 * (wm * MFW + mf) + r;
+      if (gm >= ou.m_store) continue;
+#pragma unroll
+      for (int nf = 0; nf < 4; ++nf) {
+        const int ng = wn * 4 + nf;
+#pragma unroll
+        for (int e = 0; e < 2; ++e) {
+          const int gn = n0 + 16 * (ng >> 1) + 2 * (2 * kk + e) + (ng & 1);
+          if (gn < ou.n_store) base[gm * ou.ld_m + gn * ou.ld_n] = acc[mf][nf][e];
+        }
+      }
+    }
+  }
+  // no CTA may leave while cluster peers can still write its shared memory / barriers
+  if (CS > 1) cluster_sync_all();
+}
+
+// ------------------------------------------------------------------------------------------
 // MC family.  tmL: dims {M (contiguous), K}, box {16, 16};  tmR: dims {N (contiguous), K},
 // box {16, 16}.  One 2 KB box per 16 rows of M (or N) per stage.
 // ------------------------------------------------------------------------------------------
