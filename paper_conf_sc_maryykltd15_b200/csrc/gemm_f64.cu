@@ -40,16 +40,16 @@ bool make_tmap(CUtensorMap* m, const View2D& v, uint32_t box0, uint32_t box1) {
   return r == CUDA_SUCCESS;
 }
 
-template <int MFW, bool PHILOX>
+template <int MFW>
 cudaError_t launch_kc_t(cudaStream_t st, dim3 grid, const CUtensorMap& tR, const CUtensorMap& tL, const GemmArgs& a) {
-  constexpr int smem = KCSmem<MFW, PHILOX>::TOTAL;
+  constexpr int smem = KCSmem<MFW, false>::TOTAL;
   static bool attr_set = false;  // per-instantiation; races are benign (idempotent)
   if (!attr_set) {
-    cudaError_t e = cudaFuncSetAttribute(kc_gemm_kernel<MFW, PHILOX>, cudaFuncAttributeMaxDynamicSharedMemorySize, smem);
+    cudaError_t e = cudaFuncSetAttribute(kc_gemm_kernel<MFW>, cudaFuncAttributeMaxDynamicSharedMemorySize, smem);
     if (e != cudaSuccess) return e;
     attr_set = true;
   }
-  kc_gemm_kernel<MFW, PHILOX><<<grid, GEMM_THREADS, smem, st>>>(tR, tL, a);
+  kc_gemm_kernel<MFW><<<grid, GEMM_THREADS, smem, st>>>(tR, tL, a);
   count_launch();
   return cudaGetLastError();
 }
@@ -197,7 +197,7 @@ cudaError_t gemm_kc(cudaStream_t st, int M, int N, long long K, const View2D& Lv
 #define RS_KC(W)                                                              \
   case W:                                                                     \
     return phx.enabled ? launch_phx_t<W>(st, grid, tR, a)                     \
-                       : launch_kc_t<W, false>(st, grid, tR, tL, a);
+                       : launch_kc_t<W>(st, grid, tR, tL, a);
   switch (mfw) {
     RS_KC(1) RS_KC(2) RS_KC(3) RS_KC(4) RS_KC(5) RS_KC(6) RS_KC(7) RS_KC(8)
     default:

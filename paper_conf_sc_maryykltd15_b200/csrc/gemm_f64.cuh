@@ -4,19 +4,25 @@
 // warp-level mma.sync.m8n8k4.f64 -> SASS DMMA.8x8x4 (measured 37.1 TF/s = 99.8 % of
 // 148 SM x 64 FMA/clk x 2 x 1.965 GHz, profiles/r01_probe_fp64_peak.jsonl).  Operands are
 // streamed by TMA (cp.async.bulk.tensor, 128B swizzle) through an NSTAGE mbarrier ring; 8 MMA
-// warps (2 along M x 4 along N) hold the FP64 accumulators in registers, and one elected thread
-// issues the TMA loads NSTAGE-1 stages ahead.  (A dedicated producer warp would put 3 warps on
-// one SM sub-partition and cap registers at 168/thread, which spills the 56-double accumulator
-// tile; 8 warps keep 255 available.)
+// warps hold the FP64 accumulators in registers, and one elected thread issues the TMA loads
+// NSTAGE-1 stages ahead.  (A dedicated producer warp would put 3 warps on one SM sub-partition
+// and cap registers at 168/thread, which spills the 56-double accumulator tile.)
 //
-// Two operand-layout families:
+// Every non-DMMA instruction issued on an SM sub-partition costs DMMA throughput
+// (profiles/r01_probe_dmma_interference.jsonl: ~14 % at one extra instruction per DMMA), so the
+// fragment loads are 16-byte (LDS.128) and bank-conflict-free by construction:
+//
 //  KC  "K-contiguous":  Out[MxN] = L[MxK] * R[KxN], R given as a column-major matrix whose
 //      columns run along K (A itself for B = Omega A and B = C A); L either generated on the
-//      fly (Philox, Omega never touches HBM) or a row-major matrix (rows along K).  Fragments
-//      read 8 rows/cols that are 2 apart ({2r+f}) so that 128B-swizzled rows hit distinct banks.
-//  MC  "M/N-contiguous": L column-major (M contiguous), R stored with N contiguous (e.g. A for
-//      C = B A^T, C for Linv*C).  Fragments read the K rows {2*kk + s} for the same reason.
-// Both support split-K (blockIdx.z = split, partial tiles reduced in a fixed order later).
+//      fly (Philox, Omega never touches HBM) or a row-major matrix (rows along K).  A thread
+//      loads the K pair (8p+2kk, 8p+2kk+1) of its row and feeds two MMA k-steps with it (any
+//      permutation of K inside a tile is exact).  Fragment row r of fragment f in 16-row group g
+//      is tile row 16g + 8f + r/2 + 4(r%2), so the two rows of a quarter-warp sit in opposite
+//      halves of the 128B swizzle pattern.
+//  MC  "M/N-contiguous": L column-major (M contiguous), R stored with N contiguous (A for
+//      C = B A^T, C for Linv*C, Q for Q*R^-1).  A thread loads the M (or N) pair (2r, 2r+1) at
+//      K row krow = 8(s/2) + 2kk + s%2 and feeds two fragments (even / odd rows) with it.
+// Both support split-K (blockIdx.z = split; partial tiles are reduced in a fixed order later).
 #pragma once
 #include "common.cuh"
 #include "philox.cuh"
@@ -26,10 +32,9 @@ namespace rs {
 constexpr int KT = 16;             // K per pipeline stage (one 128-byte swizzle row of FP64)
 constexpr int NT = 128;            // N per CTA
 constexpr int NSTAGE = 4;          // TMA ring depth
-constexpr int NCONS = 8;           // MMA warps: 2 (M) x 4 (N); lane 0 of warp 0 also issues TMA
+constexpr int NCONS = 8;           // MMA warps; lane 0 of warp 0 also issues TMA
 constexpr int GEMM_THREADS = NCONS * 32;  // 2 warps per SM sub-partition -> up to 255 regs/thread
-constexpr int PHX_LA = 2;          // Philox look-ahead (stages generated ahead of use)
-constexpr int PHX_LD = KT + 4;     // padded Omega tile row (doubles): conflict-free A fragments
+constexpr int PHX_LD = KT + 8;     // padded Omega tile row (doubles): LDS.128 conflict-free
 
 struct GemmOut {
   double* ptr;
@@ -72,15 +77,63 @@ RS_DEVINL unsigned char* align1024(unsigned char* p) {
   return reinterpret_cast<unsigned char*>((reinterpret_cast<uintptr_t>(p) + 1023) & ~uintptr_t(1023));
 }
 
+// KC: tile row of fragment row r in fragment f of 16-row group g
+RS_DEVINL int kc_row(int g, int f, int r) { return 16 * g + 8 * f + (r >> 1) + 4 * (r & 1); }
+// KC: byte offset of the K pair (8p + 2kk, +1) of `row` in a 128B-swizzled K-contiguous tile
+RS_DEVINL uint32_t kc_pair_off(int row, int p, int kk) {
+  return static_cast<uint32_t>(row) * 128u + ((((4 * p + kk) ^ row) & 7) << 4);
+}
+
+// KC accumulate one stage: af(mf, p) / bf(nf, p) return the double2 K pairs.
+template <int MFW, typename LA, typename LB>
+RS_DEVINL void kc_stage_mma(double (&acc)[MFW][4][2], LA&& la, LB&& lb) {
+#pragma unroll
+  for (int p = 0; p < 2; ++p) {
+    double2 b2[4];
+#pragma unroll
+    for (int nf = 0; nf < 4; ++nf) b2[nf] = lb(nf, p);
+#pragma unroll
+    for (int mf = 0; mf < MFW; ++mf) {
+      const double2 a2 = la(mf, p);
+#pragma unroll
+      for (int nf = 0; nf < 4; ++nf) {
+        dmma_8x8x4(acc[mf][nf][0], acc[mf][nf][1], a2.x, b2[nf].x);
+        dmma_8x8x4(acc[mf][nf][0], acc[mf][nf][1], a2.y, b2[nf].y);
+      }
+    }
+  }
+}
+
+// KC epilogue: fragment (mf, nf) element (r, 2kk+e); rowL(mf) gives the tile row of fragment row r
+template <int MFW, typename RL>
+RS_DEVINL void kc_store(const double (&acc)[MFW][4][2], const GemmOut& ou, int m0, int n0, int wn, int kk,
+                        RL&& rowL) {
+  double* base = ou.ptr + static_cast<long long>(blockIdx.z) * ou.split_stride;
+#pragma unroll
+  for (int mf = 0; mf < MFW; ++mf) {
+    const long long gm = m0 + rowL(mf);
+    if (gm >= ou.m_store) continue;
+#pragma unroll
+    for (int nf = 0; nf < 4; ++nf) {
+      const int ng = wn * 4 + nf;
+#pragma unroll
+      for (int e = 0; e < 2; ++e) {
+        const long long gn = n0 + 16 * (ng >> 1) + 8 * (ng & 1) + kk + 4 * e;
+        if (gn < ou.n_store) base[gm * ou.ld_m + gn * ou.ld_n] = acc[mf][nf][e];
+      }
+    }
+  }
+}
+
 // ------------------------------------------------------------------------------------------
-// KC family.  tmR: A-type tensor, dims {K (contiguous), N}, box {16, 128}.
-//             tmL: dims {K (contiguous), M}, box {16, MT} (unused when PHILOX).
+// KC family, both operands by TMA.  tmR: A-type tensor, dims {K (contiguous), N}, box {16, 128};
+// tmL: dims {K (contiguous), M}, box {16, MT}.
 // ------------------------------------------------------------------------------------------
-template <int MFW, bool PHILOX>
+template <int MFW>
 __global__ void __launch_bounds__(GEMM_THREADS, 1)
     kc_gemm_kernel(const __grid_constant__ CUtensorMap tmR, const __grid_constant__ CUtensorMap tmL,
                    const GemmArgs a) {
-  using SM = KCSmem<MFW, PHILOX>;
+  using SM = KCSmem<MFW, false>;
   constexpr int MT = SM::MT;
   extern __shared__ unsigned char smem_raw[];
   unsigned char* smem = align1024(smem_raw);
@@ -108,120 +161,46 @@ __global__ void __launch_bounds__(GEMM_THREADS, 1)
   auto issue = [&](int it) {  // one thread: fill stage `it`
     const int s = it % NSTAGE;
     if (it >= NSTAGE) mbar_wait(&empty[s], ((it / NSTAGE) - 1) & 1);
-    mbar_arrive_expect_tx(&full[s], SM::R_BYTES + (PHILOX ? 0 : SM::L_BYTES_TMA));
+    mbar_arrive_expect_tx(&full[s], SM::R_BYTES + SM::L_BYTES_TMA);
     const int kc = static_cast<int>(kb + static_cast<long long>(it) * KT);
     tma_load_2d(sR + s * SM::R_BYTES, &tmR, &full[s], kc, n0);
-    if (!PHILOX) tma_load_2d(sL + s * SM::L_BYTES, &tmL, &full[s], kc, m0);
+    tma_load_2d(sL + s * SM::L_BYTES, &tmL, &full[s], kc, m0);
   };
   if (threadIdx.x == 0) {
     tma_prefetch_desc(&tmR);
-    if (!PHILOX) tma_prefetch_desc(&tmL);
+    tma_prefetch_desc(&tmL);
     for (int it = 0; it < NSTAGE - 1 && it < nk; ++it) issue(it);
   }
 
-  // ---------------- consumers ----------------
   const int wm = warp >> 2, wn = warp & 3;
   const int r = lane >> 2, kk = lane & 3;
-
-  // Omega generator: stage `it` -> smem slot, rows [m0, m0+MT) x local k [kb+it*KT, +KT)
-  auto generate = [&](int it, int slot) {
-    double* L = reinterpret_cast<double*>(sL + slot * SM::L_BYTES);
-    const long long kbase = kb + static_cast<long long>(it) * KT;
-    for (int c = threadIdx.x; c < MT * 4; c += NCONS * 32) {
-      const int i = c >> 2, q = c & 3;
-      const int gi = m0 + i;
-      double v[4] = {0.0, 0.0, 0.0, 0.0};
-      if (gi < a.ell) {
-        const long long j = a.row_offset + kbase + 4 * q;
-        const int o = static_cast<int>(j & 3);
-        if (o == 0) {
-          omega_block4(static_cast<uint32_t>(gi), static_cast<uint64_t>(j >> 2), a.tag, a.key, v);
-        } else {
-          double v0[4], v1[4];
-          omega_block4(static_cast<uint32_t>(gi), static_cast<uint64_t>(j >> 2), a.tag, a.key, v0);
-          omega_block4(static_cast<uint32_t>(gi), static_cast<uint64_t>(j >> 2) + 1, a.tag, a.key, v1);
-#pragma unroll
-          for (int e = 0; e < 4; ++e) v[e] = (o + e < 4) ? v0[o + e] : v1[o + e - 4];
-        }
-      }
-      double2* dst = reinterpret_cast<double2*>(L + i * PHX_LD + 4 * q);
-      dst[0] = make_double2(v[0], v[1]);
-      dst[1] = make_double2(v[2], v[3]);
-    }
-  };
-
   double acc[MFW][4][2];
 #pragma unroll
   for (int mf = 0; mf < MFW; ++mf)
 #pragma unroll
     for (int nf = 0; nf < 4; ++nf) acc[mf][nf][0] = acc[mf][nf][1] = 0.0;
-
-  // per-fragment smem row indices
-  int lrow[MFW];
-#pragma unroll
-  for (int mf = 0; mf < MFW; ++mf) {
+  auto rowL = [&](int mf) {
     const int mg = wm * MFW + mf;
-    lrow[mf] = PHILOX ? (8 * mg + r) : (16 * (mg >> 1) + 2 * r + (mg & 1));
-  }
-  int rrow[4];
-#pragma unroll
-  for (int nf = 0; nf < 4; ++nf) {
+    return kc_row(mg >> 1, mg & 1, r);
+  };
+  auto rowR = [&](int nf) {
     const int ng = wn * 4 + nf;
-    rrow[nf] = 16 * (ng >> 1) + 2 * r + (ng & 1);
-  }
-
-  if (PHILOX) {
-    for (int it = 0; it < PHX_LA && it < nk; ++it) generate(it, it % NSTAGE);
-    __syncthreads();
-  }
+    return kc_row(ng >> 1, ng & 1, r);
+  };
 
   for (int it = 0; it < nk; ++it) {
     const int s = it % NSTAGE;
     if (threadIdx.x == 0 && it + NSTAGE - 1 < nk) issue(it + NSTAGE - 1);
-    if (PHILOX && it + PHX_LA < nk) generate(it + PHX_LA, (it + PHX_LA) % NSTAGE);
     mbar_wait(&full[s], (it / NSTAGE) & 1);
     const unsigned char* Ls = sL + s * SM::L_BYTES;
     const unsigned char* Rs = sR + s * SM::R_BYTES;
-#pragma unroll
-    for (int ks = 0; ks < KT / 4; ++ks) {
-      const int k = 4 * ks + kk;
-      double af[MFW], bf[4];
-#pragma unroll
-      for (int mf = 0; mf < MFW; ++mf) {
-        if (PHILOX)
-          af[mf] = reinterpret_cast<const double*>(Ls)[lrow[mf] * PHX_LD + k];
-        else
-          af[mf] = *reinterpret_cast<const double*>(Ls + swz128_off(lrow[mf], k));
-      }
-#pragma unroll
-      for (int nf = 0; nf < 4; ++nf) bf[nf] = *reinterpret_cast<const double*>(Rs + swz128_off(rrow[nf], k));
-#pragma unroll
-      for (int mf = 0; mf < MFW; ++mf)
-#pragma unroll
-        for (int nf = 0; nf < 4; ++nf) dmma_8x8x4(acc[mf][nf][0], acc[mf][nf][1], af[mf], bf[nf]);
-    }
+    kc_stage_mma<MFW>(
+        acc, [&](int mf, int p) { return *reinterpret_cast<const double2*>(Ls + kc_pair_off(rowL(mf), p, kk)); },
+        [&](int nf, int p) { return *reinterpret_cast<const double2*>(Rs + kc_pair_off(rowR(nf), p, kk)); });
     __syncwarp();
     if (lane == 0) mbar_arrive(&empty[s]);
-    if (PHILOX) __syncthreads();
   }
-
-  // ---------------- epilogue ----------------
-  const GemmOut& o = a.out;
-  double* base = o.ptr + static_cast<long long>(blockIdx.z) * o.split_stride;
-#pragma unroll
-  for (int mf = 0; mf < MFW; ++mf) {
-    const int gm = m0 + lrow[mf];
-    if (gm >= o.m_store) continue;
-#pragma unroll
-    for (int nf = 0; nf < 4; ++nf) {
-      const int ng = wn * 4 + nf;
-#pragma unroll
-      for (int e = 0; e < 2; ++e) {
-        const int gn = n0 + 16 * (ng >> 1) + 2 * (2 * kk + e) + (ng & 1);
-        if (gn < o.n_store) base[gm * o.ld_m + gn * o.ld_n] = acc[mf][nf][e];
-      }
-    }
-  }
+  kc_store<MFW>(acc, a.out, m0, n0, wn, kk, rowL);
 }
 
 // ------------------------------------------------------------------------------------------
@@ -229,6 +208,9 @@ __global__ void __launch_bounds__(GEMM_THREADS, 1)
 // one per SM sub-partition) runs Philox + RS-BM32 on the INT/FP32 pipes and issues the TMA
 // loads of A; warpgroups 1-2 (8 warps) run the FP64 DMMA tiles.  setmaxnreg moves registers
 // from the generator warps to the MMA warps.  Omega never leaves shared memory.
+// CS > 1: a thread-block cluster of CS CTAs along N shares one Omega tile; CTA rank c generates
+// rows [c*MT/CS, (c+1)*MT/CS) and stores them into every CTA's ring through distributed shared
+// memory, so each Omega value is generated once per CS*128 columns of A.
 // ------------------------------------------------------------------------------------------
 constexpr int PHX_GEN_WARPS = 4;
 constexpr int PHX_THREADS = (PHX_GEN_WARPS + NCONS) * 32;
@@ -238,9 +220,6 @@ constexpr int PHX_MMA_REGS = 224;  // 4*32*56 + 8*32*224 = 64512 <= 65536
 template <int MFW, int CS>
 __global__ void __launch_bounds__(PHX_THREADS, 1)
     kc_philox_kernel(const __grid_constant__ CUtensorMap tmR, const GemmArgs a) {
-  // CS > 1: a thread-block cluster of CS CTAs along N shares one Omega tile; CTA rank c generates
-  // rows [c*MT/CS, (c+1)*MT/CS) and stores them into every CTA's ring through distributed shared
-  // memory, so each Omega value is generated once per CS*128 columns of A.
   using SM = KCSmem<MFW, true>;
   constexpr int MT = SM::MT;
   constexpr int ROWS = MT / CS;
@@ -346,12 +325,11 @@ __global__ void __launch_bounds__(PHX_THREADS, 1)
     for (int mf = 0; mf < MFW; ++mf)
 #pragma unroll
       for (int nf = 0; nf < 4; ++nf) acc[mf][nf][0] = acc[mf][nf][1] = 0.0;
-    int rrow[4];
-#pragma unroll
-    for (int nf = 0; nf < 4; ++nf) {
+    auto rowL = [&](int mf) { return 8 * (wm * MFW + mf) + r; };  // natural rows (padded layout)
+    auto rowR = [&](int nf) {
       const int ng = wn * 4 + nf;
-      rrow[nf] = 16 * (ng >> 1) + 2 * r + (ng & 1);
-    }
+      return kc_row(ng >> 1, ng & 1, r);
+    };
     for (int it = 0; it < nk; ++it) {
       const int s = it % NSTAGE;
       if (CS > 1)
@@ -360,19 +338,10 @@ __global__ void __launch_bounds__(PHX_THREADS, 1)
         mbar_wait(&full[s], (it / NSTAGE) & 1);
       const double* Ls = reinterpret_cast<const double*>(sL + s * SM::L_BYTES);
       const unsigned char* Rs = sR + s * SM::R_BYTES;
-#pragma unroll
-      for (int ks = 0; ks < KT / 4; ++ks) {
-        const int k = 4 * ks + kk;
-        double af[MFW], bf[4];
-#pragma unroll
-        for (int mf = 0; mf < MFW; ++mf) af[mf] = Ls[(8 * (wm * MFW + mf) + r) * PHX_LD + k];
-#pragma unroll
-        for (int nf = 0; nf < 4; ++nf) bf[nf] = *reinterpret_cast<const double*>(Rs + swz128_off(rrow[nf], k));
-#pragma unroll
-        for (int mf = 0; mf < MFW; ++mf)
-#pragma unroll
-          for (int nf = 0; nf < 4; ++nf) dmma_8x8x4(acc[mf][nf][0], acc[mf][nf][1], af[mf], bf[nf]);
-      }
+      kc_stage_mma<MFW>(
+          acc,
+          [&](int mf, int p) { return *reinterpret_cast<const double2*>(Ls + rowL(mf) * PHX_LD + 8 * p + 2 * kk); },
+          [&](int nf, int p) { return *reinterpret_cast<const double2*>(Rs + kc_pair_off(rowR(nf), p, kk)); });
       __syncwarp();
       if (lane == 0) {
         mbar_arrive(&empty[s]);
@@ -380,22 +349,7 @@ __global__ void __launch_bounds__(PHX_THREADS, 1)
         for (int pc = 1; pc < CS; ++pc) mbar_arrive_remote(mapa_shared(smem_u32(&empty[s]), (crank + pc) % CS));
       }
     }
-    const GemmOut& ou = a.out;
-    double* base = ou.ptr + static_cast<long long>(blockIdx.z) * ou.split_stride;
-#pragma unroll
-    for (int mf = 0; mf < MFW; ++mf) {
-      const int gm = m0 + 8 * (wm * MFW + mf) + r;
-      if (gm >= ou.m_store) continue;
-#pragma unroll
-      for (int nf = 0; nf < 4; ++nf) {
-        const int ng = wn * 4 + nf;
-#pragma unroll
-        for (int e = 0; e < 2; ++e) {
-          const int gn = n0 + 16 * (ng >> 1) + 2 * (2 * kk + e) + (ng & 1);
-          if (gn < ou.n_store) base[gm * ou.ld_m + gn * ou.ld_n] = acc[mf][nf][e];
-        }
-      }
-    }
+    kc_store<MFW>(acc, a.out, m0, n0, wn, kk, rowL);
   }
   // no CTA may leave while cluster peers can still write its shared memory / barriers
   if (CS > 1) cluster_sync_all();
@@ -403,7 +357,8 @@ __global__ void __launch_bounds__(PHX_THREADS, 1)
 
 // ------------------------------------------------------------------------------------------
 // MC family.  tmL: dims {M (contiguous), K}, box {16, 16};  tmR: dims {N (contiguous), K},
-// box {16, 16}.  One 2 KB box per 16 rows of M (or N) per stage.
+// box {16, 16}.  One 2 KB box per 16 rows of M (or N) per stage.  Warp w owns the N box w
+// (16 columns, two fragments) and all MT rows (2*MFW fragments).
 // ------------------------------------------------------------------------------------------
 template <int MFW>
 __global__ void __launch_bounds__(GEMM_THREADS, 1)
@@ -450,50 +405,35 @@ __global__ void __launch_bounds__(GEMM_THREADS, 1)
     for (int it = 0; it < NSTAGE - 1 && it < nk; ++it) issue(it);
   }
 
-  const int wm = warp >> 2, wn = warp & 3;
   const int r = lane >> 2, kk = lane & 3;
-  double acc[MFW][4][2];
+  // acc[b][f][f'][e]: M fragment (box b, parity f), N fragment (box warp, parity f'), element e
+  double acc[MFW][2][2][2];
 #pragma unroll
-  for (int mf = 0; mf < MFW; ++mf)
+  for (int b = 0; b < MFW; ++b)
 #pragma unroll
-    for (int nf = 0; nf < 4; ++nf) acc[mf][nf][0] = acc[mf][nf][1] = 0.0;
-
-  uint32_t loff[MFW], roff[4];
+    for (int f = 0; f < 2; ++f)
 #pragma unroll
-  for (int mf = 0; mf < MFW; ++mf) {
-    const int m = 8 * (wm * MFW + mf) + r;
-    loff[mf] = (m >> 4) * 2048;
-  }
-#pragma unroll
-  for (int nf = 0; nf < 4; ++nf) {
-    const int n = 8 * (wn * 4 + nf) + r;
-    roff[nf] = (n >> 4) * 2048;
-  }
+      for (int f2 = 0; f2 < 2; ++f2) acc[b][f][f2][0] = acc[b][f][f2][1] = 0.0;
 
   for (int it = 0; it < nk; ++it) {
     const int s = it % NSTAGE;
     if (threadIdx.x == 0 && it + NSTAGE - 1 < nk) issue(it + NSTAGE - 1);
     mbar_wait(&full[s], (it / NSTAGE) & 1);
     const unsigned char* Ls = sL + s * SM::L_BYTES;
-    const unsigned char* Rs = sR + s * SM::R_BYTES;
+    const unsigned char* Rs = sR + s * SM::R_BYTES + warp * 2048;
 #pragma unroll
     for (int ks = 0; ks < KT / 4; ++ks) {
       const uint32_t krow = 8 * (ks >> 1) + 2 * kk + (ks & 1);
-      double af[MFW], bf[4];
+      const uint32_t off = krow * 128u + (((static_cast<uint32_t>(r) ^ krow) & 7u) << 4);
+      const double2 b2 = *reinterpret_cast<const double2*>(Rs + off);
 #pragma unroll
-      for (int mf = 0; mf < MFW; ++mf) {
-        const uint32_t mm = (8 * (wm * MFW + mf) + r) & 15;
-        af[mf] = *reinterpret_cast<const double*>(Ls + loff[mf] + swz128_off(krow, mm));
+      for (int b = 0; b < MFW; ++b) {
+        const double2 a2 = *reinterpret_cast<const double2*>(Ls + b * 2048 + off);
+        dmma_8x8x4(acc[b][0][0][0], acc[b][0][0][1], a2.x, b2.x);
+        dmma_8x8x4(acc[b][0][1][0], acc[b][0][1][1], a2.x, b2.y);
+        dmma_8x8x4(acc[b][1][0][0], acc[b][1][0][1], a2.y, b2.x);
+        dmma_8x8x4(acc[b][1][1][0], acc[b][1][1][1], a2.y, b2.y);
       }
-#pragma unroll
-      for (int nf = 0; nf < 4; ++nf) {
-        const uint32_t nn = (8 * (wn * 4 + nf) + r) & 15;
-        bf[nf] = *reinterpret_cast<const double*>(Rs + roff[nf] + swz128_off(krow, nn));
-      }
-#pragma unroll
-      for (int mf = 0; mf < MFW; ++mf)
-#pragma unroll
-        for (int nf = 0; nf < 4; ++nf) dmma_8x8x4(acc[mf][nf][0], acc[mf][nf][1], af[mf], bf[nf]);
     }
     __syncwarp();
     if (lane == 0) mbar_arrive(&empty[s]);
@@ -502,18 +442,19 @@ __global__ void __launch_bounds__(GEMM_THREADS, 1)
   const GemmOut& o = a.out;
   double* base = o.ptr + static_cast<long long>(blockIdx.z) * o.split_stride;
 #pragma unroll
-  for (int mf = 0; mf < MFW; ++mf) {
-    const long long gm = m0 + 8 * (wm * MFW + mf) + r;
-    if (gm >= o.m_store) continue;
+  for (int b = 0; b < MFW; ++b)
 #pragma unroll
-    for (int nf = 0; nf < 4; ++nf) {
+    for (int f = 0; f < 2; ++f) {
+      const long long gm = m0 + 16 * b + 2 * r + f;
+      if (gm >= o.m_store) continue;
 #pragma unroll
-      for (int e = 0; e < 2; ++e) {
-        const long long gn = n0 + 8 * (wn * 4 + nf) + 2 * kk + e;
-        if (gn < o.n_store) base[gm * o.ld_m + gn * o.ld_n] = acc[mf][nf][e];
-      }
+      for (int f2 = 0; f2 < 2; ++f2)
+#pragma unroll
+        for (int e = 0; e < 2; ++e) {
+          const long long gn = n0 + 16 * warp + 2 * (2 * kk + e) + f2;
+          if (gn < o.n_store) base[gm * o.ld_m + gn * o.ld_n] = acc[b][f][f2][e];
+        }
     }
-  }
 }
 
 }  // namespace rs
