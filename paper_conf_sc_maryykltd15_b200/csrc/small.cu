@@ -53,93 +53,6 @@ cudaError_t splitk_reduce(cudaStream_t st, double* out, const double* parts, int
 }
 
 // ---------------------------------------------------------------------------------------------
-// Cholesky G = R^T R (R upper, positive diagonal; "the Cholesky factor Rbar of the Gram matrix",
-// P:L477-479) and Linv = R^{-T} (lower).  One CTA.  Work matrix in shared memory when n <= 128,
-// else in `gwork` (global, L2-resident).  Breakdown (pivot <= 0 or NaN) sets *info (LAPACK potrf
-// style 1-based column) once and continues with a unit pivot so no NaN propagates.
-// ---------------------------------------------------------------------------------------------
-constexpr int CHOL_THREADS = 1024;
-constexpr int CHOL_SMEM_MAX_N = 128;
-
-__global__ void __launch_bounds__(CHOL_THREADS) chol_inv_kernel(const double* __restrict__ G, int ldg, int n,
-                                                                 double* __restrict__ R, int ldr,
-                                                                 double* __restrict__ Linv, int ldl,
-                                                                 double* __restrict__ gwork, int* info, int code,
-                                                                 int npad) {
-  extern __shared__ double sm[];
-  const bool use_smem = n <= CHOL_SMEM_MAX_N;
-  const int ldw = use_smem ? n : ldg;
-  double* W = use_smem ? sm : gwork;
-  double* bbuf = use_smem ? sm + n * n : sm;  // per-warp column buffers for the inverse
-  const int tid = threadIdx.x, nt = blockDim.x;
-  for (int idx = tid; idx < n * n; idx += nt) {
-    const int i = idx % n, j = idx / n;
-    W[i + j * ldw] = G[i + static_cast<long long>(j) * ldg];
-  }
-  __syncthreads();
-  __shared__ double s_rjj;
-  for (int j = 0; j < n; ++j) {
-    if (tid == 0) {
-      double d = W[j + j * ldw];
-      if (!(d > 0.0)) {  // breakdown (also catches NaN)
-        if (info) atomicCAS(info, 0, code), atomicCAS(info + 1, 0, j + 1);
-        d = 1.0;
-      }
-      s_rjj = sqrt(d);
-      W[j + j * ldw] = s_rjj;
-    }
-    __syncthreads();
-    const double rjj = s_rjj;
-    for (int i = j + 1 + tid; i < n; i += nt) W[j + i * ldw] /= rjj;  // row j of R
-    __syncthreads();
-    const int c = n - j - 1;
-    for (int idx = tid; idx < c * c; idx += nt) {
-      const int i = j + 1 + idx % c, i2 = j + 1 + idx / c;
-      if (i <= i2) W[i + i2 * ldw] -= W[j + i * ldw] * W[j + i2 * ldw];
-    }
-    __syncthreads();
-  }
-  // R (upper, zero below) and zero padding of R and Linv up to npad x npad
-  for (int idx = tid; idx < npad * npad; idx += nt) {
-    const int i = idx % npad, j = idx / npad;
-    R[i + static_cast<long long>(j) * ldr] = (i <= j && i < n && j < n) ? W[i + j * ldw] : 0.0;
-    if (i >= n || j >= n) Linv[i + static_cast<long long>(j) * ldl] = 0.0;
-  }
-  // Linv = R^{-T}: column c solves R^T x = e_c by forward substitution (one warp per column).
-  const int warp = tid >> 5, lane = tid & 31, nwarps = nt >> 5;
-  double* b = bbuf + warp * n;
-  for (int col = warp; col < n; col += nwarps) {
-    for (int i = lane; i < n; i += 32) b[i] = (i == col) ? 1.0 : 0.0;
-    __syncwarp();
-    for (int i = col; i < n; ++i) {
-      const double xi = b[i] / W[i + i * ldw];
-      __syncwarp();
-      if (lane == 0) b[i] = xi;
-      for (int i2 = i + 1 + lane; i2 < n; i2 += 32) b[i2] -= xi * W[i + i2 * ldw];  // (R^T)[i2][i] = R[i][i2]
-      __syncwarp();
-    }
-    for (int i = lane; i < n; i += 32) Linv[i + static_cast<long long>(col) * ldl] = (i >= col) ? b[i] : 0.0;
-    __syncwarp();
-  }
-}
-
-cudaError_t chol_inv(cudaStream_t st, const double* G, int ldg, int n, int npad, double* R, int ldr, double* Linv,
-                     int ldl, double* gwork, int* info, int info_code) {
-  const bool use_smem = n <= CHOL_SMEM_MAX_N;
-  const size_t smem = (use_smem ? static_cast<size_t>(n) * n : 0) * 8 + static_cast<size_t>(CHOL_THREADS / 32) * n * 8;
-  static bool attr = false;
-  if (!attr) {
-    cudaError_t e = cudaFuncSetAttribute(chol_inv_kernel, cudaFuncAttributeMaxDynamicSharedMemorySize, 220 * 1024);
-    if (e != cudaSuccess) return e;
-    attr = true;
-  }
-  if (smem > 220 * 1024) return cudaErrorInvalidValue;
-  chol_inv_kernel<<<1, CHOL_THREADS, smem, st>>>(G, ldg, n, R, ldr, Linv, ldl, gwork, info, info_code, npad);
-  count_launch();
-  return cudaGetLastError();
-}
-
-// ---------------------------------------------------------------------------------------------
 // Small dense product C = A*B (+C), general element strides, 64x64 tiles, FP64 FMA.
 // ---------------------------------------------------------------------------------------------
 __global__ void __launch_bounds__(256) small_gemm_kernel(int M, int N, int K, const double* __restrict__ A,
