@@ -43,9 +43,9 @@ def describe(c: dict) -> str:
 
 
 def row_split(m: int, nranks: int, rank: int):
-    base, extra = divmod(m, nranks)
-    r0 = rank * base + min(rank, extra)
-    return r0, r0 + base + (1 if rank < extra else 0)
+    from paper_conf_sc_maryykltd15_b200.partition import row_split as _rs
+
+    return _rs(m, nranks, rank)
 
 
 def gemm_flops(c: dict) -> float:

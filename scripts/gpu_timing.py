@@ -51,12 +51,12 @@ def main():
     out = {"cfg": args.cfg, "m": m, "n": n, "k": k, "p": p, "q": q}
     for nm, v in prof.items():
         if v["launches"]:
-            v["ms_per_rep"] = v["ms"] / args.reps
+            v["ms_per_rep"] = v["ms"] / max(args.reps, 1)
             v["tflops"] = v["flops"] / (v["ms"] * 1e9) if v["ms"] > 0 else 0
             out[nm] = v
-    gemm_ms = sum(prof[x]["ms"] for x in ("gemm_sample", "gemm_power_c", "gemm_power_b")) / args.reps
+    gemm_ms = sum(prof[x]["ms"] for x in ("gemm_sample", "gemm_power_c", "gemm_power_b")) / max(args.reps, 1)
     gemm_fl = 2.0 * ell * m * n * (1 + 2 * q)
-    out["gemm_tflops"] = gemm_fl / (gemm_ms * 1e9)
+    out["gemm_tflops"] = gemm_fl / (gemm_ms * 1e9) if gemm_ms > 0 else None
     print(json.dumps(out, indent=1))
     rs.destroy(h)
 
