@@ -67,6 +67,20 @@ RS_DEVINL void st_cluster_v2(uint32_t addr, double a, double b) {
 RS_DEVINL void mbar_arrive_remote(uint32_t cluster_bar_addr) {
   asm volatile("mbarrier.arrive.release.cluster.shared::cluster.b64 _, [%0];" ::"r"(cluster_bar_addr) : "memory");
 }
+// asynchronous DSMEM store that completes 16 transaction bytes on the destination CTA's mbarrier
+// (no fence, no arrive: the consumer's phase completes when all expected bytes have landed)
+RS_DEVINL void st_async_v2(uint32_t remote_addr, double a, double b, uint32_t remote_mbar) {
+  asm volatile("st.async.shared::cluster.mbarrier::complete_tx::bytes.v2.f64 [%0], {%1, %2}, [%3];" ::"r"(
+                   remote_addr),
+               "d"(a), "d"(b), "r"(remote_mbar)
+               : "memory");
+}
+// remote arrive with the default (.release.cta) semantics: used by MMA warps to hand a ring slot
+// back to a peer CTA -- the slot's smem reads have completed (their values were consumed by the
+// DMMAs issued before the arrive), and no cluster-scope MEMBAR lands on the MMA warps
+RS_DEVINL void mbar_arrive_remote_cta(uint32_t cluster_bar_addr) {
+  asm volatile("mbarrier.arrive.shared::cluster.b64 _, [%0];" ::"r"(cluster_bar_addr) : "memory");
+}
 RS_DEVINL void cluster_sync_all() {
   asm volatile("barrier.cluster.arrive.release.aligned;\n\tbarrier.cluster.wait.acquire.aligned;" ::: "memory");
 }

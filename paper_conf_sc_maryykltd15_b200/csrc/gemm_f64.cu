@@ -185,6 +185,11 @@ cudaError_t gemm_kc(cudaStream_t st, int M, int N, long long K, const View2D& Lv
     a.tag = phx.tag;
     a.row_offset = phx.row_offset;
     a.ell = phx.ell;
+    static const int gen_mode = [] {  // RS_PHILOX_GENMODE: cost experiments only (results invalid)
+      const char* v = getenv("RS_PHILOX_GENMODE");
+      return v ? atoi(v) : 0;
+    }();
+    a.gen_mode = gen_mode;
   }
   CUtensorMap tR, tL;
   if (!make_tmap(&tR, Rv, 16, NT)) return cudaErrorInvalidValue;

@@ -53,6 +53,7 @@ struct GemmArgs {
   uint32_t tag;
   long long row_offset;
   int ell;
+  int gen_mode;  // 0 = Philox + RS-BM32 (production); 1, 2 = generation-cost experiments only
 };
 
 template <int MFW, bool PHILOX>
@@ -212,10 +213,12 @@ __global__ void __launch_bounds__(GEMM_THREADS, 1)
 // rows [c*MT/CS, (c+1)*MT/CS) and stores them into every CTA's ring through distributed shared
 // memory, so each Omega value is generated once per CS*128 columns of A.
 // ------------------------------------------------------------------------------------------
-constexpr int PHX_GEN_WARPS = 4;
+// Two generator warpgroups (2 warps per SM sub-partition): Philox/RS-BM32 is a long dependent
+// chain per Omega block, so generation is latency-bound; a second warp per sub-partition hides it.
+constexpr int PHX_GEN_WARPS = 8;
 constexpr int PHX_THREADS = (PHX_GEN_WARPS + NCONS) * 32;
 constexpr int PHX_GEN_REGS = 56;
-constexpr int PHX_MMA_REGS = 224;  // 4*32*56 + 8*32*224 = 64512 <= 65536
+constexpr int PHX_MMA_REGS = 200;  // 8*32*56 + 8*32*200 = 65536
 
 template <int MFW, int CS>
 __global__ void __launch_bounds__(PHX_THREADS, 1)
@@ -240,7 +243,7 @@ __global__ void __launch_bounds__(PHX_THREADS, 1)
   if (threadIdx.x == 0) {
 #pragma unroll
     for (int s = 0; s < NSTAGE; ++s) {
-      mbar_init(&full[s], 1 + PHX_GEN_WARPS * CS);
+      mbar_init(&full[s], 1 + PHX_GEN_WARPS);  // TMA producer + local generator warps (+ peers' tx bytes)
       mbar_init(&empty[s], NCONS * CS);
     }
     fence_mbar_init();
@@ -262,16 +265,11 @@ __global__ void __launch_bounds__(PHX_THREADS, 1)
     for (int it = 0; it < nk; ++it) {
       const int s = it % NSTAGE;
       if (it >= NSTAGE) {
-        if (lane == 0) {
-          if (CS > 1)
-            mbar_wait_cluster(&empty[s], ((it / NSTAGE) - 1) & 1);
-          else
-            mbar_wait(&empty[s], ((it / NSTAGE) - 1) & 1);
-        }
+        if (lane == 0) mbar_wait(&empty[s], ((it / NSTAGE) - 1) & 1);
         __syncwarp();
       }
       if (g == 0) {
-        mbar_arrive_expect_tx(&full[s], SM::R_BYTES);
+        mbar_arrive_expect_tx(&full[s], SM::R_BYTES + (MT - ROWS) * KT * 8);  // A tile + peers' Omega rows
         tma_load_2d(sR + s * SM::R_BYTES, &tmR, &full[s], static_cast<int>(kb + static_cast<long long>(it) * KT), n0);
       }
       const long long j0 = a.row_offset + kb + static_cast<long long>(it) * KT;  // global row of A
@@ -283,7 +281,17 @@ __global__ void __launch_bounds__(PHX_THREADS, 1)
         const int gi = m0 + lrow;
         double* dst = reinterpret_cast<double*>(sL + s * SM::L_BYTES) + lrow * PHX_LD + 4 * q;
         double v0 = 0.0, v1 = 0.0, v2 = 0.0, v3 = 0.0;
-        if (gi < a.ell) {
+        if (a.gen_mode != 0) {  // experiments: 1 = Philox words only, 2 = no generation
+          if (a.gen_mode == 1 && gi < a.ell) {
+            uint32_t c0 = static_cast<uint32_t>(t0 + q), c1 = static_cast<uint32_t>(gi), c2 = a.tag,
+                     c3 = static_cast<uint32_t>((t0 + q) >> 32);
+            philox4x32_10(c0, c1, c2, c3, a.key);
+            v0 = static_cast<int>(c0) * 0x1p-31, v1 = static_cast<int>(c1) * 0x1p-31;
+            v2 = static_cast<int>(c2) * 0x1p-31, v3 = static_cast<int>(c3) * 0x1p-31;
+          } else if (gi < a.ell) {
+            v0 = v1 = v2 = v3 = 1.0;
+          }
+        } else if (gi < a.ell) {
           const float4 z = omega_block4f(static_cast<uint32_t>(gi), t0 + q, a.tag, a.key);
           if (o == 0) {
             v0 = z.x, v1 = z.y, v2 = z.z, v3 = z.w;
@@ -297,22 +305,21 @@ __global__ void __launch_bounds__(PHX_THREADS, 1)
         }
         reinterpret_cast<double2*>(dst)[0] = make_double2(v0, v1);
         reinterpret_cast<double2*>(dst)[1] = make_double2(v2, v3);
-        if (CS > 1) {
+        if (CS > 1) {  // the same 32 bytes into every peer's ring; completes tx on its full[s]
           const uint32_t sa = smem_u32(dst);
+          const uint32_t fb = smem_u32(&full[s]);
 #pragma unroll
           for (int pc = 1; pc < CS; ++pc) {
-            const uint32_t ra = mapa_shared(sa, (crank + pc) % CS);
-            st_cluster_v2(ra, v0, v1);
-            st_cluster_v2(ra + 16, v2, v3);
+            const uint32_t peer = (crank + pc) % CS;
+            const uint32_t ra = mapa_shared(sa, peer);
+            const uint32_t rb = mapa_shared(fb, peer);
+            st_async_v2(ra, v0, v1, rb);
+            st_async_v2(ra + 16, v2, v3, rb);
           }
         }
       }
       __syncwarp();
-      if (lane == 0) {
-        mbar_arrive(&full[s]);
-#pragma unroll
-        for (int pc = 1; pc < CS; ++pc) mbar_arrive_remote(mapa_shared(smem_u32(&full[s]), (crank + pc) % CS));
-      }
+      if (lane == 0) mbar_arrive(&full[s]);
     }
   } else {
     // ------------------------- MMA warpgroups -------------------------
@@ -332,10 +339,9 @@ __global__ void __launch_bounds__(PHX_THREADS, 1)
     };
     for (int it = 0; it < nk; ++it) {
       const int s = it % NSTAGE;
-      if (CS > 1)
-        mbar_wait_cluster(&full[s], (it / NSTAGE) & 1);
-      else
-        mbar_wait(&full[s], (it / NSTAGE) & 1);
+      // CTA-scope wait: the slot's data is in this CTA's shared memory (no L1 to invalidate);
+      // the remote generators' stores are ordered before their release.cluster arrive
+      mbar_wait(&full[s], (it / NSTAGE) & 1);
       const double* Ls = reinterpret_cast<const double*>(sL + s * SM::L_BYTES);
       const unsigned char* Rs = sR + s * SM::R_BYTES;
       kc_stage_mma<MFW>(
@@ -346,7 +352,7 @@ __global__ void __launch_bounds__(PHX_THREADS, 1)
       if (lane == 0) {
         mbar_arrive(&empty[s]);
 #pragma unroll
-        for (int pc = 1; pc < CS; ++pc) mbar_arrive_remote(mapa_shared(smem_u32(&empty[s]), (crank + pc) % CS));
+        for (int pc = 1; pc < CS; ++pc) mbar_arrive_remote_cta(mapa_shared(smem_u32(&empty[s]), (crank + pc) % CS));
       }
     }
     kc_store<MFW>(acc, a.out, m0, n0, wn, kk, rowL);
