@@ -1,18 +1,19 @@
 // Cholesky factor of a Gram matrix and its inverse in one pass: CholQR steps (ii)-(iii)
 // ("R^T R := G, R upper-triangular with non-negative diagonal; Q = R^{-T} B").
 //
-// Right-looking elimination on the packed upper triangle S of G with the same row operations
-// applied to an identity E (E becomes the unit-lower L^{-1} up to row scaling), one
-// __syncthreads per pivot: at step k every thread updates the elements it owns,
-//     S[i][j] -= S[k][i] S[k][j] / d_k          (k < i <= j)
-//     E[i][c] -= S[k][i] / d_k * E[k][c]         (c <= k < i)
-// then R[k][j] = S[k][j] / sqrt(d_k) and Linv = R^{-T} has rows E[i][:] / sqrt(d_i).
-// Both triangles are stored ROW-packed so that row k (read by every thread at step k) is
-// contiguous: consecutive lanes own consecutive elements of one row -> conflict-free LDS and
-// broadcasts.  One CTA of 1024 threads; packed triangles in shared memory for n <= 128 (element
-// coordinates kept in registers), in the L2-resident workspace otherwise.  A pivot d_k <= 0 or
-// NaN is a CholQR breakdown: it is reported through *info (LAPACK potrf-style 1-based column) and
-// replaced by 1 so no NaN propagates.
+// Right-looking LDL^T elimination of G with the same row operations applied to an identity E,
+// which becomes L_unit^{-1}:   at pivot k, for every row i > k,
+//     S[i][j] -= S[k][i] S[k][j] / d_k          (j >= i)
+//     E[i][c] -= S[k][i] / d_k * E[k][c]         (c <= k, E[k][k] = 1)
+// Then R[i][j] = S[i][j] / sqrt(d_i) and Linv = R^{-T} = D^{-1/2} E.  S (upper) and E (strict
+// lower; its unit diagonal is implicit) share one n x n array M.
+//
+// One CTA of 1024 threads.  Each thread owns strips of 8 consecutive columns of a row and keeps
+// them in registers (n <= 128); row k is published to shared memory by its owners right after
+// step k-1, so each pivot costs one __syncthreads and every active thread does ~16 FMAs per step
+// on registers with row k read as broadcast LDS.128.  For n > 128 the same schedule runs on an
+// L2-resident copy in the workspace.  A pivot d_k <= 0 or NaN is a CholQR breakdown: reported
+// through *info (LAPACK potrf-style 1-based column) and replaced by 1 so no NaN propagates.
 #include <cstdio>
 
 #include "common.cuh"
@@ -22,96 +23,130 @@ namespace rs {
 
 constexpr int CH_THREADS = 1024;
 constexpr int CH_SMEM_MAX_N = 128;
-constexpr int CH_MAXE = (CH_SMEM_MAX_N * (CH_SMEM_MAX_N + 1) / 2 + CH_THREADS - 1) / CH_THREADS;  // 9
+constexpr int CH_SW = 8;                                                          // strip width
+constexpr int CH_MAXS = (CH_SMEM_MAX_N * (CH_SMEM_MAX_N / CH_SW) + CH_THREADS - 1) / CH_THREADS;  // 2
 
-// upper triangle, row-packed: (i, j), i <= j < n, at up(i) + j - i,  up(i) = i*n - i*(i-1)/2
-RS_DEVINL int up_off(int i, int n) { return i * n - i * (i - 1) / 2; }
-RS_DEVINL void up_decode(int e, int n, int& i, int& j) {
-  const double b = 2.0 * n + 1.0;
-  int ii = static_cast<int>((b - sqrt(b * b - 8.0 * e)) * 0.5);
-  if (ii < 0) ii = 0;
-  while (ii > 0 && up_off(ii, n) > e) --ii;
-  while (ii + 1 < n && up_off(ii + 1, n) <= e) ++ii;
-  i = ii;
-  j = ii + (e - up_off(ii, n));
-}
-// lower triangle, row-packed: (r, c), c <= r, at r(r+1)/2 + c
-RS_DEVINL int lo_off(int r) { return r * (r + 1) / 2; }
-RS_DEVINL void lo_decode(int e, int& r, int& c) {
-  int rr = static_cast<int>((sqrt(8.0 * e + 1.0) - 1.0) * 0.5);
-  while (lo_off(rr + 1) <= e) ++rr;
-  while (lo_off(rr) > e) --rr;
-  r = rr;
-  c = e - lo_off(rr);
-}
-
-template <bool SMEM>
-__global__ void __launch_bounds__(CH_THREADS) chol_inv_kernel(const double* __restrict__ G, int ldg, int n,
-                                                               double* __restrict__ R, int ldr,
-                                                               double* __restrict__ Linv, int ldl,
-                                                               double* __restrict__ gwork, int* info, int code,
-                                                               int npad) {
+template <bool SMALL>
+__global__ void __launch_bounds__(CH_THREADS, 1) chol_inv_kernel(const double* __restrict__ G, int ldg, int n,
+                                                                  double* __restrict__ R, int ldr,
+                                                                  double* __restrict__ Linv, int ldl,
+                                                                  double* __restrict__ gwork, int* info, int code,
+                                                                  int npad) {
   extern __shared__ double sm[];
-  const int T = n * (n + 1) / 2;
-  double* S = SMEM ? sm : gwork;
-  double* E = S + T;
+  __shared__ double s_inv[CH_SMEM_MAX_N > 512 ? CH_SMEM_MAX_N : 512];
   const int tid = threadIdx.x;
+  const int ns = (n + CH_SW - 1) / CH_SW;  // strips per row
+  const int ldm = ns * CH_SW;              // row pitch of M (multiple of 8 -> 64-byte aligned strips)
+  double* M = SMALL ? sm : gwork;
+  const int nstrips = n * ns;
 
-  constexpr int NE = SMEM ? CH_MAXE : 1;
-  int si[NE], sj[NE], er[NE], ec[NE];
-  if (SMEM) {
-#pragma unroll
-    for (int s = 0; s < NE; ++s) {
-      const int e = tid + s * CH_THREADS;
-      si[s] = sj[s] = er[s] = ec[s] = -1;
-      if (e < T) {
-        up_decode(e, n, si[s], sj[s]);
-        lo_decode(e, er[s], ec[s]);
-      }
+  auto pivot_inv = [&](int k, double d) {  // by the owner of M[k][k]
+    if (!(d > 0.0)) {
+      if (info) atomicCAS(info, 0, code), atomicCAS(info + 1, 0, k + 1);
+      d = 1.0;
     }
-  }
-  for (int e = tid; e < T; e += CH_THREADS) {
-    int i, j, r, c;
-    up_decode(e, n, i, j);
-    lo_decode(e, r, c);
-    S[e] = G[i + static_cast<long long>(j) * ldg];
-    E[e] = (r == c) ? 1.0 : 0.0;
-  }
-  __syncthreads();
+    s_inv[k] = 1.0 / d;
+  };
 
-  for (int k = 0; k < n; ++k) {
-    const double* Sk = S + up_off(k, n) - k;  // Sk[j] = S[k][j], j >= k
-    const double* Ek = E + lo_off(k);         // Ek[c] = E[k][c], c <= k
-    const double dk = Sk[k];
-    const double inv = 1.0 / (dk > 0.0 ? dk : 1.0);
-    if (tid == 0 && !(dk > 0.0) && info) atomicCAS(info, 0, code), atomicCAS(info + 1, 0, k + 1);
-    if (SMEM) {
+  if (SMALL) {
+    double reg[CH_MAXS][CH_SW];
+    int ri[CH_MAXS], rj[CH_MAXS];
 #pragma unroll
-      for (int s = 0; s < NE; ++s) {
-        const int e = tid + s * CH_THREADS;
-        if (si[s] > k) S[e] -= Sk[si[s]] * Sk[sj[s]] * inv;
-        if (er[s] > k && ec[s] <= k) E[e] -= Sk[er[s]] * inv * Ek[ec[s]];
+    for (int u = 0; u < CH_MAXS; ++u) {
+      const int id = tid + u * CH_THREADS;
+      ri[u] = id < nstrips ? id / ns : n;  // n = no strip
+      rj[u] = id < nstrips ? (id % ns) * CH_SW : 0;
+#pragma unroll
+      for (int e = 0; e < CH_SW; ++e) {
+        const int j = rj[u] + e;
+        reg[u][e] = (ri[u] < n && j < n) ? (j >= ri[u] ? G[ri[u] + static_cast<long long>(j) * ldg] : 0.0) : 0.0;
       }
-    } else {
-      for (int e = tid; e < T; e += CH_THREADS) {
-        int i, j, r, c;
-        up_decode(e, n, i, j);
-        lo_decode(e, r, c);
-        if (i > k) S[e] -= Sk[i] * Sk[j] * inv;
-        if (r > k && c <= k) E[e] -= Sk[r] * inv * Ek[c];
+      if (ri[u] == 0) {  // publish row 0
+#pragma unroll
+        for (int e = 0; e < CH_SW; ++e) M[rj[u] + e] = reg[u][e];
+        if (rj[u] == 0) pivot_inv(0, reg[u][0]);
       }
     }
     __syncthreads();
+    for (int k = 0; k < n - 1; ++k) {
+      const double* Mk = M + static_cast<long long>(k) * ldm;
+      const double inv = s_inv[k];
+#pragma unroll
+      for (int u = 0; u < CH_MAXS; ++u) {
+        const int i = ri[u];
+        if (i <= k || i >= n) continue;
+        const double l = Mk[i] * inv;  // S[k][i] / d_k
+        const double2* rk = reinterpret_cast<const double2*>(Mk + rj[u]);
+#pragma unroll
+        for (int e2 = 0; e2 < CH_SW / 2; ++e2) {
+          const double2 m2 = rk[e2];
+#pragma unroll
+          for (int h = 0; h < 2; ++h) {
+            const int e = 2 * e2 + h;
+            const int j = rj[u] + e;
+            const double mkj = h ? m2.y : m2.x;
+            if (j >= i)
+              reg[u][e] = fma(-l, mkj, reg[u][e]);                     // S part
+            else if (j <= k)
+              reg[u][e] = fma(-l, j == k ? 1.0 : mkj, reg[u][e]);      // E part (E[k][k] = 1)
+          }
+        }
+        if (i == k + 1) {  // row k+1 is final: publish it and its pivot
+          double* dst = M + static_cast<long long>(i) * ldm + rj[u];
+#pragma unroll
+          for (int e = 0; e < CH_SW; ++e) dst[e] = reg[u][e];
+          if (rj[u] <= i && i < rj[u] + CH_SW) {
+#pragma unroll
+            for (int e = 0; e < CH_SW; ++e)
+              if (rj[u] + e == i) pivot_inv(i, reg[u][e]);
+          }
+        }
+      }
+      __syncthreads();
+    }
+  } else {
+    // large n: M lives in the L2-resident workspace, updated in place
+    for (int id = tid; id < nstrips; id += CH_THREADS) {
+      const int i = id / ns, j0 = (id % ns) * CH_SW;
+      for (int e = 0; e < CH_SW; ++e) {
+        const int j = j0 + e;
+        M[static_cast<long long>(i) * ldm + j] = (j < n && j >= i) ? G[i + static_cast<long long>(j) * ldg] : 0.0;
+      }
+    }
+    __syncthreads();
+    if (tid == 0) pivot_inv(0, M[0]);
+    __syncthreads();
+    for (int k = 0; k < n - 1; ++k) {
+      const double* Mk = M + static_cast<long long>(k) * ldm;
+      const double inv = s_inv[k];
+      for (int id = tid; id < nstrips; id += CH_THREADS) {
+        const int i = id / ns, j0 = (id % ns) * CH_SW;
+        if (i <= k) continue;
+        const double l = Mk[i] * inv;
+        double* row = M + static_cast<long long>(i) * ldm + j0;
+        for (int e = 0; e < CH_SW; ++e) {
+          const int j = j0 + e;
+          if (j >= n) break;
+          if (j >= i)
+            row[e] = fma(-l, Mk[j], row[e]);
+          else if (j <= k)
+            row[e] = fma(-l, j == k ? 1.0 : Mk[j], row[e]);
+        }
+        if (i == k + 1 && j0 <= i && i < j0 + CH_SW) pivot_inv(i, row[i - j0]);
+      }
+      __syncthreads();
+    }
   }
-  // R (upper, zero below) and Linv = R^{-T} (lower, zero above), zero-padded to npad x npad
+  // R (upper, zero below) and Linv = D^{-1/2} E (lower, unit diagonal scaled), zero-padded
   for (int idx = tid; idx < npad * npad; idx += CH_THREADS) {
     const int i = idx % npad, j = idx / npad;
     double rv = 0.0, lv = 0.0;
     if (i < n && j < n) {
-      const double di = S[up_off(i, n)];
-      const double ri = sqrt(di > 0.0 ? di : 1.0);
-      if (i <= j) rv = S[up_off(i, n) + j - i] / ri;
-      if (j <= i) lv = E[lo_off(i) + j] / ri;
+      const double rs = sqrt(s_inv[i]);  // 1/sqrt(d_i)
+      const double mij = M[static_cast<long long>(i) * ldm + j];
+      if (i <= j) rv = mij * rs;
+      if (j < i) lv = mij * rs;
+      if (j == i) lv = rs;
     }
     R[i + static_cast<long long>(j) * ldr] = rv;
     Linv[i + static_cast<long long>(j) * ldl] = lv;
@@ -121,12 +156,14 @@ __global__ void __launch_bounds__(CH_THREADS) chol_inv_kernel(const double* __re
 cudaError_t chol_inv(cudaStream_t st, const double* G, int ldg, int n, int npad, double* R, int ldr, double* Linv,
                      int ldl, double* gwork, int* info, int info_code) {
   if (n <= 0) return cudaSuccess;
-  const size_t work = static_cast<size_t>(n) * (n + 1) * 8;  // both packed triangles
+  if (n > 512) return cudaErrorInvalidValue;
+  const int ldm = (n + CH_SW - 1) / CH_SW * CH_SW;
+  const size_t work = static_cast<size_t>(n) * ldm * 8;
   if (n <= CH_SMEM_MAX_N) {
     static bool attr = false;
     if (!attr) {
       cudaError_t e = cudaFuncSetAttribute(chol_inv_kernel<true>, cudaFuncAttributeMaxDynamicSharedMemorySize,
-                                           CH_SMEM_MAX_N * (CH_SMEM_MAX_N + 1) * 8);
+                                           CH_SMEM_MAX_N * CH_SMEM_MAX_N * 8);
       if (e != cudaSuccess) return e;
       attr = true;
     }

@@ -3,26 +3,29 @@
 // remaining column with the largest residual 2-norm (Sec. 2).
 //
 // B200 design: one persistent cooperative kernel.  The columns of B are distributed over NB CTAs
-// and stay resident in shared memory for all k steps; per step each CTA (A) recomputes the
-// residual norms of its active columns with warp-shuffle reductions (reading R5: exact
-// recomputation instead of downdating, P:L189-192/L212-217 -- every column is touched by the
-// trailing update anyway, so the recompute costs no extra pass) and publishes its best candidate
-// column, (grid barrier), (B) every CTA reads all candidates in parallel, picks the same global
-// pivot (largest norm, ties -> lowest original index), forms the dlarfg reflector from the
-// published column and applies it to its own columns.  One grid barrier and two dependent L2
-// round trips per step; pivots and R̂ rows are final as soon as they are produced.
+// (<= 256 columns each) and stay resident in shared memory for all k steps.  Four lanes own one
+// column (rows i = q mod 4), so residual norms and reflector dot products are short independent
+// chains plus two shuffles.  Per step each CTA (A) recomputes the residual norms of its active
+// columns (reading R5: exact recomputation instead of downdating, P:L189-192/L212-217 -- every
+// column is touched by the trailing update anyway) and publishes its best candidate column,
+// (grid barrier), (B) every CTA reads all candidates in parallel, picks the same global pivot
+// (largest norm, ties -> lowest original index), forms the dlarfg reflector from the published
+// column and applies it to its own columns.  Pivots and R̂ rows are final as soon as they are
+// produced; perm (LAPACK swap order) is assembled from the pivot sequence afterwards.
 #include <algorithm>
 #include <cstdio>
+#include <cstdlib>
 
 #include "common.cuh"
 #include "internal.h"
 
 namespace rs {
 
-constexpr int QR_THREADS = 512;
+constexpr int QR_THREADS = 1024;
 constexpr int QR_WARPS = QR_THREADS / 32;
-constexpr int QR_MAX_COLS = 1024;    // columns per CTA (smem flags)
-constexpr int QR_COLS_TARGET = 160;  // preferred columns per CTA: few CTAs -> cheap grid barrier
+constexpr int QR_LANES = 4;                            // lanes per column
+constexpr int QR_MAX_COLS = QR_THREADS / QR_LANES;     // 256 columns per CTA
+constexpr size_t QR_SMEM_MAX = 200 * 1024;
 
 struct QrCand {
   double best;    // squared residual norm of the CTA's best active column (-1 if none)
@@ -34,7 +37,7 @@ struct QrCand {
 struct QrWork {
   unsigned int count;  // monotone grid-barrier counter
   unsigned int pad[3];
-  // followed by: QrCand cand[2][NB]; double candcol[2][NB][ell]; int64 inv[n]
+  // followed by: QrCand cand[2][NB]; double candcol[2][NB][ell]; int64 piv[n]; int64 pos[n]
 };
 
 RS_DEVINL bool better(double a, long long ia, double b, long long ib) {
@@ -58,111 +61,111 @@ RS_DEVINL void grid_sync_count(unsigned int* count, unsigned int target) {
   __syncthreads();
 }
 
-// (value, index, owner) argmax with ties to the lowest index, across the CTA
+// (value, index, owner) argmax with ties to the lowest index
 struct Arg {
   double v;
   long long i;
   int b;
 };
-RS_DEVINL Arg warp_argmax(Arg a) {
+RS_DEVINL Arg shfl_arg(const Arg& a, int o) {
+  return Arg{__shfl_xor_sync(0xffffffffu, a.v, o), __shfl_xor_sync(0xffffffffu, a.i, o),
+             __shfl_xor_sync(0xffffffffu, a.b, o)};
+}
+// warp-wide best and runner-up (value only) of per-lane (best a, runner-up sec)
+RS_DEVINL void warp_top2(Arg& a, double& sec) {
 #pragma unroll
   for (int o = 16; o > 0; o >>= 1) {
-    Arg x{__shfl_xor_sync(0xffffffffu, a.v, o), __shfl_xor_sync(0xffffffffu, a.i, o),
-          __shfl_xor_sync(0xffffffffu, a.b, o)};
-    if (better(x.v, x.i, a.v, a.i)) a = x;
+    const Arg x = shfl_arg(a, o);
+    const double xs = __shfl_xor_sync(0xffffffffu, sec, o);
+    sec = fmax(sec, xs);
+    if (better(x.v, x.i, a.v, a.i)) {
+      if (a.i >= 0) sec = fmax(sec, a.v);
+      a = x;
+    } else if (x.i >= 0) {
+      sec = fmax(sec, x.v);
+    }
   }
-  return a;
-}
-RS_DEVINL double warp_max(double v) {
-#pragma unroll
-  for (int o = 16; o > 0; o >>= 1) v = fmax(v, __shfl_xor_sync(0xffffffffu, v, o));
-  return v;
 }
 
 __global__ void __launch_bounds__(QR_THREADS, 1)
     qrcp_kernel(const double* __restrict__ B, int ldb, int ell, long long n, int k, QrWork* work, int NB,
-                int cols_per, int64_t* __restrict__ perm, double* __restrict__ Rho, int ldr,
-                double* __restrict__ gaps, int* info) {
+                int cols_per, int ldw, int64_t* __restrict__ Rho_piv, double* __restrict__ Rho, int ldr,
+                double* __restrict__ gaps, int* info, long long* tbuf) {
   extern __shared__ double sh[];
   const int blk = blockIdx.x;
+  const int tid = threadIdx.x, warp = tid >> 5, lane = tid & 31;
   const long long c0 = static_cast<long long>(blk) * cols_per;
   const long long c1 = (c0 + cols_per < n) ? c0 + cols_per : n;
   const int nc = c1 > c0 ? static_cast<int>(c1 - c0) : 0;
-  double* W = sh;                                       // nc x ell, column c at W + c*ell
-  double* v = W + static_cast<size_t>(cols_per) * ell;  // Householder vector (ell)
-  __shared__ unsigned char active[QR_MAX_COLS];
+  double* W = sh;                                       // column c at W + c*ldw (ldw = 4 mod 16)
+  double* v = W + static_cast<size_t>(cols_per) * ldw;  // Householder vector (ell)
   __shared__ Arg s_warg[QR_WARPS];
   __shared__ double s_wsec[QR_WARPS];
-  __shared__ double s_tau, s_beta, s_gbest, s_gsecond;
+  __shared__ double s_tau, s_beta, s_gbest, s_gsecond, s_den;
   __shared__ long long s_gidx;
   __shared__ int s_gblk, s_bloc;
 
   QrCand* cand = reinterpret_cast<QrCand*>(work + 1);
   double* candcol = reinterpret_cast<double*>(cand + 2 * NB);
-  int64_t* inv = reinterpret_cast<int64_t*>(candcol + 2 * static_cast<size_t>(NB) * ell);
+  int64_t* piv = Rho_piv;
 
-  const int tid = threadIdx.x, warp = tid >> 5, lane = tid & 31;
   for (int idx = tid; idx < nc * ell; idx += QR_THREADS) {
     const int c = idx / ell, i = idx % ell;
-    W[c * ell + i] = B[i + (c0 + c) * static_cast<long long>(ldb)];
+    W[c * ldw + i] = B[i + (c0 + c) * static_cast<long long>(ldb)];
   }
-  for (int c = tid; c < nc; c += QR_THREADS) active[c] = 1;
+  const int mc = tid / QR_LANES, q = tid % QR_LANES;  // my column and row phase
+  bool active = mc < nc;
+  double* col = W + mc * ldw;
   __syncthreads();
 
+#define QT(ph) \
+  if (tbuf && blk == 0 && tid == 0) tbuf[j * 8 + (ph)] = clock64();
   for (int j = 0; j < k; ++j) {
     const int par = j & 1;
-    // ---- (A) residual norms of the local active columns; local best and runner-up ----
-    Arg wb{-1.0, -1, -1};
-    double ws = -1.0;
-    for (int c = warp; c < nc; c += QR_WARPS) {
-      if (!active[c]) continue;
-      double s = 0.0;
-      for (int i = j + lane; i < ell; i += 32) {
-        const double x = W[c * ell + i];
-        s = fma(x, x, s);
-      }
-#pragma unroll
-      for (int o = 16; o > 0; o >>= 1) s += __shfl_xor_sync(0xffffffffu, s, o);
-      const long long gi = c0 + c;
-      if (better(s, gi, wb.v, wb.i)) {
-        ws = fmax(ws, wb.v);
-        wb = Arg{s, gi, c};
-      } else {
-        ws = fmax(ws, s);
-      }
-    }
-    if (lane == 0) {
-      s_warg[warp] = wb;
-      s_wsec[warp] = ws;
-    }
-    __syncthreads();
-    if (warp == 0) {
-      Arg a = lane < QR_WARPS ? s_warg[lane] : Arg{-1.0, -1, -1};
-      const Arg best = warp_argmax(a);
-      double sec = lane < QR_WARPS ? s_wsec[lane] : -1.0;
-      if (lane < QR_WARPS && a.i != best.i) sec = fmax(sec, a.v);
-      sec = warp_max(sec);
+    QT(0)
+    // ---- (A) residual norms of the local active columns; CTA best and runner-up ----
+    double s = 0.0;
+    if (active)
+      for (int i = j + q; i < ell; i += QR_LANES) s = fma(col[i], col[i], s);
+    s += __shfl_xor_sync(0xffffffffu, s, 1);
+    s += __shfl_xor_sync(0xffffffffu, s, 2);
+    {
+      Arg a = (active && q == 0) ? Arg{s, c0 + mc, mc} : Arg{-1.0, -1, -1};
+      double sec = -1.0;
+      warp_top2(a, sec);
       if (lane == 0) {
-        QrCand cd;
-        cd.best = best.v;
-        cd.second = sec;
-        cd.idx = best.i;
-        cd.pad = 0;
-        cand[par * NB + blk] = cd;
-        s_bloc = best.i >= 0 ? best.b : -1;
+        s_warg[warp] = a;
+        s_wsec[warp] = sec;
       }
+      __syncthreads();
+      if (warp == 0) {
+        Arg x = s_warg[lane];
+        double xs = s_wsec[lane];
+        warp_top2(x, xs);
+        if (lane == 0) {
+          QrCand cd;
+          cd.best = x.v;
+          cd.second = xs;
+          cd.idx = x.i;
+          cd.pad = 0;
+          cand[par * NB + blk] = cd;
+          s_bloc = x.i >= 0 ? x.b : -1;
+        }
+      }
+      __syncthreads();
     }
-    __syncthreads();
+    QT(1)
     if (s_bloc >= 0)
       for (int i = j + tid; i < ell; i += QR_THREADS)
-        candcol[(static_cast<size_t>(par) * NB + blk) * ell + i] = W[s_bloc * ell + i];
+        candcol[(static_cast<size_t>(par) * NB + blk) * ell + i] = W[s_bloc * ldw + i];
     grid_sync_count(&work->count, static_cast<unsigned int>(j + 1) * NB);
+    QT(2)
 
     // ---- (B) global pivot: every CTA reads all candidates in parallel ----
-    {
+    if (warp == 0) {
       Arg a{-1.0, -1, -1};
       double sec = -1.0;
-      for (int b = tid; b < NB; b += QR_THREADS) {
+      for (int b = lane; b < NB; b += 32) {
         const long long ci = __ldcg(&cand[par * NB + b].idx);
         const double cb = __ldcg(&cand[par * NB + b].best);
         const double cs = __ldcg(&cand[par * NB + b].second);
@@ -174,57 +177,39 @@ __global__ void __launch_bounds__(QR_THREADS, 1)
           sec = fmax(sec, cb);
         }
       }
-      const Arg wbest = warp_argmax(a);
-      if (a.i >= 0 && a.i != wbest.i) sec = fmax(sec, a.v);
-      sec = warp_max(sec);
+      warp_top2(a, sec);
       if (lane == 0) {
-        s_warg[warp] = wbest;
-        s_wsec[warp] = sec;
+        s_gbest = a.v;
+        s_gsecond = sec;
+        s_gidx = a.i;
+        s_gblk = a.b;
       }
-      __syncthreads();
-      if (warp == 0) {
-        Arg x = lane < QR_WARPS ? s_warg[lane] : Arg{-1.0, -1, -1};
-        const Arg g = warp_argmax(x);
-        double s2 = lane < QR_WARPS ? s_wsec[lane] : -1.0;
-        if (lane < QR_WARPS && x.i >= 0 && x.i != g.i) s2 = fmax(s2, x.v);
-        s2 = warp_max(s2);
-        if (lane == 0) {
-          s_gbest = g.v;
-          s_gsecond = s2;
-          s_gidx = g.i;
-          s_gblk = g.b;
-        }
-      }
-      __syncthreads();
     }
+    __syncthreads();
+    QT(3)
     const int gblk = s_gblk;
     const long long gidx = s_gidx;
     const int len = ell - j;
     for (int i = tid; i < len; i += QR_THREADS)
       v[i] = __ldcg(&candcol[(static_cast<size_t>(par) * NB + (gblk < 0 ? 0 : gblk)) * ell + j + i]);
     __syncthreads();
+    QT(4)
     if (warp == 0) {  // dlarfg on x = v[0..len)
       double xs = 0.0;
       for (int i = 1 + lane; i < len; i += 32) xs = fma(v[i], v[i], xs);
 #pragma unroll
       for (int o = 16; o > 0; o >>= 1) xs += __shfl_xor_sync(0xffffffffu, xs, o);
-      const double alpha = v[0];
-      double tau = 0.0, beta = alpha;
-      if (gblk >= 0 && xs > 0.0) {
-        const double h = sqrt(fma(alpha, alpha, xs));
-        beta = alpha >= 0.0 ? -h : h;
-        tau = (beta - alpha) / beta;
-      }
-      __syncwarp();
-      if (tau != 0.0) {
-        const double den = alpha - beta;
-        for (int i = 1 + lane; i < len; i += 32) v[i] = v[i] / den;
-      }
-      __syncwarp();
       if (lane == 0) {
-        v[0] = 1.0;
+        const double alpha = v[0];
+        double tau = 0.0, beta = alpha;
+        if (gblk >= 0 && xs > 0.0) {
+          const double h = sqrt(fma(alpha, alpha, xs));
+          beta = alpha >= 0.0 ? -h : h;
+          tau = (beta - alpha) / beta;
+        }
         s_tau = tau;
         s_beta = beta;
+        s_den = alpha - beta;
         if (gblk < 0 || !(s_gbest > 0.0)) {
           if (info && blk == 0) atomicCAS(info, 0, 6 /* RS_ERR_RANK_DEFICIENT */), atomicCAS(info + 1, 0, j + 1);
         }
@@ -232,41 +217,44 @@ __global__ void __launch_bounds__(QR_THREADS, 1)
     }
     __syncthreads();
     const double tau = s_tau, beta = s_beta;
+    if (tau != 0.0)
+      for (int i = 1 + tid; i < len; i += QR_THREADS) v[i] = v[i] / s_den;
+    __syncthreads();
+    QT(5)
     // ---- apply H = I - tau v v^T to the local active columns; retire the pivot column ----
-    for (int c = warp; c < nc; c += QR_WARPS) {
-      if (!active[c]) continue;
-      const long long gi = c0 + c;
-      double* col = W + c * ell;
-      if (gi == gidx) {
-        for (int i = lane; i < k; i += 32) {
+    {
+      const long long gi = c0 + mc;
+      const bool is_piv = active && gi == gidx;
+      const bool upd = active && !is_piv && tau != 0.0;
+      double w = 0.0;
+      if (upd)
+        for (int i = j + q; i < ell; i += QR_LANES) w = fma(i == j ? 1.0 : v[i - j], col[i], w);
+      w += __shfl_xor_sync(0xffffffffu, w, 1);  // all lanes participate; groups of 4 are aligned
+      w += __shfl_xor_sync(0xffffffffu, w, 2);
+      if (upd) {
+        const double tw = tau * w;
+        for (int i = j + q; i < ell; i += QR_LANES) col[i] = fma(-tw, i == j ? 1.0 : v[i - j], col[i]);
+      }
+      if (is_piv) {
+        for (int i = q; i < k; i += QR_LANES) {
           const double val = (i < j) ? col[i] : (i == j ? beta : 0.0);
           Rho[i + gi * static_cast<long long>(ldr)] = val;
         }
-        __syncwarp();
-        if (lane == 0) active[c] = 0;
-        continue;
+        active = false;
       }
-      if (tau == 0.0) continue;
-      double w = 0.0;
-      for (int i = lane; i < len; i += 32) w = fma(v[i], col[j + i], w);
-#pragma unroll
-      for (int o = 16; o > 0; o >>= 1) w += __shfl_xor_sync(0xffffffffu, w, o);
-      const double tw = tau * w;
-      for (int i = lane; i < len; i += 32) col[j + i] = fma(-tw, v[i], col[j + i]);
     }
-    if (blk == 0 && tid == 0) {  // pivot sequence (perm is assembled afterwards) and the gap
-      inv[j] = gidx;              // `inv` holds the pivot sequence piv[0..k)
+    QT(6)
+    if (blk == 0 && tid == 0) {  // pivot sequence and the relative gap of this step
+      piv[j] = gidx;
       const double nb = sqrt(fmax(s_gbest, 0.0)), ns = sqrt(fmax(s_gsecond, 0.0));
       if (gaps) gaps[j] = nb > 0.0 ? (nb - ns) / nb : 0.0;
     }
     __syncthreads();
   }
+#undef QT
   // rows 0..k-1 of the never-pivoted columns
-  for (int c = warp; c < nc; c += QR_WARPS) {
-    if (!active[c]) continue;
-    const long long gi = c0 + c;
-    for (int i = lane; i < k; i += 32) Rho[i + gi * static_cast<long long>(ldr)] = W[c * ell + i];
-  }
+  if (active)
+    for (int i = q; i < k; i += QR_LANES) Rho[i + (c0 + mc) * static_cast<long long>(ldr)] = col[i];
 }
 
 // perm from the pivot sequence with LAPACK swap semantics: step j exchanges positions j and
@@ -311,6 +299,11 @@ __global__ void qrcp_perm_kernel(const int64_t* __restrict__ piv, int k, long lo
   }
 }
 
+namespace {
+int qr_ldw(int ell) { return (ell + 11) / 16 * 16 + 4; }  // >= ell, = 4 mod 16 doubles
+size_t qr_smem(int cols, int ell) { return (static_cast<size_t>(cols) * qr_ldw(ell) + ell) * 8; }
+}  // namespace
+
 size_t qrcp_workspace_bytes(int ell, long long n) {
   const int NB = 1024;  // upper bound on blocks
   return sizeof(QrWork) + 2 * NB * sizeof(QrCand) + 2 * static_cast<size_t>(NB) * ell * 8 + 2 * n * 8 + 256;
@@ -318,46 +311,59 @@ size_t qrcp_workspace_bytes(int ell, long long n) {
 
 cudaError_t qrcp_truncated(cudaStream_t st, const double* B, int ldb, int ell, long long n, int k, void* work,
                            int64_t* perm, double* Rho, int ldr, double* gaps, int* info, int num_sms) {
-  constexpr size_t kSmemMax = 200 * 1024;
-  int NB = static_cast<int>(std::max<long long>(1, std::min<long long>(num_sms, (n + QR_COLS_TARGET - 1) / QR_COLS_TARGET)));
-  int cols_per = static_cast<int>((n + NB - 1) / NB);
-  auto smem_of = [&](int cp) { return (static_cast<size_t>(cp) * ell + ell) * 8; };
-  while ((smem_of(cols_per) > kSmemMax || cols_per > QR_MAX_COLS) && NB < num_sms) {
-    ++NB;
-    cols_per = static_cast<int>((n + NB - 1) / NB);
-  }
-  if (smem_of(cols_per) > kSmemMax || cols_per > QR_MAX_COLS) return cudaErrorInvalidValue;
-  const size_t smem = smem_of(cols_per);
+  int cols_per = QR_MAX_COLS;
+  while (cols_per > 1 && qr_smem(cols_per, ell) > QR_SMEM_MAX) --cols_per;
+  int NB = static_cast<int>((n + cols_per - 1) / cols_per);
+  if (NB > num_sms || qr_smem(cols_per, ell) > QR_SMEM_MAX) return cudaErrorInvalidValue;
+  cols_per = static_cast<int>((n + NB - 1) / NB);  // balance
+  const size_t smem = qr_smem(cols_per, ell);
+  const int ldw = qr_ldw(ell);
   static bool attr = false;
   if (!attr) {
     cudaError_t e = cudaFuncSetAttribute(qrcp_kernel, cudaFuncAttributeMaxDynamicSharedMemorySize,
-                                         static_cast<int>(kSmemMax));
+                                         static_cast<int>(QR_SMEM_MAX));
+    if (e != cudaSuccess) return e;
+    e = cudaFuncSetAttribute(qrcp_perm_kernel, cudaFuncAttributeMaxDynamicSharedMemorySize,
+                             static_cast<int>(QR_SMEM_MAX));
     if (e != cudaSuccess) return e;
     attr = true;
   }
   cudaError_t e = cudaMemsetAsync(work, 0, sizeof(QrWork), st);
   if (e != cudaSuccess) return e;
   QrWork* w = static_cast<QrWork*>(work);
-  void* args[] = {(void*)&B, (void*)&ldb, (void*)&ell, (void*)&n, (void*)&k, (void*)&w, (void*)&NB, (void*)&cols_per,
-                  (void*)&perm, (void*)&Rho, (void*)&ldr, (void*)&gaps, (void*)&info};
-  count_launch();
-  e = cudaLaunchCooperativeKernel(reinterpret_cast<void*>(qrcp_kernel), dim3(NB), dim3(QR_THREADS), args, smem, st);
-  if (e != cudaSuccess) return e;
-  // assemble perm from the pivot sequence (stored by the kernel where `inv` lives)
   QrCand* cand = reinterpret_cast<QrCand*>(w + 1);
   double* candcol = reinterpret_cast<double*>(cand + 2 * NB);
   int64_t* piv = reinterpret_cast<int64_t*>(candcol + 2 * static_cast<size_t>(NB) * ell);
   int64_t* gpos = piv + n;
+  // RS_QRCP_TIMING=1: per-phase cycle counts of CTA 0 printed to stderr (development aid)
+  static long long* tbuf = nullptr;
+  static const bool timing = getenv("RS_QRCP_TIMING") != nullptr;
+  if (timing && !tbuf && cudaMalloc(&tbuf, 8 * 8 * 1024) != cudaSuccess) tbuf = nullptr;
+  long long* tb = (timing && k <= 1024) ? tbuf : nullptr;
+  void* args[] = {(void*)&B,   (void*)&ldb, (void*)&ell, (void*)&n,    (void*)&k,  (void*)&w,
+                  (void*)&NB,  (void*)&cols_per, (void*)&ldw, (void*)&piv, (void*)&Rho, (void*)&ldr,
+                  (void*)&gaps, (void*)&info, (void*)&tb};
+  count_launch();
+  e = cudaLaunchCooperativeKernel(reinterpret_cast<void*>(qrcp_kernel), dim3(NB), dim3(QR_THREADS), args, smem, st);
+  if (e != cudaSuccess) return e;
   const size_t psmem = static_cast<size_t>(n) * 8;
-  const bool use_smem = psmem <= kSmemMax;
-  static bool pattr = false;
-  if (!pattr) {
-    e = cudaFuncSetAttribute(qrcp_perm_kernel, cudaFuncAttributeMaxDynamicSharedMemorySize, static_cast<int>(kSmemMax));
-    if (e != cudaSuccess) return e;
-    pattr = true;
-  }
+  const bool use_smem = psmem <= QR_SMEM_MAX;
   qrcp_perm_kernel<<<1, 1024, use_smem ? psmem : 0, st>>>(piv, k, n, perm, gpos, use_smem);
   count_launch();
+  if (tb) {
+    static long long h[8 * 1024];
+    cudaStreamSynchronize(st);
+    cudaMemcpy(h, tb, 8 * 8 * static_cast<size_t>(k), cudaMemcpyDeviceToHost);
+    double acc[7] = {0};
+    for (int j = 1; j < k; ++j)
+      for (int p = 0; p < 6; ++p) acc[p] += static_cast<double>(h[j * 8 + p + 1] - h[j * 8 + p]);
+    for (int j = 1; j < k; ++j) acc[6] += static_cast<double>(h[j * 8] - h[(j - 1) * 8 + 6]);
+    fprintf(stderr,
+            "QRCP NB=%d cols=%d cycles/step: A=%.0f barrier=%.0f scan=%.0f vload=%.0f dlarfg=%.0f update=%.0f "
+            "tail=%.0f\n",
+            NB, cols_per, acc[0] / (k - 1), acc[1] / (k - 1), acc[2] / (k - 1), acc[3] / (k - 1), acc[4] / (k - 1),
+            acc[5] / (k - 1), acc[6] / (k - 1));
+  }
   return cudaGetLastError();
 }
 

@@ -74,7 +74,7 @@ Layout plan(long long m_local, long long n, int k, int p) {
   L.off_G = take(sq);
   L.off_Rf = take(sq);
   L.off_Linv = take(sq);
-  L.off_cholw = take(static_cast<size_t>(L.lmax) * (L.lmax + 1) * 8);  // packed S and E of chol_inv
+  L.off_cholw = take(static_cast<size_t>(L.lmax) * (L.lmax + 8) * 8);  // chol_inv work array (n > 128)
   L.off_Rho = take(static_cast<size_t>(L.kp) * n * 8);
   L.off_Rhat = take(static_cast<size_t>(L.kp) * n * 8);
   L.off_T = take(static_cast<size_t>(L.kp) * std::max<long long>(n - k, 1) * 8);
