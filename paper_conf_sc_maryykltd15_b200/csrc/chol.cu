@@ -1,19 +1,18 @@
-// Cholesky factor of a Gram matrix and its inverse in one pass: CholQR steps (ii)-(iii)
+// Cholesky factor of a Gram matrix and its inverse: CholQR steps (ii)-(iii)
 // ("R^T R := G, R upper-triangular with non-negative diagonal; Q = R^{-T} B").
 //
-// Right-looking LDL^T elimination of G with the same row operations applied to an identity E,
-// which becomes L_unit^{-1}:   at pivot k, for every row i > k,
-//     S[i][j] -= S[k][i] S[k][j] / d_k          (j >= i)
-//     E[i][c] -= S[k][i] / d_k * E[k][c]         (c <= k, E[k][k] = 1)
-// Then R[i][j] = S[i][j] / sqrt(d_i) and Linv = R^{-T} = D^{-1/2} E.  S (upper) and E (strict
-// lower; its unit diagonal is implicit) share one n x n array M.
-//
-// One CTA of 1024 threads.  Each thread owns strips of 8 consecutive columns of a row and keeps
-// them in registers (n <= 128); row k is published to shared memory by its owners right after
-// step k-1, so each pivot costs one __syncthreads and every active thread does ~16 FMAs per step
-// on registers with row k read as broadcast LDS.128.  For n > 128 the same schedule runs on an
-// L2-resident copy in the workspace.  A pivot d_k <= 0 or NaN is a CholQR breakdown: reported
-// through *info (LAPACK potrf-style 1-based column) and replaced by 1 so no NaN propagates.
+// n <= 128: blocked (16 x 16) right-looking Cholesky in one CTA, then a blocked forward solve
+// R^T X = I for X = R^{-T} (= Linv), all in shared memory.  Per 16-wide block:
+//   (1) one warp factors the diagonal block in registers (shuffles, rsqrt per pivot),
+//   (2) every thread solves one column of the panel R12 = R11^{-T} A12,
+//   (3) the trailing update A22 -= R12^T R12 is spread over all threads,
+// so a block costs 2 __syncthreads instead of 16 (one per pivot).  The inverse proceeds by block
+// rows of X: a parallel update from the finished block rows, then a 16-step in-block solve per
+// column.  R (upper part of M) and X (strict lower part of M, its diagonal 1/R_ii kept apart)
+// share one padded n x n array.
+// n > 128: right-looking strip elimination on an L2-resident copy (one sync per pivot).
+// A pivot d_k <= 0 or NaN is a CholQR breakdown: reported through *info (LAPACK potrf-style
+// 1-based column) and replaced by 1 so no NaN propagates.
 #include <cstdio>
 
 #include "common.cuh"
@@ -21,128 +20,230 @@
 
 namespace rs {
 
-constexpr int CH_THREADS = 1024;
+constexpr int CB = 16;              // block size
+constexpr int CH_BLK_THREADS = 512;
 constexpr int CH_SMEM_MAX_N = 128;
-constexpr int CH_SW = 8;                                                          // strip width
-constexpr int CH_MAXS = (CH_SMEM_MAX_N * (CH_SMEM_MAX_N / CH_SW) + CH_THREADS - 1) / CH_THREADS;  // 2
 
-template <bool SMALL>
-__global__ void __launch_bounds__(CH_THREADS, 1) chol_inv_kernel(const double* __restrict__ G, int ldg, int n,
-                                                                  double* __restrict__ R, int ldr,
-                                                                  double* __restrict__ Linv, int ldl,
-                                                                  double* __restrict__ gwork, int* info, int code,
-                                                                  int npad) {
-  extern __shared__ double sm[];
-  __shared__ double s_inv[CH_SMEM_MAX_N > 512 ? CH_SMEM_MAX_N : 512];
+// ------------------------------------------------------------------------------------------
+// blocked kernel (n <= 128)
+// ------------------------------------------------------------------------------------------
+__global__ void __launch_bounds__(CH_BLK_THREADS, 1)
+    chol_blocked_kernel(const double* __restrict__ G, int ldg, int n, double* __restrict__ R, int ldr,
+                        double* __restrict__ Linv, int ldl, int* info, int code, int npad) {
+  extern __shared__ double M[];          // np x (np+1), column-major: M[i + j*LM]
+  __shared__ double rdinv[CH_SMEM_MAX_N];  // 1 / R_ii
+  const int np = (n + CB - 1) / CB * CB;
+  const int LM = np + 1;
+  const int tid = threadIdx.x, warp = tid >> 5, lane = tid & 31;
+  const int nb = np / CB;
+
+  // load the upper triangle of G; identity on the padding
+  for (int idx = tid; idx < np * np; idx += CH_BLK_THREADS) {
+    const int i = idx % np, j = idx / np;
+    double v = 0.0;
+    if (i <= j) v = (j < n) ? G[i + static_cast<long long>(j) * ldg] : (i == j ? 1.0 : 0.0);
+    M[i + j * LM] = v;
+  }
+  __syncthreads();
+
+  for (int b = 0; b < nb; ++b) {
+    const int b0 = b * CB;
+    // (1) diagonal block: lane j < 16 owns column b0+j (rows b0..b0+15) in registers
+    if (warp == 0) {
+      double col[CB];
+#pragma unroll
+      for (int i = 0; i < CB; ++i) col[i] = (lane < CB && i <= lane) ? M[(b0 + i) + (b0 + lane) * LM] : 0.0;
+#pragma unroll
+      for (int kk = 0; kk < CB; ++kk) {
+        double d = __shfl_sync(0xffffffffu, col[kk], kk);
+        if (!(d > 0.0)) {
+          if (lane == 0 && info && b0 + kk < n) atomicCAS(info, 0, code), atomicCAS(info + 1, 0, b0 + kk + 1);
+          d = 1.0;
+        }
+        const double ri = rsqrt(d);  // 1 / R_kk
+        if (lane == kk) {
+          col[kk] = d * ri;           // R_kk = sqrt(d)
+          rdinv[b0 + kk] = ri;
+        } else if (lane > kk) {
+          col[kk] *= ri;              // R[kk][lane]
+        }
+        const double rkj = col[kk];
+#pragma unroll
+        for (int i = kk + 1; i < CB; ++i) {
+          const double rki = __shfl_sync(0xffffffffu, col[kk], i);  // R[kk][i] from lane i
+          if (lane >= i && lane < CB) col[i] = fma(-rki, rkj, col[i]);
+        }
+      }
+      if (lane < CB) {
+#pragma unroll
+        for (int i = 0; i < CB; ++i)
+          if (i <= lane) M[(b0 + i) + (b0 + lane) * LM] = col[i];
+      }
+    }
+    __syncthreads();
+    // (2) panel: R12 = R11^{-T} A12, one thread per trailing column
+    const int t2 = np - b0 - CB;
+    if (tid < t2) {
+      const int c = b0 + CB + tid;
+      double x[CB];
+#pragma unroll
+      for (int i = 0; i < CB; ++i) x[i] = M[(b0 + i) + c * LM];
+#pragma unroll
+      for (int kk = 0; kk < CB; ++kk) {
+        x[kk] *= rdinv[b0 + kk];
+#pragma unroll
+        for (int i = kk + 1; i < CB; ++i) x[i] = fma(-M[(b0 + kk) + (b0 + i) * LM], x[kk], x[i]);
+      }
+#pragma unroll
+      for (int i = 0; i < CB; ++i) M[(b0 + i) + c * LM] = x[i];
+    }
+    __syncthreads();
+    // (3) trailing update A22 -= R12^T R12 (upper part); 1 x 2 micro-tiles
+    if (t2 > 0) {
+      const int half = (t2 + 1) / 2;
+      for (int idx = tid; idx < t2 * half; idx += CH_BLK_THREADS) {
+        const int i = b0 + CB + idx % t2;
+        const int j0 = b0 + CB + 2 * (idx / t2);
+        if (i > j0 + 1) continue;
+        const double* pi = M + b0 + i * LM;
+        const double* pj0 = M + b0 + j0 * LM;
+        const double* pj1 = pj0 + LM;
+        double s0 = 0.0, s1 = 0.0;
+#pragma unroll
+        for (int kk = 0; kk < CB; ++kk) {
+          const double a = pi[kk];
+          s0 = fma(a, pj0[kk], s0);
+          if (j0 + 1 < np) s1 = fma(a, pj1[kk], s1);
+        }
+        if (i <= j0) M[i + j0 * LM] -= s0;
+        if (j0 + 1 < np && i <= j0 + 1) M[i + (j0 + 1) * LM] -= s1;
+      }
+    }
+    __syncthreads();
+  }
+
+  // ---- X = R^{-T} (lower), block row by block row; X[l][c] (l > c) stored at M[l + c*LM] ----
+  for (int bi = 0; bi < nb; ++bi) {
+    const int I0 = bi * CB;
+    // (a) X[i][c] = delta_ic - sum_{l=c}^{I0-1} R[l][i] X[l][c],  i in block, c < I0 + 16, c < i
+    //     (the c == i diagonal is handled in (b))
+    for (int idx = tid; idx < CB * I0; idx += CH_BLK_THREADS) {
+      const int i = I0 + idx % CB, c = idx / CB;  // c < I0
+      double s = M[c + i * LM] * rdinv[c];        // l = c term: R[c][i] * X[c][c]
+      for (int l = c + 1; l < I0; ++l) s = fma(M[l + i * LM], M[l + c * LM], s);
+      M[i + c * LM] = -s;
+    }
+    __syncthreads();
+    // (b) in-block forward solve, one thread per column c < I0 + 16
+    if (tid < I0 + CB) {
+      const int c = tid;
+      double x[CB];
+#pragma unroll
+      for (int ii = 0; ii < CB; ++ii) {
+        const int i = I0 + ii;
+        x[ii] = (i > c) ? M[i + c * LM] : 0.0;  // rhs from (a) (zero for c inside the block)
+      }
+#pragma unroll
+      for (int ii = 0; ii < CB; ++ii) {
+        const int i = I0 + ii;
+        if (i < c) continue;
+        double v;
+        if (i == c) {
+          v = rdinv[i];                          // X[c][c] = 1 / R_cc
+        } else {
+          double s = x[ii];
+#pragma unroll
+          for (int jj = 0; jj < ii; ++jj) {
+            const int l = I0 + jj;
+            if (l >= c) s = fma(-M[l + i * LM], x[jj], s);  // R[l][i] * X[l][c]
+          }
+          v = s * rdinv[i];
+        }
+        x[ii] = v;
+      }
+#pragma unroll
+      for (int ii = 0; ii < CB; ++ii) {
+        const int i = I0 + ii;
+        if (i > c) M[i + c * LM] = x[ii];
+      }
+    }
+    __syncthreads();
+  }
+
+  // outputs, zero-padded to npad x npad
+  for (int idx = tid; idx < npad * npad; idx += CH_BLK_THREADS) {
+    const int i = idx % npad, j = idx / npad;
+    double rv = 0.0, lv = 0.0;
+    if (i < n && j < n) {
+      if (i <= j) rv = M[i + j * LM];
+      if (i == j) lv = rdinv[i];
+      else if (i > j) lv = M[i + j * LM];
+    }
+    R[i + static_cast<long long>(j) * ldr] = rv;
+    Linv[i + static_cast<long long>(j) * ldl] = lv;
+  }
+}
+
+// ------------------------------------------------------------------------------------------
+// strip kernel for n > 128 (L2-resident working copy; one sync per pivot)
+//   S[i][j] -= S[k][i] S[k][j] / d_k (j >= i > k);  E[i][c] -= S[k][i] / d_k * E[k][c] (c <= k)
+//   R = D^{-1/2} S,  Linv = D^{-1/2} E  (E unit lower, S and E share one array)
+// ------------------------------------------------------------------------------------------
+constexpr int CH_THREADS = 1024;
+constexpr int CH_SW = 8;
+
+__global__ void __launch_bounds__(CH_THREADS, 1) chol_strip_kernel(const double* __restrict__ G, int ldg, int n,
+                                                                    double* __restrict__ R, int ldr,
+                                                                    double* __restrict__ Linv, int ldl,
+                                                                    double* __restrict__ M, int* info, int code,
+                                                                    int npad) {
+  __shared__ double s_inv[512];
   const int tid = threadIdx.x;
-  const int ns = (n + CH_SW - 1) / CH_SW;  // strips per row
-  const int ldm = ns * CH_SW;              // row pitch of M (multiple of 8 -> 64-byte aligned strips)
-  double* M = SMALL ? sm : gwork;
+  const int ns = (n + CH_SW - 1) / CH_SW;
+  const int ldm = ns * CH_SW;
   const int nstrips = n * ns;
-
-  auto pivot_inv = [&](int k, double d) {  // by the owner of M[k][k]
+  auto pivot_inv = [&](int k, double d) {
     if (!(d > 0.0)) {
       if (info) atomicCAS(info, 0, code), atomicCAS(info + 1, 0, k + 1);
       d = 1.0;
     }
     s_inv[k] = 1.0 / d;
   };
-
-  if (SMALL) {
-    double reg[CH_MAXS][CH_SW];
-    int ri[CH_MAXS], rj[CH_MAXS];
-#pragma unroll
-    for (int u = 0; u < CH_MAXS; ++u) {
-      const int id = tid + u * CH_THREADS;
-      ri[u] = id < nstrips ? id / ns : n;  // n = no strip
-      rj[u] = id < nstrips ? (id % ns) * CH_SW : 0;
-#pragma unroll
-      for (int e = 0; e < CH_SW; ++e) {
-        const int j = rj[u] + e;
-        reg[u][e] = (ri[u] < n && j < n) ? (j >= ri[u] ? G[ri[u] + static_cast<long long>(j) * ldg] : 0.0) : 0.0;
-      }
-      if (ri[u] == 0) {  // publish row 0
-#pragma unroll
-        for (int e = 0; e < CH_SW; ++e) M[rj[u] + e] = reg[u][e];
-        if (rj[u] == 0) pivot_inv(0, reg[u][0]);
-      }
-    }
-    __syncthreads();
-    for (int k = 0; k < n - 1; ++k) {
-      const double* Mk = M + static_cast<long long>(k) * ldm;
-      const double inv = s_inv[k];
-#pragma unroll
-      for (int u = 0; u < CH_MAXS; ++u) {
-        const int i = ri[u];
-        if (i <= k || i >= n) continue;
-        const double l = Mk[i] * inv;  // S[k][i] / d_k
-        const double2* rk = reinterpret_cast<const double2*>(Mk + rj[u]);
-#pragma unroll
-        for (int e2 = 0; e2 < CH_SW / 2; ++e2) {
-          const double2 m2 = rk[e2];
-#pragma unroll
-          for (int h = 0; h < 2; ++h) {
-            const int e = 2 * e2 + h;
-            const int j = rj[u] + e;
-            const double mkj = h ? m2.y : m2.x;
-            if (j >= i)
-              reg[u][e] = fma(-l, mkj, reg[u][e]);                     // S part
-            else if (j <= k)
-              reg[u][e] = fma(-l, j == k ? 1.0 : mkj, reg[u][e]);      // E part (E[k][k] = 1)
-          }
-        }
-        if (i == k + 1) {  // row k+1 is final: publish it and its pivot
-          double* dst = M + static_cast<long long>(i) * ldm + rj[u];
-#pragma unroll
-          for (int e = 0; e < CH_SW; ++e) dst[e] = reg[u][e];
-          if (rj[u] <= i && i < rj[u] + CH_SW) {
-#pragma unroll
-            for (int e = 0; e < CH_SW; ++e)
-              if (rj[u] + e == i) pivot_inv(i, reg[u][e]);
-          }
-        }
-      }
-      __syncthreads();
-    }
-  } else {
-    // large n: M lives in the L2-resident workspace, updated in place
-    for (int id = tid; id < nstrips; id += CH_THREADS) {
-      const int i = id / ns, j0 = (id % ns) * CH_SW;
-      for (int e = 0; e < CH_SW; ++e) {
-        const int j = j0 + e;
-        M[static_cast<long long>(i) * ldm + j] = (j < n && j >= i) ? G[i + static_cast<long long>(j) * ldg] : 0.0;
-      }
-    }
-    __syncthreads();
-    if (tid == 0) pivot_inv(0, M[0]);
-    __syncthreads();
-    for (int k = 0; k < n - 1; ++k) {
-      const double* Mk = M + static_cast<long long>(k) * ldm;
-      const double inv = s_inv[k];
-      for (int id = tid; id < nstrips; id += CH_THREADS) {
-        const int i = id / ns, j0 = (id % ns) * CH_SW;
-        if (i <= k) continue;
-        const double l = Mk[i] * inv;
-        double* row = M + static_cast<long long>(i) * ldm + j0;
-        for (int e = 0; e < CH_SW; ++e) {
-          const int j = j0 + e;
-          if (j >= n) break;
-          if (j >= i)
-            row[e] = fma(-l, Mk[j], row[e]);
-          else if (j <= k)
-            row[e] = fma(-l, j == k ? 1.0 : Mk[j], row[e]);
-        }
-        if (i == k + 1 && j0 <= i && i < j0 + CH_SW) pivot_inv(i, row[i - j0]);
-      }
-      __syncthreads();
+  for (int id = tid; id < nstrips; id += CH_THREADS) {
+    const int i = id / ns, j0 = (id % ns) * CH_SW;
+    for (int e = 0; e < CH_SW; ++e) {
+      const int j = j0 + e;
+      M[static_cast<long long>(i) * ldm + j] = (j < n && j >= i) ? G[i + static_cast<long long>(j) * ldg] : 0.0;
     }
   }
-  // R (upper, zero below) and Linv = D^{-1/2} E (lower, unit diagonal scaled), zero-padded
+  __syncthreads();
+  if (tid == 0) pivot_inv(0, M[0]);
+  __syncthreads();
+  for (int k = 0; k < n - 1; ++k) {
+    const double* Mk = M + static_cast<long long>(k) * ldm;
+    const double inv = s_inv[k];
+    for (int id = tid; id < nstrips; id += CH_THREADS) {
+      const int i = id / ns, j0 = (id % ns) * CH_SW;
+      if (i <= k) continue;
+      const double l = Mk[i] * inv;
+      double* row = M + static_cast<long long>(i) * ldm + j0;
+      for (int e = 0; e < CH_SW; ++e) {
+        const int j = j0 + e;
+        if (j >= n) break;
+        if (j >= i)
+          row[e] = fma(-l, Mk[j], row[e]);
+        else if (j <= k)
+          row[e] = fma(-l, j == k ? 1.0 : Mk[j], row[e]);
+      }
+      if (i == k + 1 && j0 <= i && i < j0 + CH_SW) pivot_inv(i, row[i - j0]);
+    }
+    __syncthreads();
+  }
   for (int idx = tid; idx < npad * npad; idx += CH_THREADS) {
     const int i = idx % npad, j = idx / npad;
     double rv = 0.0, lv = 0.0;
     if (i < n && j < n) {
-      const double rs = sqrt(s_inv[i]);  // 1/sqrt(d_i)
+      const double rs = sqrt(s_inv[i]);
       const double mij = M[static_cast<long long>(i) * ldm + j];
       if (i <= j) rv = mij * rs;
       if (j < i) lv = mij * rs;
@@ -157,19 +258,19 @@ cudaError_t chol_inv(cudaStream_t st, const double* G, int ldg, int n, int npad,
                      int ldl, double* gwork, int* info, int info_code) {
   if (n <= 0) return cudaSuccess;
   if (n > 512) return cudaErrorInvalidValue;
-  const int ldm = (n + CH_SW - 1) / CH_SW * CH_SW;
-  const size_t work = static_cast<size_t>(n) * ldm * 8;
   if (n <= CH_SMEM_MAX_N) {
+    const int np = (n + CB - 1) / CB * CB;
+    const size_t smem = static_cast<size_t>(np) * (np + 1) * 8;
     static bool attr = false;
     if (!attr) {
-      cudaError_t e = cudaFuncSetAttribute(chol_inv_kernel<true>, cudaFuncAttributeMaxDynamicSharedMemorySize,
-                                           CH_SMEM_MAX_N * CH_SMEM_MAX_N * 8);
+      cudaError_t e = cudaFuncSetAttribute(chol_blocked_kernel, cudaFuncAttributeMaxDynamicSharedMemorySize,
+                                           CH_SMEM_MAX_N * (CH_SMEM_MAX_N + 1) * 8);
       if (e != cudaSuccess) return e;
       attr = true;
     }
-    chol_inv_kernel<true><<<1, CH_THREADS, work, st>>>(G, ldg, n, R, ldr, Linv, ldl, gwork, info, info_code, npad);
+    chol_blocked_kernel<<<1, CH_BLK_THREADS, smem, st>>>(G, ldg, n, R, ldr, Linv, ldl, info, info_code, npad);
   } else {
-    chol_inv_kernel<false><<<1, CH_THREADS, 0, st>>>(G, ldg, n, R, ldr, Linv, ldl, gwork, info, info_code, npad);
+    chol_strip_kernel<<<1, CH_THREADS, 0, st>>>(G, ldg, n, R, ldr, Linv, ldl, gwork, info, info_code, npad);
   }
   count_launch();
   return cudaGetLastError();
