@@ -74,8 +74,11 @@ struct MCSmem {
   static constexpr int TOTAL = 1024 + NSTAGE * (R_BYTES + L_BYTES) + 2 * NSTAGE * 8;
 };
 
+// Align the dynamic shared-memory base to 1024 bytes (128B-swizzle atoms) by pointer arithmetic
+// on the __shared__ array itself, so the compiler keeps the shared address space and emits
+// LDS.128 (a uintptr round trip would turn every fragment load into a generic LD).
 RS_DEVINL unsigned char* align1024(unsigned char* p) {
-  return reinterpret_cast<unsigned char*>((reinterpret_cast<uintptr_t>(p) + 1023) & ~uintptr_t(1023));
+  return p + ((1024u - (smem_u32(p) & 1023u)) & 1023u);
 }
 
 // KC: tile row of fragment row r in fragment f of 16-row group g
