@@ -10,7 +10,7 @@
 // rows of X: a parallel update from the finished block rows, then a 16-step in-block solve per
 // column.  R (upper part of M) and X (strict lower part of M, its diagonal 1/R_ii kept apart)
 // share one padded n x n array.
-// n > 128: right-looking strip elimination on an L2-resident copy (one sync per pivot).
+// n > 128: the same blocked schedule on an L2-resident copy in the workspace.
 // A pivot d_k <= 0 or NaN is a CholQR breakdown: reported through *info (LAPACK potrf-style
 // 1-based column) and replaced by 1 so no NaN propagates.
 #include <cstdio>
@@ -27,11 +27,14 @@ constexpr int CH_SMEM_MAX_N = 128;
 // ------------------------------------------------------------------------------------------
 // blocked kernel (n <= 128)
 // ------------------------------------------------------------------------------------------
+template <bool SMEM>
 __global__ void __launch_bounds__(CH_BLK_THREADS, 1)
     chol_blocked_kernel(const double* __restrict__ G, int ldg, int n, double* __restrict__ R, int ldr,
-                        double* __restrict__ Linv, int ldl, int* info, int code, int npad) {
-  extern __shared__ double M[];          // np x (np+1), column-major: M[i + j*LM]
-  __shared__ double rdinv[CH_SMEM_MAX_N];  // 1 / R_ii
+                        double* __restrict__ Linv, int ldl, double* __restrict__ gwork, int* info, int code,
+                        int npad) {
+  extern __shared__ double sm[];
+  double* M = SMEM ? sm : gwork;  // np x (np+1), column-major: M[i + j*LM]
+  __shared__ double rdinv[512];   // 1 / R_ii
   const int np = (n + CB - 1) / CB * CB;
   const int LM = np + 1;
   const int tid = threadIdx.x, warp = tid >> 5, lane = tid & 31;
@@ -184,76 +187,6 @@ __global__ void __launch_bounds__(CH_BLK_THREADS, 1)
   }
 }
 
-// ------------------------------------------------------------------------------------------
-// strip kernel for n > 128 (L2-resident working copy; one sync per pivot)
-//   S[i][j] -= S[k][i] S[k][j] / d_k (j >= i > k);  E[i][c] -= S[k][i] / d_k * E[k][c] (c <= k)
-//   R = D^{-1/2} S,  Linv = D^{-1/2} E  (E unit lower, S and E share one array)
-// ------------------------------------------------------------------------------------------
-constexpr int CH_THREADS = 1024;
-constexpr int CH_SW = 8;
-
-__global__ void __launch_bounds__(CH_THREADS, 1) chol_strip_kernel(const double* __restrict__ G, int ldg, int n,
-                                                                    double* __restrict__ R, int ldr,
-                                                                    double* __restrict__ Linv, int ldl,
-                                                                    double* __restrict__ M, int* info, int code,
-                                                                    int npad) {
-  __shared__ double s_inv[512];
-  const int tid = threadIdx.x;
-  const int ns = (n + CH_SW - 1) / CH_SW;
-  const int ldm = ns * CH_SW;
-  const int nstrips = n * ns;
-  auto pivot_inv = [&](int k, double d) {
-    if (!(d > 0.0)) {
-      if (info) atomicCAS(info, 0, code), atomicCAS(info + 1, 0, k + 1);
-      d = 1.0;
-    }
-    s_inv[k] = 1.0 / d;
-  };
-  for (int id = tid; id < nstrips; id += CH_THREADS) {
-    const int i = id / ns, j0 = (id % ns) * CH_SW;
-    for (int e = 0; e < CH_SW; ++e) {
-      const int j = j0 + e;
-      M[static_cast<long long>(i) * ldm + j] = (j < n && j >= i) ? G[i + static_cast<long long>(j) * ldg] : 0.0;
-    }
-  }
-  __syncthreads();
-  if (tid == 0) pivot_inv(0, M[0]);
-  __syncthreads();
-  for (int k = 0; k < n - 1; ++k) {
-    const double* Mk = M + static_cast<long long>(k) * ldm;
-    const double inv = s_inv[k];
-    for (int id = tid; id < nstrips; id += CH_THREADS) {
-      const int i = id / ns, j0 = (id % ns) * CH_SW;
-      if (i <= k) continue;
-      const double l = Mk[i] * inv;
-      double* row = M + static_cast<long long>(i) * ldm + j0;
-      for (int e = 0; e < CH_SW; ++e) {
-        const int j = j0 + e;
-        if (j >= n) break;
-        if (j >= i)
-          row[e] = fma(-l, Mk[j], row[e]);
-        else if (j <= k)
-          row[e] = fma(-l, j == k ? 1.0 : Mk[j], row[e]);
-      }
-      if (i == k + 1 && j0 <= i && i < j0 + CH_SW) pivot_inv(i, row[i - j0]);
-    }
-    __syncthreads();
-  }
-  for (int idx = tid; idx < npad * npad; idx += CH_THREADS) {
-    const int i = idx % npad, j = idx / npad;
-    double rv = 0.0, lv = 0.0;
-    if (i < n && j < n) {
-      const double rs = sqrt(s_inv[i]);
-      const double mij = M[static_cast<long long>(i) * ldm + j];
-      if (i <= j) rv = mij * rs;
-      if (j < i) lv = mij * rs;
-      if (j == i) lv = rs;
-    }
-    R[i + static_cast<long long>(j) * ldr] = rv;
-    Linv[i + static_cast<long long>(j) * ldl] = lv;
-  }
-}
-
 cudaError_t chol_inv(cudaStream_t st, const double* G, int ldg, int n, int npad, double* R, int ldr, double* Linv,
                      int ldl, double* gwork, int* info, int info_code) {
   if (n <= 0) return cudaSuccess;
@@ -263,14 +196,16 @@ cudaError_t chol_inv(cudaStream_t st, const double* G, int ldg, int n, int npad,
     const size_t smem = static_cast<size_t>(np) * (np + 1) * 8;
     static bool attr = false;
     if (!attr) {
-      cudaError_t e = cudaFuncSetAttribute(chol_blocked_kernel, cudaFuncAttributeMaxDynamicSharedMemorySize,
+      cudaError_t e = cudaFuncSetAttribute(chol_blocked_kernel<true>, cudaFuncAttributeMaxDynamicSharedMemorySize,
                                            CH_SMEM_MAX_N * (CH_SMEM_MAX_N + 1) * 8);
       if (e != cudaSuccess) return e;
       attr = true;
     }
-    chol_blocked_kernel<<<1, CH_BLK_THREADS, smem, st>>>(G, ldg, n, R, ldr, Linv, ldl, info, info_code, npad);
-  } else {
-    chol_strip_kernel<<<1, CH_THREADS, 0, st>>>(G, ldg, n, R, ldr, Linv, ldl, gwork, info, info_code, npad);
+    chol_blocked_kernel<true><<<1, CH_BLK_THREADS, smem, st>>>(G, ldg, n, R, ldr, Linv, ldl, gwork, info, info_code,
+                                                                npad);
+  } else {  // same schedule on an L2-resident copy in the workspace (np x (np+1) doubles)
+    chol_blocked_kernel<false><<<1, CH_BLK_THREADS, 0, st>>>(G, ldg, n, R, ldr, Linv, ldl, gwork, info, info_code,
+                                                             npad);
   }
   count_launch();
   return cudaGetLastError();

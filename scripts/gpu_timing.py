@@ -19,10 +19,16 @@ def main():
     ap.add_argument("--cfg", default="cfg2")
     ap.add_argument("--reps", type=int, default=3)
     ap.add_argument("--m", type=int, default=0)
+    ap.add_argument("--k", type=int, default=0)
+    ap.add_argument("--q", type=int, default=-1)
     args = ap.parse_args()
     c = dict(CONFIGS[args.cfg])
     if args.m:
         c["m"] = args.m
+    if args.k:
+        c["k"] = args.k
+    if args.q >= 0:
+        c["q"] = args.q
     m, n, k, p, q = c["m"], c["n"], c["k"], c["p"], c["q"]
     t0 = time.time()
     A, _ = make_matrix_torch(m, n, c["law"], k, seed=2015, device="cuda")

@@ -129,3 +129,10 @@ OMEGA_SEED = 0x5C15
 
 def matrix_spec(name: str) -> dict:
     return dict(CONFIGS[name])
+
+
+def config_variant(name: str, **over) -> dict:
+    """A BASELINE config with overrides (e.g. the cfg5 k / q sweep)."""
+    c = dict(CONFIGS[name])
+    c.update(over)
+    return c

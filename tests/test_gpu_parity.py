@@ -158,6 +158,8 @@ def test_pipeline_cfg1(q):
     (20000, 1000, 50, 10, 1, "exp-k"),    # several N tiles, split-K
     (2000, 400, 120, 8, 1, "exp-k"),      # l = 128: full M tile
     (4000, 500, 150, 10, 0, "exp-k"),     # l = 160 > 128: two M tiles, k > 128
+    (6000, 900, 400, 10, 1, "exp-k"),     # cfg5's largest k: l = 410, four M tiles, Cholesky n > 128
+    (8000, 1000, 200, 20, 2, "power"),    # cfg3 law and (k, p, q) at reduced m, n
 ])
 def test_pipeline_ragged_and_multitile(m, n, k, p, q, law):
     A, _ = make_matrix(m, n, law, k, seed=m + 3 * n)
