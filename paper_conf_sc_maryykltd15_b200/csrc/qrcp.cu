@@ -299,6 +299,188 @@ __global__ void qrcp_perm_kernel(const int64_t* __restrict__ piv, int k, long lo
   }
 }
 
+// ------------------------------------------------------------------------------------------
+// Register-resident variant for l <= 128 (the paper-shaped configs): each column of B lives in
+// the registers of 4 lanes (rows q + 4t, t < 32) for all k steps, so residual norms, reflector
+// dot products and updates never touch shared memory; the next step's residual norm is fused
+// into the update.  Every warp scans the candidates itself (no CTA broadcast), loads its rows
+// of the winning column straight from L2 and forms the dlarfg reflector redundantly.
+// ------------------------------------------------------------------------------------------
+constexpr int QRR_THREADS = 512;
+constexpr int QRR_COLS = QRR_THREADS / 4;  // 128 columns per CTA
+constexpr int QRR_ROWS = 32;               // rows per lane: l <= 128
+
+__global__ void __launch_bounds__(QRR_THREADS, 1)
+    qrcp_reg_kernel(const double* __restrict__ B, int ldb, int ell, long long n, int k, QrWork* work, int NB,
+                    int64_t* __restrict__ piv, double* __restrict__ Rho, int ldr, double* __restrict__ gaps,
+                    int* info) {
+  const int blk = blockIdx.x;
+  const int tid = threadIdx.x, warp = tid >> 5, lane = tid & 31;
+  const int mc = tid >> 2, q = tid & 3;
+  const long long c0 = static_cast<long long>(blk) * QRR_COLS;
+  const long long gi = c0 + mc;  // my column (original index)
+  bool active = gi < n;
+  __shared__ Arg s_warg[QRR_THREADS / 32];
+  __shared__ double s_wsec[QRR_THREADS / 32];
+  __shared__ double s_v[QRR_THREADS / 32][4 * QRR_ROWS];
+  QrCand* cand = reinterpret_cast<QrCand*>(work + 1);
+  double* candcol = reinterpret_cast<double*>(cand + 2 * NB);
+
+  double x[QRR_ROWS];
+#pragma unroll
+  for (int t = 0; t < QRR_ROWS; ++t) {
+    const int i = q + 4 * t;
+    x[t] = (active && i < ell) ? B[i + gi * static_cast<long long>(ldb)] : 0.0;
+  }
+  // residual norm^2 over rows >= 0
+  double s = 0.0;
+#pragma unroll
+  for (int t = 0; t < QRR_ROWS; ++t) s = fma(x[t], x[t], s);
+
+  for (int j = 0; j < k; ++j) {
+    const int par = j & 1;
+    // ---- (A) CTA best / runner-up of the residual norms (s holds rows >= j) ----
+    double sc = s;
+    sc += __shfl_xor_sync(0xffffffffu, sc, 1);
+    sc += __shfl_xor_sync(0xffffffffu, sc, 2);
+    {
+      Arg a = (active && q == 0) ? Arg{sc, gi, mc} : Arg{-1.0, -1, -1};
+      double sec = -1.0;
+      warp_top2(a, sec);
+      if (lane == 0) {
+        s_warg[warp] = a;
+        s_wsec[warp] = sec;
+      }
+      __syncthreads();
+      if (warp == 0) {
+        Arg xx = lane < QRR_THREADS / 32 ? s_warg[lane] : Arg{-1.0, -1, -1};
+        double xs = lane < QRR_THREADS / 32 ? s_wsec[lane] : -1.0;
+        warp_top2(xx, xs);
+        if (lane == 0) {
+          QrCand cd;
+          cd.best = xx.v;
+          cd.second = xs;
+          cd.idx = xx.i;
+          cd.pad = 0;
+          cand[par * NB + blk] = cd;
+          s_warg[0] = xx;  // this CTA's winner (read by its owner lanes below)
+        }
+      }
+      __syncthreads();
+    }
+    // the owner of this CTA's best column publishes rows j..ell-1
+    if (active && s_warg[0].i == gi) {
+      double* dst = candcol + (static_cast<size_t>(par) * NB + blk) * ell;
+#pragma unroll
+      for (int t = 0; t < QRR_ROWS; ++t) {
+        const int i = q + 4 * t;
+        if (i >= j && i < ell) dst[i] = x[t];
+      }
+    }
+    grid_sync_count(&work->count, static_cast<unsigned int>(j + 1) * NB);
+
+    // ---- (B) every warp scans the NB candidates (no CTA broadcast needed) ----
+    Arg g{-1.0, -1, -1};
+    double g2 = -1.0;
+    for (int b = lane; b < NB; b += 32) {
+      const long long ci = __ldcg(&cand[par * NB + b].idx);
+      const double cb = __ldcg(&cand[par * NB + b].best);
+      const double cs = __ldcg(&cand[par * NB + b].second);
+      g2 = fmax(g2, cs);
+      if (better(cb, ci, g.v, g.i)) {
+        if (g.i >= 0) g2 = fmax(g2, g.v);
+        g = Arg{cb, ci, b};
+      } else if (ci >= 0) {
+        g2 = fmax(g2, cb);
+      }
+    }
+    warp_top2(g, g2);
+    const long long gidx = g.i;
+    const int gblk = g.b < 0 ? 0 : g.b;
+    // this warp's copy of the pivot column (rows >= j) in shared memory; alpha and
+    // xs = ||x_p[j+1:]||^2 by a warp reduction, reflector formed redundantly per warp
+    const double* src = candcol + (static_cast<size_t>(par) * NB + gblk) * ell;
+    double* vw = s_v[warp];
+    double pv[QRR_ROWS / 8];
+    double xs = 0.0, alpha = 0.0;
+#pragma unroll
+    for (int u = 0; u < QRR_ROWS / 8; ++u) {
+      const int i = lane + 32 * u;
+      pv[u] = (i >= j && i < ell) ? __ldcg(src + i) : 0.0;
+      if (i > j) xs = fma(pv[u], pv[u], xs);
+      if (i == j) alpha = pv[u];
+    }
+#pragma unroll
+    for (int o = 16; o > 0; o >>= 1) {
+      xs += __shfl_xor_sync(0xffffffffu, xs, o);
+      alpha += __shfl_xor_sync(0xffffffffu, alpha, o);  // only lane j%32 holds a nonzero term
+    }
+    double tau = 0.0, beta = alpha;
+    if (g.i >= 0 && xs > 0.0) {
+      const double h = sqrt(fma(alpha, alpha, xs));
+      beta = alpha >= 0.0 ? -h : h;
+      tau = (beta - alpha) / beta;
+    }
+    const double den = alpha - beta;
+#pragma unroll
+    for (int u = 0; u < QRR_ROWS / 8; ++u) {
+      const int i = lane + 32 * u;
+      vw[i] = (i < j) ? 0.0 : (i == j ? 1.0 : (tau != 0.0 ? pv[u] / den : 0.0));
+    }
+    __syncwarp();
+    if (blk == 0 && tid == 0) {
+      if (g.i < 0 || !(g.v > 0.0)) {
+        if (info) atomicCAS(info, 0, 6 /* RS_ERR_RANK_DEFICIENT */), atomicCAS(info + 1, 0, j + 1);
+      }
+      piv[j] = gidx;
+      const double nb = sqrt(fmax(g.v, 0.0)), ns = sqrt(fmax(g2, 0.0));
+      if (gaps) gaps[j] = nb > 0.0 ? (nb - ns) / nb : 0.0;
+    }
+    // ---- apply H = I - tau v v^T; retire the pivot column; fuse the next residual norm ----
+    const bool is_piv = active && gi == gidx;
+    const bool upd = active && !is_piv && tau != 0.0;
+    double w = 0.0;
+    if (upd) {
+#pragma unroll
+      for (int t = 0; t < QRR_ROWS; ++t) w = fma(vw[q + 4 * t], x[t], w);  // v = 0 outside rows >= j
+    }
+    w += __shfl_xor_sync(0xffffffffu, w, 1);
+    w += __shfl_xor_sync(0xffffffffu, w, 2);
+    s = 0.0;
+    if (upd) {
+      const double tw = tau * w;
+#pragma unroll
+      for (int t = 0; t < QRR_ROWS; ++t) {
+        x[t] = fma(-tw, vw[q + 4 * t], x[t]);
+        const int i = q + 4 * t;
+        if (i > j) s = fma(x[t], x[t], s);
+      }
+    } else if (active && !is_piv) {
+#pragma unroll
+      for (int t = 0; t < QRR_ROWS; ++t) {
+        const int i = q + 4 * t;
+        if (i > j) s = fma(x[t], x[t], s);
+      }
+    }
+    if (is_piv) {
+#pragma unroll
+      for (int t = 0; t < QRR_ROWS; ++t) {
+        const int i = q + 4 * t;
+        if (i < k) Rho[i + gi * static_cast<long long>(ldr)] = (i < j) ? x[t] : (i == j ? beta : 0.0);
+      }
+      active = false;
+    }
+    __syncthreads();  // s_warg reuse and candidate buffers of parity `par`
+  }
+  if (active) {
+#pragma unroll
+    for (int t = 0; t < QRR_ROWS; ++t) {
+      const int i = q + 4 * t;
+      if (i < k) Rho[i + gi * static_cast<long long>(ldr)] = x[t];
+    }
+  }
+}
+
 namespace {
 int qr_ldw(int ell) { return (ell + 11) / 16 * 16 + 4; }  // >= ell, = 4 mod 16 doubles
 size_t qr_smem(int cols, int ell) { return (static_cast<size_t>(cols) * qr_ldw(ell) + ell) * 8; }
@@ -311,12 +493,14 @@ size_t qrcp_workspace_bytes(int ell, long long n) {
 
 cudaError_t qrcp_truncated(cudaStream_t st, const double* B, int ldb, int ell, long long n, int k, void* work,
                            int64_t* perm, double* Rho, int ldr, double* gaps, int* info, int num_sms) {
-  int cols_per = QR_MAX_COLS;
-  while (cols_per > 1 && qr_smem(cols_per, ell) > QR_SMEM_MAX) --cols_per;
+  static const bool force_smem = getenv("RS_QRCP_SMEM") != nullptr;  // development switch
+  const bool use_reg = !force_smem && ell <= 4 * QRR_ROWS && (n + QRR_COLS - 1) / QRR_COLS <= num_sms;
+  int cols_per = use_reg ? QRR_COLS : QR_MAX_COLS;
+  while (!use_reg && cols_per > 1 && qr_smem(cols_per, ell) > QR_SMEM_MAX) --cols_per;
   int NB = static_cast<int>((n + cols_per - 1) / cols_per);
-  if (NB > num_sms || qr_smem(cols_per, ell) > QR_SMEM_MAX) return cudaErrorInvalidValue;
-  cols_per = static_cast<int>((n + NB - 1) / NB);  // balance
-  const size_t smem = qr_smem(cols_per, ell);
+  if (NB > num_sms || (!use_reg && qr_smem(cols_per, ell) > QR_SMEM_MAX)) return cudaErrorInvalidValue;
+  if (!use_reg) cols_per = static_cast<int>((n + NB - 1) / NB);  // balance
+  const size_t smem = use_reg ? 0 : qr_smem(cols_per, ell);
   const int ldw = qr_ldw(ell);
   static bool attr = false;
   if (!attr) {
@@ -344,7 +528,15 @@ cudaError_t qrcp_truncated(cudaStream_t st, const double* B, int ldb, int ell, l
                   (void*)&NB,  (void*)&cols_per, (void*)&ldw, (void*)&piv, (void*)&Rho, (void*)&ldr,
                   (void*)&gaps, (void*)&info, (void*)&tb};
   count_launch();
-  e = cudaLaunchCooperativeKernel(reinterpret_cast<void*>(qrcp_kernel), dim3(NB), dim3(QR_THREADS), args, smem, st);
+  if (use_reg) {
+    void* rargs[] = {(void*)&B, (void*)&ldb, (void*)&ell, (void*)&n,  (void*)&k,    (void*)&w,
+                     (void*)&NB, (void*)&piv, (void*)&Rho, (void*)&ldr, (void*)&gaps, (void*)&info};
+    e = cudaLaunchCooperativeKernel(reinterpret_cast<void*>(qrcp_reg_kernel), dim3(NB), dim3(QRR_THREADS), rargs, 0,
+                                    st);
+    tb = nullptr;
+  } else {
+    e = cudaLaunchCooperativeKernel(reinterpret_cast<void*>(qrcp_kernel), dim3(NB), dim3(QR_THREADS), args, smem, st);
+  }
   if (e != cudaSuccess) return e;
   const size_t psmem = static_cast<size_t>(n) * 8;
   const bool use_smem = psmem <= QR_SMEM_MAX;
