@@ -1,0 +1,80 @@
+"""Pins for oracle/adaptive.py (Fig. 3, the fixed-accuracy adaptive scheme)."""
+
+import math
+
+import numpy as np
+import pytest
+
+from oracle import adaptive as AD
+from oracle import pipeline as PL
+from oracle.linalg import rows_orth
+from synth.matrices import make_matrix
+
+
+def _proj(B):
+    return B.T @ B
+
+
+def test_bcgs2_makes_rows_orthogonal():
+    rng = np.random.default_rng(0)
+    X, _ = rows_orth(rng.standard_normal((5, 40)))
+    Y = rng.standard_normal((3, 40)) + 1e3 * X[:3]          # nearly in span(X): needs the second pass
+    Z = AD.bcgs2(X, Y)
+    assert np.abs(Z @ X.T).max() <= 1e-12 * np.abs(Y).max()
+    np.testing.assert_array_equal(AD.bcgs2(np.zeros((0, 40)), Y), Y)
+
+
+def test_single_round_q0_equals_fixed_rank_orthonormal_sample():
+    """One round with l_inc = l: B = QR(Omega[0:l] A), the fixed-rank sample (R16)."""
+    A, _ = make_matrix(300, 80, "exp-paper", 10, seed=1)
+    res = AD.adaptive_sample(A, eps=0.0, ell_inc=12, q=0, seed=7, ell_max=12)
+    Bf, _ = rows_orth(PL.sample(A, 12, 7))
+    np.testing.assert_allclose(res.B, Bf, atol=1e-13)
+    assert res.ell == 12 and not res.converged
+
+
+@pytest.mark.parametrize("q", [0, 1])
+def test_blocks_are_orthonormal_and_q0_span_matches(q):
+    A, _ = make_matrix(400, 120, "exp-paper", 10, seed=2)
+    res = AD.adaptive_sample(A, eps=0.0, ell_inc=8, q=q, seed=3, ell_max=40)
+    assert res.ell == 40
+    np.testing.assert_allclose(res.B @ res.B.T, np.eye(40), atol=1e-13)
+    if q == 0:  # block Gram-Schmidt does not change the span of Omega[0:l] A
+        Bf, _ = rows_orth(PL.sample(A, 40, 3))
+        np.testing.assert_allclose(_proj(res.B), _proj(Bf), atol=1e-11)
+
+
+def test_estimator_bounds_the_range_error():
+    """Bound (4) (HMT eq. (4.3), c_ad = 10): ||A - A B^T B||_2 <= 10 sqrt(2/pi) eps~,
+    with failure probability <= min(m, n) 10^-l_inc; and eps~ never falls below the true error of
+    the projected Gaussian test vectors' expectation by more than chance (eps~ > 0)."""
+    A, s = make_matrix(600, 200, "exp-paper", 20, seed=4)
+    res = AD.adaptive_sample(A, eps=1e-6, ell_inc=8, q=0, seed=5, ell_max=160)
+    assert res.converged
+    est = res.history[-1][1]
+    err = np.linalg.norm(A - (A @ res.B.T) @ res.B, 2)
+    assert err <= 10 * math.sqrt(2 / math.pi) * est
+    assert est <= 1e-6
+    # the rank found is close to where sigma drops below eps (10^(-i/10) = 1e-6 at i = 60)
+    assert 56 <= res.ell <= 96
+
+
+def test_error_estimates_decrease_with_power_iteration():
+    """The paper's Fig. 16: with q > 0 the same accuracy is reached with fewer vectors."""
+    A, _ = make_matrix(600, 300, "power", 20, seed=6)
+    r0 = AD.adaptive_sample(A, eps=1e-5, ell_inc=8, q=0, seed=9, ell_max=200)
+    r1 = AD.adaptive_sample(A, eps=1e-5, ell_inc=8, q=1, seed=9, ell_max=200)
+    assert r0.converged and r1.converged
+    assert r1.ell <= r0.ell
+
+
+@pytest.mark.slow
+def test_fig16_exponent_matrix_reaches_1e12_near_l_120_160():
+    """Fig. 16: exponent matrix, eps = 1e-12, l_init = l_inc = 8,
+    q = 0 reaches eps~ < 1e-12 at l ~ 120-160 (n = 500 suffices by rotation invariance)."""
+    A, _ = make_matrix(1000, 500, "exp-paper", 50, seed=7)
+    res = AD.adaptive_sample(A, eps=1e-12, ell_inc=8, q=0, seed=11, ell_max=400)
+    assert res.converged
+    assert 112 <= res.ell <= 176
+    ests = [e for _, e in res.history]
+    assert ests[-1] <= 1e-12 and ests[0] > 1e-2
