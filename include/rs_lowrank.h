@@ -63,7 +63,8 @@ typedef enum {
   RS_ERR_NOT_SPD = 5,        /* CholQR breakdown: Gram matrix not numerically SPD (see get_info) */
   RS_ERR_RANK_DEFICIENT = 6, /* QRCP found a zero residual norm before k steps (see get_info) */
   RS_ERR_WORKSPACE = 7,      /* workspace too small */
-  RS_ERR_UNSUPPORTED = 8     /* device is not sm_100 / size outside the supported range */
+  RS_ERR_UNSUPPORTED = 8,    /* device is not sm_100 / size outside the supported range */
+  RS_ERR_NOT_CONVERGED = 9   /* adaptive sampling reached l_max before eps~ <= eps */
 } rs_status_t;
 
 /* Bytes of device workspace rs_lowrank_create needs for these sizes (no device access). */
@@ -106,6 +107,19 @@ RS_API rs_status_t rs_lowrank_factor(rs_lowrank_t h, const double* A, int64_t ld
 RS_API rs_status_t rs_lowrank_run_host(rs_lowrank_t h, const double* A_host, int64_t lda, double* A_dev, int64_t ld_dev,
                                 int32_t q, int64_t* perm_host, double* Q_host, int64_t ldq, double* R_host,
                                 int64_t ldr, double* Q_dev, int64_t ld_qdev, double* R_dev, int64_t ld_rdev);
+
+/* Adaptive sample size for the fixed-accuracy problem (Fig. 3; Sec. 10):
+ * grows l by l_inc (a multiple of 8) per round -- new rows of the same Omega (Philox rows
+ * [l, l+l_inc)), q power iterations of the new block with block Gram-Schmidt (BCGS2) against
+ * the previous blocks (Fig. 2(a) lines 4/9), BOrth + CholQR2 of the block -- until the estimate
+ * eps~ = max_i ||b_i - b_i B^T B|| of the next block's rows is <= eps (bound (4)).
+ * The handle must be created with k = l_max and p = 0.  On return B holds l orthonormal rows and
+ * pivot/factor run with k = l.  history (host, may be NULL) receives up to history_len pairs
+ * (l, eps~).  Returns RS_ERR_NOT_CONVERGED (B still valid, *ell_out = l_max) if l_max is reached.
+ * Synchronises once per round (eps~ is read on the host).                                      */
+RS_API rs_status_t rs_lowrank_sample_adaptive(rs_lowrank_t h, const double* A, int64_t lda, double eps,
+                                              int32_t ell_inc, int32_t q, int32_t* ell_out, double* est_out,
+                                              double* history, int32_t history_len);
 
 RS_API rs_status_t rs_lowrank_destroy(rs_lowrank_t h);
 

@@ -170,6 +170,7 @@ static GemmArgs make_args(int M, int N, long long K, int splits, const GemmOutDe
   a.out.split_stride = out.split_stride;
   a.out.m_store = out.m_store;
   a.out.n_store = out.n_store;
+  a.out.mode = out.mode;
   return a;
 }
 
@@ -185,6 +186,7 @@ cudaError_t gemm_kc(cudaStream_t st, int M, int N, long long K, const View2D& Lv
     a.tag = phx.tag;
     a.row_offset = phx.row_offset;
     a.ell = phx.ell;
+    a.omega_row0 = phx.omega_row0;
     static const int gen_mode = [] {  // RS_PHILOX_GENMODE: cost experiments only (results invalid)
       const char* v = getenv("RS_PHILOX_GENMODE");
       return v ? atoi(v) : 0;

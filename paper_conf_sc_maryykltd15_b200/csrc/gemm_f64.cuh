@@ -41,7 +41,13 @@ struct GemmOut {
   long long ld_m, ld_n;       // element (m, n) at ptr[m*ld_m + n*ld_n]
   long long split_stride;     // + blockIdx.z * split_stride
   int m_store, n_store;       // store only m < m_store, n < n_store
+  int mode;                   // 0: out = acc, 1: out -= acc (block Gram-Schmidt updates)
 };
+
+RS_DEVINL void gemm_put(double* p, double v, int mode) {
+  if (mode) *p -= v;
+  else *p = v;
+}
 
 struct GemmArgs {
   int M, N;                   // rows / cols covered by the grid
@@ -52,7 +58,8 @@ struct GemmArgs {
   PhiloxKey key;
   uint32_t tag;
   long long row_offset;
-  int ell;
+  long long omega_row0;  // first Omega row of this tile set (adaptive rounds draw rows [l, l + l_inc))
+  int ell;               // number of Omega rows generated (rows >= ell of the tile are zero)
   int gen_mode;  // 0 = Philox + RS-BM32 (production); 1, 2 = generation-cost experiments only
 };
 
@@ -123,7 +130,7 @@ RS_DEVINL void kc_store(const double (&acc)[MFW][4][2], const GemmOut& ou, int m
 #pragma unroll
       for (int e = 0; e < 2; ++e) {
         const long long gn = n0 + 16 * (ng >> 1) + 8 * (ng & 1) + kk + 4 * e;
-        if (gn < ou.n_store) base[gm * ou.ld_m + gn * ou.ld_n] = acc[mf][nf][e];
+        if (gn < ou.n_store) gemm_put(base + gm * ou.ld_m + gn * ou.ld_n, acc[mf][nf][e], ou.mode);
       }
     }
   }
@@ -295,11 +302,11 @@ __global__ void __launch_bounds__(PHX_THREADS, 1)
             v0 = v1 = v2 = v3 = 1.0;
           }
         } else if (gi < a.ell) {
-          const float4 z = omega_block4f(static_cast<uint32_t>(gi), t0 + q, a.tag, a.key);
+          const float4 z = omega_block4f(static_cast<uint32_t>(a.omega_row0 + gi), t0 + q, a.tag, a.key);
           if (o == 0) {
             v0 = z.x, v1 = z.y, v2 = z.z, v3 = z.w;
           } else {
-            const float4 z2 = omega_block4f(static_cast<uint32_t>(gi), t0 + q + 1, a.tag, a.key);
+            const float4 z2 = omega_block4f(static_cast<uint32_t>(a.omega_row0 + gi), t0 + q + 1, a.tag, a.key);
             v0 = o + 0 < 4 ? f4_get(z, o + 0) : f4_get(z2, o - 4);
             v1 = o + 1 < 4 ? f4_get(z, o + 1) : f4_get(z2, o - 3);
             v2 = o + 2 < 4 ? f4_get(z, o + 2) : f4_get(z2, o - 2);
@@ -461,7 +468,7 @@ __global__ void __launch_bounds__(GEMM_THREADS, 1)
 #pragma unroll
         for (int e = 0; e < 2; ++e) {
           const long long gn = n0 + 16 * warp + 2 * (2 * kk + e) + f2;
-          if (gn < o.n_store) base[gm * o.ld_m + gn * o.ld_n] = acc[b][f][f2][e];
+          if (gn < o.n_store) gemm_put(base + gm * o.ld_m + gn * o.ld_n, acc[b][f][f2][e], o.mode);
         }
     }
 }

@@ -17,6 +17,7 @@ struct GemmOutDesc {
   double* ptr;
   long long ld_m, ld_n, split_stride;
   int m_store, n_store;
+  int mode = 0;  // 0: store, 1: subtract from the existing output
 };
 
 struct PhiloxDesc {
@@ -24,7 +25,8 @@ struct PhiloxDesc {
   uint64_t seed;
   uint32_t tag;
   long long row_offset;
-  int ell;
+  int ell;                   // Omega rows generated
+  long long omega_row0 = 0;  // first Omega row (global sample index)
 };
 
 // Out[M x N] (+split partials) = L[M x K] * R[K x N]
@@ -53,7 +55,9 @@ cudaError_t chol_inv(cudaStream_t st, const double* G, int ldg, int n, int npad,
 // C[M x N] = A[M x K] * B[K x N] (+ C if accumulate); element strides (row, col) for each.
 cudaError_t small_gemm(cudaStream_t st, int M, int N, int K, const double* A, long long a_rs, long long a_cs,
                        const double* B, long long b_rs, long long b_cs, double* C, long long c_rs, long long c_cs,
-                       bool accumulate);
+                       bool accumulate, double alpha = 1.0);
+// out[0] = max_i ||X[i, :]||_2 over rows i < rows (X column-major, ld)
+cudaError_t rows_maxnorm(cudaStream_t st, const double* X, long long ld, int rows, long long ncols, double* out);
 cudaError_t gather_cols(cudaStream_t st, const double* A, long long lda, long long m, const int64_t* perm, int k,
                         double* Q, long long ldq);
 cudaError_t permute_cols(cudaStream_t st, const double* Rorig, int ldro, int k, long long n, const int64_t* perm,

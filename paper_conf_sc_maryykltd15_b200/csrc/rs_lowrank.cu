@@ -78,7 +78,7 @@ Layout plan(long long m_local, long long n, int k, int p) {
   L.off_cholw = take(np16 * (np16 + 1) * 8);  // chol_inv work array (n > 128)
   L.off_Rho = take(static_cast<size_t>(L.kp) * n * 8);
   L.off_Rhat = take(static_cast<size_t>(L.kp) * n * 8);
-  L.off_T = take(static_cast<size_t>(L.kp) * std::max<long long>(n - k, 1) * 8);
+  L.off_T = take(static_cast<size_t>(L.kp) * std::max<long long>(n - 1, 1) * 8);  // adaptive runs use k < k0
   L.off_Q1 = take(static_cast<size_t>(L.ldq1) * std::max(k, 1) * 8);
   L.off_R1 = take(static_cast<size_t>(L.kp) * L.kp * 8);
   L.off_R2 = take(static_cast<size_t>(L.kp) * L.kp * 8);
@@ -96,6 +96,8 @@ Layout plan(long long m_local, long long n, int k, int p) {
 struct rs_lowrank_s {
   long long m_global, m_local, row_offset, n;
   int k, p, ell;
+  int k0;                // k at create (fixed-rank runs); adaptive runs set k = ell = l found
+  bool adaptive = false;
   uint64_t seed;
   cudaStream_t st;
   ncclComm_t comm;
@@ -224,37 +226,40 @@ rs_status_t gram_rows_kc(rs_lowrank_t h, const double* X, long long ldx, long lo
   return RS_OK;
 }
 
-// CholQR2 of the replicated short-wide X (lp x n, column-major, ld lp) into Y:
-// G = X X^T, R^T R = G, Y = R^{-T} X, twice.
-rs_status_t cholqr2_rows_small(rs_lowrank_t h, const double* X, double* Y) {
-  const Layout& L = h->L;
+// CholQR2 of a replicated short-wide block X (rp x n, column-major, ld rp; rows >= rr are zero)
+// into Y: G = X X^T, R^T R = G, Y = R^{-T} X, twice.
+rs_status_t cholqr2_block(rs_lowrank_t h, const double* X, int rr, int rp, double* Y) {
   const double* src = X;
   for (int pass = 0; pass < 2; ++pass) {
     double* dst = pass == 0 ? h->B1 : Y;
-    const int splits = gemm_choose_splits(L.lp, L.lp, h->n, max_splits_for(h, static_cast<long long>(L.lp) * L.lp), h->sms);
+    const int splits = gemm_choose_splits(rp, rp, h->n, max_splits_for(h, static_cast<long long>(rp) * rp), h->sms);
     const int ns = gemm_nsplit(h->n, splits);
     {
-      Scope sc(h, "gram", 2.0 * L.lp * L.lp * static_cast<double>(h->n));
-      View2D Xv{src, L.lp, h->n, L.lp};
-      GemmOutDesc out{h->part, 1, L.lp, static_cast<long long>(L.lp) * L.lp, L.lp, L.lp};
-      RS_CUDA(h, gemm_mc(h->st, L.lp, L.lp, h->n, Xv, Xv, out, splits));
+      Scope sc(h, "gram", 2.0 * rp * rp * static_cast<double>(h->n));
+      View2D Xv{src, rp, h->n, rp};
+      GemmOutDesc out{h->part, 1, rp, static_cast<long long>(rp) * rp, rp, rp};
+      RS_CUDA(h, gemm_mc(h->st, rp, rp, h->n, Xv, Xv, out, splits));
     }
     {
       Scope sc(h, "reduce", 0.0);
-      RS_CUDA(h, splitk_reduce(h->st, h->G, h->part, ns, static_cast<long long>(L.lp) * L.lp,
-                               static_cast<long long>(L.lp) * L.lp));
+      RS_CUDA(h, splitk_reduce(h->st, h->G, h->part, ns, static_cast<long long>(rp) * rp,
+                               static_cast<long long>(rp) * rp));
     }
     {
-      Scope sc(h, "chol", L.ell * static_cast<double>(L.ell) * L.ell / 3.0);
-      RS_CUDA(h, chol_inv(h->st, h->G, L.lp, L.ell, L.lp, h->Rf, L.lp, h->Linv, L.lp, h->cholw, h->info, RS_ERR_NOT_SPD));
+      Scope sc(h, "chol", rr * static_cast<double>(rr) * rr / 3.0);
+      RS_CUDA(h, chol_inv(h->st, h->G, rp, rr, rp, h->Rf, rp, h->Linv, rp, h->cholw, h->info, RS_ERR_NOT_SPD));
     }
     {
-      Scope sc(h, "apply", 2.0 * L.ell * L.ell * static_cast<double>(h->n));
-      RS_CUDA(h, small_gemm(h->st, L.lp, static_cast<int>(h->n), L.lp, h->Linv, 1, L.lp, src, 1, L.lp, dst, 1, L.lp, false));
+      Scope sc(h, "apply", 2.0 * rr * rr * static_cast<double>(h->n));
+      RS_CUDA(h, small_gemm(h->st, rp, static_cast<int>(h->n), rp, h->Linv, 1, rp, src, 1, rp, dst, 1, rp, false));
     }
     src = dst;
   }
   return RS_OK;
+}
+
+rs_status_t cholqr2_rows_small(rs_lowrank_t h, const double* X, double* Y) {
+  return cholqr2_block(h, X, h->L.ell, h->L.lp, Y);
 }
 
 rs_status_t check_matrix(rs_lowrank_t h, const void* p, long long ld, long long rows, const char* name) {
@@ -307,6 +312,7 @@ rs_status_t rs_lowrank_create(rs_lowrank_t* out, int64_t m_global, int64_t m_loc
   h->row_offset = row_offset;
   h->n = n;
   h->k = k;
+  h->k0 = k;
   h->p = p;
   h->ell = static_cast<int>(ell);
   h->seed = seed;
@@ -387,12 +393,16 @@ rs_status_t rs_lowrank_sample(rs_lowrank_t h, const double* A, int64_t lda) {
   if (s != RS_OK) return s;
   h->state = ST_SAMPLED;
   h->powers = 0;
+  h->ell = L.ell;
+  h->k = h->k0;
+  h->adaptive = false;
   return RS_OK;
 }
 
 rs_status_t rs_lowrank_power_iterate(rs_lowrank_t h, const double* A, int64_t lda, int32_t q) {
   if (!h) return RS_ERR_INVALID_ARG;
   if (h->state != ST_SAMPLED) return fail(h, RS_ERR_BAD_STATE, "power_iterate needs a fresh sample");
+  if (h->adaptive) return fail(h, RS_ERR_BAD_STATE, "the adaptive sample already includes its power iterations");
   if (q < 0) return fail(h, RS_ERR_INVALID_ARG, "q < 0");
   if (q == 0) return RS_OK;
   const Layout& L = h->L;
@@ -472,7 +482,7 @@ rs_status_t rs_lowrank_pivot(rs_lowrank_t h, int64_t* perm) {
   const Layout& L = h->L;
   {
     Scope sc(h, "qrcp", 0.0);
-    RS_CUDA(h, qrcp_truncated(h->st, h->B, L.lp, L.ell, h->n, h->k, h->qr, h->perm, h->Rho, L.kp, h->gaps, h->info,
+    RS_CUDA(h, qrcp_truncated(h->st, h->B, L.lp, h->ell, h->n, h->k, h->qr, h->perm, h->Rho, L.kp, h->gaps, h->info,
                               h->sms));
   }
   {
@@ -547,6 +557,223 @@ rs_status_t rs_lowrank_factor(rs_lowrank_t h, const double* A, int64_t lda, doub
   if (s != RS_OK) return s;
   h->state = ST_FACTORED;
   return RS_OK;
+}
+
+// ---------------------------------------------------------------------------------------------
+// Adaptive sample-size scheme (Fig. 3; readings R16-R19 in DESIGN.md)
+// ---------------------------------------------------------------------------------------------
+}  // extern "C"
+
+namespace {
+
+// Bn (rp x n, ld rp) := Bn - (Bn Bold^T) Bold, twice (BCGS2) -- replicated, no communication.
+rs_status_t borth_small(rs_lowrank_t h, const double* Bold, int ldo, int lold, double* Bn, int rp) {
+  if (lold <= 0) return RS_OK;
+  const long long n = h->n;
+  for (int pass = 0; pass < 2; ++pass) {
+    const int splits = gemm_choose_splits(rp, lold, n, max_splits_for(h, static_cast<long long>(rp) * lold), h->sms);
+    const int ns = gemm_nsplit(n, splits);
+    {
+      Scope sc(h, "borth", 2.0 * rp * lold * static_cast<double>(n));
+      View2D Xv{Bn, rp, n, rp};
+      View2D Ov{Bold, lold, n, ldo};
+      GemmOutDesc out{h->part, 1, rp, static_cast<long long>(rp) * lold, rp, lold};
+      RS_CUDA(h, gemm_mc(h->st, rp, lold, n, Xv, Ov, out, splits));
+      RS_CUDA(h, splitk_reduce(h->st, h->G, h->part, ns, static_cast<long long>(rp) * lold,
+                               static_cast<long long>(rp) * lold));
+      RS_CUDA(h, small_gemm(h->st, rp, static_cast<int>(n), lold, h->G, 1, rp, Bold, 1, ldo, Bn, 1, rp, true, -1.0));
+    }
+  }
+  return RS_OK;
+}
+
+// Cn (rr rows at Cn, row-major, ld ldc, distributed over ranks) := Cn - (Cn Cold^T) Cold, twice.
+rs_status_t borth_dist(rs_lowrank_t h, const double* Cold, int lold, double* Cn, int rr) {
+  if (lold <= 0) return RS_OK;
+  const Layout& L = h->L;
+  const long long ml = h->m_local;
+  for (int pass = 0; pass < 2; ++pass) {
+    const int splits = gemm_choose_splits(rr, lold, ml, max_splits_for(h, static_cast<long long>(rr) * lold), h->sms);
+    const int ns = gemm_nsplit(ml, splits);
+    Scope sc(h, "borth", 4.0 * rr * lold * static_cast<double>(ml));
+    if (ml > 0) {
+      View2D Xv{Cn, ml, rr, L.ldc};
+      View2D Ov{Cold, ml, lold, L.ldc};
+      GemmOutDesc out{h->part, 1, rr, static_cast<long long>(rr) * lold, rr, lold};
+      PhiloxDesc nophx{false, 0, 0, 0, 0};
+      RS_CUDA(h, gemm_kc(h->st, rr, lold, ml, Xv, Ov, nophx, out, splits));
+      RS_CUDA(h, splitk_reduce(h->st, h->G, h->part, ns, static_cast<long long>(rr) * lold,
+                               static_cast<long long>(rr) * lold));
+    } else {
+      RS_CUDA(h, cudaMemsetAsync(h->G, 0, static_cast<size_t>(rr) * lold * 8, h->st));
+    }
+    rs_status_t s = allreduce(h, h->G, static_cast<long long>(rr) * lold);
+    if (s != RS_OK) return s;
+    if (ml > 0) {
+      View2D Wv{h->G, rr, lold, rr};
+      View2D Ov{Cold, ml, lold, L.ldc};
+      GemmOutDesc out{Cn, L.ldc, 1, 0, rr, static_cast<int>(ml)};
+      out.mode = 1;  // Cn -= W Cold
+      RS_CUDA(h, gemm_mc(h->st, rr, static_cast<int>(ml), lold, Wv, Ov, out, 1));
+    }
+  }
+  return RS_OK;
+}
+
+// Bn (rr x n, ld rr) := Omega[row0 : row0+rr] A, summed over ranks
+rs_status_t sample_block(rs_lowrank_t h, const double* A, long long lda, int row0, int rr, double* Bn) {
+  const long long ml = h->m_local, n = h->n;
+  const long long cnt = static_cast<long long>(rr) * n;
+  if (ml > 0) {
+    const int splits = gemm_choose_splits(rr, static_cast<int>(n), ml, max_splits_for(h, cnt), h->sms);
+    const int ns = gemm_nsplit(ml, splits);
+    {
+      Scope sc(h, "gemm_sample", 2.0 * rr * static_cast<double>(ml) * n);
+      View2D Av{A, ml, n, lda};
+      GemmOutDesc out{h->part, 1, rr, cnt, rr, static_cast<int>(n)};
+      PhiloxDesc phx{true, h->seed, 0u, h->row_offset, rr};
+      phx.omega_row0 = row0;
+      RS_CUDA(h, gemm_kc(h->st, rr, static_cast<int>(n), ml, Av, Av, phx, out, splits));
+    }
+    Scope sc(h, "reduce", 0.0);
+    RS_CUDA(h, splitk_reduce(h->st, Bn, h->part, ns, cnt, cnt));
+  } else {
+    RS_CUDA(h, cudaMemsetAsync(Bn, 0, cnt * 8, h->st));
+  }
+  return allreduce(h, Bn, cnt);
+}
+
+// POWER (Fig. 2(a)) on the new block (rows [l, l+rr)) with BOrth against rows [0, l)
+rs_status_t power_block(rs_lowrank_t h, const double* A, long long lda, int l, int rr, int q, double* Bn) {
+  const Layout& L = h->L;
+  const long long ml = h->m_local, n = h->n;
+  const long long cnt = static_cast<long long>(rr) * n;
+  double* Cn = h->C + static_cast<long long>(l) * L.ldc;
+  rs_status_t s;
+  for (int it = 0; it < q; ++it) {
+    if ((s = borth_small(h, h->B, L.lp, l, Bn, rr)) != RS_OK) return s;        // line 4
+    if ((s = cholqr2_block(h, Bn, rr, rr, Bn)) != RS_OK) return s;            // line 5
+    if (ml > 0) {                                                               // line 7: C := B A^T
+      Scope sc(h, "gemm_power_c", 2.0 * rr * static_cast<double>(ml) * n);
+      View2D Bv{Bn, rr, n, rr};
+      View2D Av{A, ml, n, lda};
+      GemmOutDesc out{Cn, L.ldc, 1, 0, rr, static_cast<int>(ml)};
+      RS_CUDA(h, gemm_mc(h->st, rr, static_cast<int>(ml), n, Bv, Av, out, 1));
+    }
+    if ((s = borth_dist(h, h->C, l, Cn, rr)) != RS_OK) return s;              // line 9
+    // line 10: distributed CholQR2 of Cn, result stored back into C rows [l, l+rr)
+    for (int pass = 0; pass < 2; ++pass) {
+      const double* src = pass == 0 ? Cn : h->C1;
+      double* dst = pass == 0 ? h->C1 : Cn;
+      if ((s = gram_rows_kc(h, src, L.ldc, ml, rr, rr)) != RS_OK) return s;
+      if ((s = allreduce(h, h->G, static_cast<long long>(rr) * rr)) != RS_OK) return s;
+      {
+        Scope sc(h, "chol", rr * static_cast<double>(rr) * rr / 3.0);
+        RS_CUDA(h, chol_inv(h->st, h->G, rr, rr, rr, h->Rf, rr, h->Linv, rr, h->cholw, h->info, RS_ERR_NOT_SPD));
+      }
+      if (ml > 0) {
+        Scope sc(h, "apply", 2.0 * rr * static_cast<double>(rr) * ml);
+        View2D Lv{h->Linv, rr, rr, rr};
+        View2D Cv{src, ml, rr, L.ldc};
+        GemmOutDesc out{dst, L.ldc, 1, 0, rr, static_cast<int>(ml)};
+        RS_CUDA(h, gemm_mc(h->st, rr, static_cast<int>(ml), rr, Lv, Cv, out, 1));
+      }
+    }
+    // line 12: B := C A
+    if (ml > 0) {
+      const int splits = gemm_choose_splits(rr, static_cast<int>(n), ml, max_splits_for(h, cnt), h->sms);
+      const int ns = gemm_nsplit(ml, splits);
+      {
+        Scope sc(h, "gemm_power_b", 2.0 * rr * static_cast<double>(ml) * n);
+        View2D Cv{Cn, ml, rr, L.ldc};
+        View2D Av{A, ml, n, lda};
+        GemmOutDesc out{h->part, 1, rr, cnt, rr, static_cast<int>(n)};
+        PhiloxDesc nophx{false, 0, 0, 0, 0};
+        RS_CUDA(h, gemm_kc(h->st, rr, static_cast<int>(n), ml, Cv, Av, nophx, out, splits));
+      }
+      Scope sc(h, "reduce", 0.0);
+      RS_CUDA(h, splitk_reduce(h->st, Bn, h->part, ns, cnt, cnt));
+    } else {
+      RS_CUDA(h, cudaMemsetAsync(Bn, 0, cnt * 8, h->st));
+    }
+    if ((s = allreduce(h, Bn, cnt)) != RS_OK) return s;
+  }
+  return RS_OK;
+}
+
+}  // namespace
+
+extern "C" {
+
+rs_status_t rs_lowrank_sample_adaptive(rs_lowrank_t h, const double* A, int64_t lda, double eps, int32_t ell_inc,
+                                       int32_t q, int32_t* ell_out, double* est_out, double* history,
+                                       int32_t history_len) {
+  if (!h) return RS_ERR_INVALID_ARG;
+  const Layout& L = h->L;
+  if (h->p != 0) return fail(h, RS_ERR_INVALID_ARG, "adaptive sampling needs a handle created with p = 0 (k = l_max)");
+  if (ell_inc < 8 || ell_inc % 8 != 0 || ell_inc > L.ell || q < 0 || !(eps >= 0.0))
+    return fail(h, RS_ERR_INVALID_ARG, "need l_inc a positive multiple of 8, l_inc <= l_max, q >= 0, eps >= 0");
+  if (h->m_local > 0) {
+    rs_status_t s = check_matrix(h, A, lda, h->m_local, "A");
+    if (s != RS_OK) return s;
+  }
+  RS_CUDA(h, cudaMemsetAsync(h->info, 0, 16, h->st));
+  RS_CUDA(h, cudaMemsetAsync(h->B, 0, static_cast<size_t>(L.lp) * h->n * 8, h->st));
+  const int rr = ell_inc;
+  const long long n = h->n;
+  double* Bn = h->Bt;           // new block, rr x n, ld rr
+  double* E = h->Rho;           // error block rr x n (Rho is free until pivot)
+  double* dscal = h->gaps;      // device scalar for eps~
+  rs_status_t s = sample_block(h, A, lda, 0, rr, Bn);  // lines 2-3
+  if (s != RS_OK) return s;
+  int l = 0, hist = 0;
+  double est = -1.0;
+  bool converged = false;
+  for (;;) {
+    if ((s = power_block(h, A, lda, l, rr, q, Bn)) != RS_OK) return s;      // line 7
+    if ((s = borth_small(h, h->B, L.lp, l, Bn, rr)) != RS_OK) return s;      // line 8 (R17)
+    if ((s = cholqr2_block(h, Bn, rr, rr, Bn)) != RS_OK) return s;
+    RS_CUDA(h, copy_2d(h->st, Bn, rr, h->B + l, L.lp, rr, n));
+    l += rr;                                                                  // line 9
+    if (l + rr > L.ell) break;
+    if ((s = sample_block(h, A, lda, l, rr, Bn)) != RS_OK) return s;          // lines 12-13
+    // line 15: eps~ = max_i || b_i - b_i B_{1:l}^T B_{1:l} ||  (R18)
+    RS_CUDA(h, copy_2d(h->st, Bn, rr, E, rr, rr, n));
+    {
+      const int splits = gemm_choose_splits(rr, l, n, max_splits_for(h, static_cast<long long>(rr) * l), h->sms);
+      const int ns = gemm_nsplit(n, splits);
+      Scope sc(h, "borth", 4.0 * rr * l * static_cast<double>(n));
+      View2D Xv{Bn, rr, n, rr};
+      View2D Ov{h->B, l, n, L.lp};
+      GemmOutDesc out{h->part, 1, rr, static_cast<long long>(rr) * l, rr, l};
+      RS_CUDA(h, gemm_mc(h->st, rr, l, n, Xv, Ov, out, splits));
+      RS_CUDA(h, splitk_reduce(h->st, h->G, h->part, ns, static_cast<long long>(rr) * l,
+                               static_cast<long long>(rr) * l));
+      RS_CUDA(h, small_gemm(h->st, rr, static_cast<int>(n), l, h->G, 1, rr, h->B, 1, L.lp, E, 1, rr, true, -1.0));
+      RS_CUDA(h, rows_maxnorm(h->st, E, rr, rr, n, dscal));
+    }
+    RS_CUDA(h, cudaMemcpyAsync(&est, dscal, sizeof(double), cudaMemcpyDeviceToHost, h->st));
+    RS_CUDA(h, cudaStreamSynchronize(h->st));
+    if (history && hist < history_len) {
+      history[2 * hist] = l;
+      history[2 * hist + 1] = est;
+    }
+    ++hist;
+    if (est <= eps) {                                                         // line 16
+      converged = true;
+      break;
+    }
+  }
+  rs_status_t st = sync_and_check(h);
+  if (st != RS_OK) return st;
+  h->ell = l;
+  h->k = l;
+  h->adaptive = true;
+  h->state = ST_SAMPLED;
+  h->powers = q;
+  if (ell_out) *ell_out = l;
+  if (est_out) *est_out = est;
+  return converged ? RS_OK : fail(h, RS_ERR_NOT_CONVERGED, "eps~ = %g > eps after l = %d (l_max = %d)", est, l, L.ell);
 }
 
 rs_status_t rs_lowrank_run_host(rs_lowrank_t h, const double* A_host, int64_t lda, double* A_dev, int64_t ld_dev,

@@ -58,7 +58,8 @@ cudaError_t splitk_reduce(cudaStream_t st, double* out, const double* parts, int
 __global__ void __launch_bounds__(256) small_gemm_kernel(int M, int N, int K, const double* __restrict__ A,
                                                          long long a_rs, long long a_cs, const double* __restrict__ B,
                                                          long long b_rs, long long b_cs, double* __restrict__ C,
-                                                         long long c_rs, long long c_cs, bool accumulate) {
+                                                         long long c_rs, long long c_cs, bool accumulate,
+                                                         double alpha) {
   __shared__ double As[16][64 + 1];
   __shared__ double Bs[16][64 + 1];
   const int tx = threadIdx.x & 15, ty = threadIdx.x >> 4;
@@ -94,17 +95,17 @@ __global__ void __launch_bounds__(256) small_gemm_kernel(int M, int N, int K, co
       const int gm = m0 + ty + 16 * i, gn = n0 + tx + 16 * j;
       if (gm < M && gn < N) {
         double* p = C + gm * c_rs + gn * c_cs;
-        *p = accumulate ? *p + acc[i][j] : acc[i][j];
+        *p = accumulate ? fma(alpha, acc[i][j], *p) : alpha * acc[i][j];
       }
     }
 }
 
 cudaError_t small_gemm(cudaStream_t st, int M, int N, int K, const double* A, long long a_rs, long long a_cs,
                        const double* B, long long b_rs, long long b_cs, double* C, long long c_rs, long long c_cs,
-                       bool accumulate) {
+                       bool accumulate, double alpha) {
   if (M <= 0 || N <= 0) return cudaSuccess;
   dim3 grid((N + 63) / 64, (M + 63) / 64);
-  small_gemm_kernel<<<grid, 256, 0, st>>>(M, N, K, A, a_rs, a_cs, B, b_rs, b_cs, C, c_rs, c_cs, accumulate);
+  small_gemm_kernel<<<grid, 256, 0, st>>>(M, N, K, A, a_rs, a_cs, B, b_rs, b_cs, C, c_rs, c_cs, accumulate, alpha);
   count_launch();
   return cudaGetLastError();
 }
@@ -237,6 +238,38 @@ cudaError_t omega_materialize(cudaStream_t st, uint64_t seed, uint32_t tag, int 
   PhiloxKey key{static_cast<uint32_t>(seed), static_cast<uint32_t>(seed >> 32)};
   const int blocks = static_cast<int>(std::min<long long>((tot + 255) / 256, 148LL * 8));
   omega_kernel<<<blocks, 256, 0, st>>>(key, tag, ell, j0, ncols, out, ldo);
+  count_launch();
+  return cudaGetLastError();
+}
+
+// out[0] = max over rows of the row 2-norms of X (rows x ncols, column-major): the adaptive
+// scheme's error estimate eps~ (Fig. 3 line 15, reading R18).  One CTA.
+__global__ void rows_maxnorm_kernel(const double* __restrict__ X, long long ld, int rows, long long ncols,
+                                    double* out) {
+  __shared__ double red[1024 / 32];
+  double best = 0.0;
+  for (int i = 0; i < rows; ++i) {
+    double s = 0.0;
+    for (long long c = threadIdx.x; c < ncols; c += blockDim.x) {
+      const double x = X[i + c * ld];
+      s = fma(x, x, s);
+    }
+#pragma unroll
+    for (int o = 16; o > 0; o >>= 1) s += __shfl_xor_sync(0xffffffffu, s, o);
+    if ((threadIdx.x & 31) == 0) red[threadIdx.x >> 5] = s;
+    __syncthreads();
+    if (threadIdx.x == 0) {
+      double t = 0.0;
+      for (int w = 0; w < static_cast<int>(blockDim.x >> 5); ++w) t += red[w];
+      best = fmax(best, sqrt(t));
+    }
+    __syncthreads();
+  }
+  if (threadIdx.x == 0) out[0] = best;
+}
+
+cudaError_t rows_maxnorm(cudaStream_t st, const double* X, long long ld, int rows, long long ncols, double* out) {
+  rows_maxnorm_kernel<<<1, 1024, 0, st>>>(X, ld, rows, ncols, out);
   count_launch();
   return cudaGetLastError();
 }

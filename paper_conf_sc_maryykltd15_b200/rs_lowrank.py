@@ -21,11 +21,13 @@ _PKG = os.path.dirname(os.path.abspath(__file__))
 LIB_PATH = os.path.join(_PKG, "lib", "librs_lowrank.so")
 
 STATUS = {0: "RS_OK", 1: "RS_ERR_INVALID_ARG", 2: "RS_ERR_BAD_STATE", 3: "RS_ERR_CUDA", 4: "RS_ERR_NCCL",
-          5: "RS_ERR_NOT_SPD", 6: "RS_ERR_RANK_DEFICIENT", 7: "RS_ERR_WORKSPACE", 8: "RS_ERR_UNSUPPORTED"}
+          5: "RS_ERR_NOT_SPD", 6: "RS_ERR_RANK_DEFICIENT", 7: "RS_ERR_WORKSPACE", 8: "RS_ERR_UNSUPPORTED",
+          9: "RS_ERR_NOT_CONVERGED"}
 
 ABI_FUNCTIONS = (
     "rs_lowrank_workspace_bytes", "rs_lowrank_create", "rs_lowrank_sample", "rs_lowrank_power_iterate",
-    "rs_lowrank_pivot", "rs_lowrank_factor", "rs_lowrank_run_host", "rs_lowrank_destroy",
+    "rs_lowrank_pivot", "rs_lowrank_factor", "rs_lowrank_run_host", "rs_lowrank_sample_adaptive",
+    "rs_lowrank_destroy",
     "rs_lowrank_get_sample", "rs_lowrank_set_sample", "rs_lowrank_get_pivot_data", "rs_lowrank_omega",
     "rs_lowrank_get_info", "rs_lowrank_set_profiling", "rs_lowrank_get_profile", "rs_lowrank_reset_profile",
     "rs_lowrank_kernel_launches",
@@ -62,6 +64,8 @@ def load_library(path: str = LIB_PATH):
         "rs_lowrank_pivot": (ctypes.c_int, [P, P]),
         "rs_lowrank_factor": (ctypes.c_int, [P, P, I64, P, I64, P, I64]),
         "rs_lowrank_run_host": (ctypes.c_int, [P, P, I64, P, I64, I32, P, P, I64, P, I64, P, I64, P, I64]),
+        "rs_lowrank_sample_adaptive": (ctypes.c_int, [P, P, I64, ctypes.c_double, I32, I32, ctypes.POINTER(I32),
+                                                      D, D, I32]),
         "rs_lowrank_destroy": (ctypes.c_int, [P]),
         "rs_lowrank_get_sample": (ctypes.c_int, [P, P, I64]),
         "rs_lowrank_set_sample": (ctypes.c_int, [P, P, I64]),
@@ -142,10 +146,15 @@ class Handle:
     p: int
     seed: int
     stream: torch.cuda.Stream
+    adaptive_ell: int = 0  # set by sample_adaptive (then pivot/factor use k = l = adaptive_ell)
 
     @property
     def ell(self) -> int:
-        return self.k + self.p
+        return self.adaptive_ell or (self.k + self.p)
+
+    @property
+    def k_eff(self) -> int:
+        return self.adaptive_ell or self.k
 
 
 def create(m_global: int, m_local: int, row_offset: int, n: int, k: int, p: int, seed: int = 0x5C15, *,
@@ -166,6 +175,7 @@ def create(m_global: int, m_local: int, row_offset: int, n: int, k: int, p: int,
 
 def sample(h: Handle, A: torch.Tensor):
     _check(load_library().rs_lowrank_sample(h.ptr, A.data_ptr(), colmajor_ld(A, "A")), h.ptr)
+    h.adaptive_ell = 0
 
 
 def power_iterate(h: Handle, A: torch.Tensor, q: int):
@@ -192,6 +202,27 @@ def run_host(h: Handle, A_host: torch.Tensor, A_dev: torch.Tensor, q: int, perm_
         colmajor_ld(R_dev, "R_dev")), h.ptr)
 
 
+def sample_adaptive(h: Handle, A: torch.Tensor, eps: float, ell_inc: int, q: int = 0, *, raise_on_max=True):
+    """Fig. 3 adaptive sampling; returns (l, eps~, [(l, eps~) per round]).  The handle must have
+    been created with k = l_max and p = 0."""
+    ell = ctypes.c_int32()
+    est = ctypes.c_double()
+    hist = (ctypes.c_double * 2048)()
+    code = load_library().rs_lowrank_sample_adaptive(h.ptr, A.data_ptr(), colmajor_ld(A, "A"), eps, ell_inc, q,
+                                                     ctypes.byref(ell), ctypes.byref(est), hist, 1024)
+    rounds = []
+    for r in range(1024):
+        if hist[2 * r] == 0:
+            break
+        rounds.append((int(hist[2 * r]), hist[2 * r + 1]))
+    if code in (0, 9):
+        h.adaptive_ell = int(ell.value)
+    if code == 9 and not raise_on_max:
+        return int(ell.value), est.value, rounds
+    _check(code, h.ptr)
+    return int(ell.value), est.value, rounds
+
+
 def destroy(h: Handle):
     if h.ptr:
         _check(load_library().rs_lowrank_destroy(h.ptr))
@@ -211,12 +242,13 @@ def set_sample(h: Handle, B: torch.Tensor):
 def get_pivot_data(h: Handle):
     """(T k x (n-k), R̂ k x n in pivot order, gaps[k]) after pivot."""
     dev = h.workspace.device
-    T = empty_colmajor(h.k, max(h.n - h.k, 1), device=dev)
-    Rh = empty_colmajor(h.k, h.n, device=dev)
-    gaps = (ctypes.c_double * h.k)()
+    k = h.k_eff
+    T = empty_colmajor(k, max(h.n - k, 1), device=dev)
+    Rh = empty_colmajor(k, h.n, device=dev)
+    gaps = (ctypes.c_double * k)()
     _check(load_library().rs_lowrank_get_pivot_data(h.ptr, T.data_ptr(), colmajor_ld(T), Rh.data_ptr(),
                                                     colmajor_ld(Rh), gaps), h.ptr)
-    return T[:, : h.n - h.k], Rh, list(gaps)
+    return T[:, : h.n - k], Rh, list(gaps)
 
 
 def omega(h: Handle, j0: int, ncols: int) -> torch.Tensor:
