@@ -58,6 +58,8 @@ cudaError_t small_gemm(cudaStream_t st, int M, int N, int K, const double* A, lo
                        bool accumulate, double alpha = 1.0);
 // out[0] = max_i ||X[i, :]||_2 over rows i < rows (X column-major, ld)
 cudaError_t rows_maxnorm(cudaStream_t st, const double* X, long long ld, int rows, long long ncols, double* out);
+// G[i][i] += c * trace(G), i < n  (shifted CholeskyQR: c = 11 (N n + n(n+1)) u, ||X||_2^2 <= trace(G))
+cudaError_t shift_diag(cudaStream_t st, double* G, int ldg, int n, double c);
 cudaError_t gather_cols(cudaStream_t st, const double* A, long long lda, long long m, const int64_t* perm, int k,
                         double* Q, long long ldq);
 cudaError_t permute_cols(cudaStream_t st, const double* Rorig, int ldro, int k, long long n, const int64_t* perm,

@@ -228,10 +228,16 @@ rs_status_t gram_rows_kc(rs_lowrank_t h, const double* X, long long ldx, long lo
 
 // CholQR2 of a replicated short-wide block X (rp x n, column-major, ld rp; rows >= rr are zero)
 // into Y: G = X X^T, R^T R = G, Y = R^{-T} X, twice.
-rs_status_t cholqr2_block(rs_lowrank_t h, const double* X, int rr, int rp, double* Y) {
+// shifted = true: shifted CholeskyQR3 (a first pass on X X^T + s I with
+// s = 11 (n rp + rp (rp+1)) u ||X||_F^2, then CholQR2) -- breakdown-free for kappa(X) < ~1/u;
+// the remedy for "unstable for an ill-conditioned matrix" the paper lists.
+rs_status_t cholqr2_block(rs_lowrank_t h, const double* X, int rr, int rp, double* Y, bool shifted = false) {
   const double* src = X;
-  for (int pass = 0; pass < 2; ++pass) {
-    double* dst = pass == 0 ? h->B1 : Y;
+  const int npass = shifted ? 3 : 2;
+  for (int pass = 0; pass < npass; ++pass) {
+    // X -> B1 (-> Rho) -> Y: Y may alias X; Rho (k x n) is free outside pivot and holds rp x n
+    // whenever shifted passes are used (adaptive runs, p = 0)
+    double* dst = pass + 1 < npass ? (pass == 0 ? h->B1 : h->Rho) : Y;
     const int splits = gemm_choose_splits(rp, rp, h->n, max_splits_for(h, static_cast<long long>(rp) * rp), h->sms);
     const int ns = gemm_nsplit(h->n, splits);
     {
@@ -247,6 +253,8 @@ rs_status_t cholqr2_block(rs_lowrank_t h, const double* X, int rr, int rp, doubl
     }
     {
       Scope sc(h, "chol", rr * static_cast<double>(rr) * rr / 3.0);
+      if (shifted && pass == 0)
+        RS_CUDA(h, shift_diag(h->st, h->G, rp, rr, 11.0 * (static_cast<double>(h->n) * rr + rr * (rr + 1.0)) * 0x1p-53));
       RS_CUDA(h, chol_inv(h->st, h->G, rp, rr, rp, h->Rf, rp, h->Linv, rp, h->cholw, h->info, RS_ERR_NOT_SPD));
     }
     {
@@ -513,47 +521,74 @@ rs_status_t rs_lowrank_factor(rs_lowrank_t h, const double* A, int64_t lda, doub
     if ((s = check_matrix(h, Q, ldq, ml, "Q")) != RS_OK) return s;
   }
   if ((s = check_matrix(h, R, ldr, k, "R")) != RS_OK) return s;
-  // Q := A(:, P_{1:k})
-  if (ml > 0) {
-    Scope sc(h, "factor", 0.0);
-    RS_CUDA(h, gather_cols(h->st, A, lda, ml, h->perm, k, Q, ldq));
-  }
-  const double* src = Q;
-  long long ld_src = ldq;
-  for (int pass = 0; pass < 2; ++pass) {
-    double* dst = pass == 0 ? h->Q1 : Q;
-    const long long ld_dst = pass == 0 ? L.ldq1 : ldq;
-    // Gram G = X^T X (k x k) of the tall X = src (m_local x k column-major)
-    s = gram_rows_kc(h, src, ld_src, ml, k, L.kp);
-    if (s != RS_OK) return s;
-    s = allreduce(h, h->G, static_cast<long long>(L.kp) * L.kp);
-    if (s != RS_OK) return s;
-    double* Rk = pass == 0 ? h->R1 : h->R2;
-    {
-      Scope sc(h, "chol", k * static_cast<double>(k) * k / 3.0);
-      RS_CUDA(h, chol_inv(h->st, h->G, L.kp, k, L.kp, Rk, L.kp, h->Linv, L.kp, h->cholw, h->info, RS_ERR_NOT_SPD));
-    }
-    // dst = src * Rk^{-1}  (Rk^{-1}[kk, c] = Linv[c + kk*kp]: N-contiguous operand)
+  // CholQR with npass passes (even, so the last pass lands in Q); the first nshift Grams get
+  // + 11 (m k + k(k+1)) u ||X||_F^2 I (shifted CholeskyQR: each shifted pass is breakdown-free and
+  // cuts kappa by ~ 1/sqrt(11 m k u), so the plain passes that follow see kappa^2 u < 1)
+  auto run = [&](int npass, int nshift) -> rs_status_t {
+    // Q := A(:, P_{1:k})
     if (ml > 0) {
-      Scope sc(h, "factor", 2.0 * k * static_cast<double>(k) * ml);
-      View2D Xv{src, ml, k, ld_src};
-      View2D Wv{h->Linv, k, k, L.kp};
-      GemmOutDesc out{dst, 1, ld_dst, 0, static_cast<int>(ml), k};
-      RS_CUDA(h, gemm_mc(h->st, static_cast<int>(ml), k, k, Xv, Wv, out, 1));
+      Scope sc(h, "factor", 0.0);
+      RS_CUDA(h, gather_cols(h->st, A, lda, ml, h->perm, k, Q, ldq));
     }
-    src = dst;
-    ld_src = ld_dst;
+    const double* src = Q;
+    long long ld_src = ldq;
+    double* bufs[2] = {h->Rbar, h->R2};
+    int which = -1;  // index of the running product Rbar = R_p ... R_1 (-1: identity)
+    for (int pass = 0; pass < npass; ++pass) {
+      double* dst = pass % 2 == 0 ? h->Q1 : Q;
+      const long long ld_dst = pass % 2 == 0 ? L.ldq1 : ldq;
+      // Gram G = X^T X (k x k) of the tall X = src (m_local x k column-major)
+      rs_status_t st2 = gram_rows_kc(h, src, ld_src, ml, k, L.kp);
+      if (st2 != RS_OK) return st2;
+      st2 = allreduce(h, h->G, static_cast<long long>(L.kp) * L.kp);
+      if (st2 != RS_OK) return st2;
+      {
+        Scope sc(h, "chol", k * static_cast<double>(k) * k / 3.0);
+        if (pass < nshift)
+          RS_CUDA(h, shift_diag(h->st, h->G, L.kp, k,
+                                11.0 * (static_cast<double>(h->m_global) * k + k * (k + 1.0)) * 0x1p-53));
+        RS_CUDA(h, chol_inv(h->st, h->G, L.kp, k, L.kp, h->R1, L.kp, h->Linv, L.kp, h->cholw, h->info,
+                            RS_ERR_NOT_SPD));
+      }
+      // dst = src * R_p^{-1}  (R_p^{-1}[kk, c] = Linv[c + kk*kp]: N-contiguous operand)
+      if (ml > 0) {
+        Scope sc(h, "factor", 2.0 * k * static_cast<double>(k) * ml);
+        View2D Xv{src, ml, k, ld_src};
+        View2D Wv{h->Linv, k, k, L.kp};
+        GemmOutDesc out{dst, 1, ld_dst, 0, static_cast<int>(ml), k};
+        RS_CUDA(h, gemm_mc(h->st, static_cast<int>(ml), k, k, Xv, Wv, out, 1));
+      }
+      {
+        Scope sc(h, "other", 2.0 * k * static_cast<double>(k) * k);
+        if (which < 0) {
+          which = 0;
+          RS_CUDA(h, copy_2d(h->st, h->R1, L.kp, bufs[0], L.kp, L.kp, L.kp));
+        } else {  // Rbar := R_p Rbar
+          RS_CUDA(h, small_gemm(h->st, k, k, k, h->R1, 1, L.kp, bufs[which], 1, L.kp, bufs[1 - which], 1, L.kp,
+                                false));
+          which = 1 - which;
+        }
+      }
+      src = dst;
+      ld_src = ld_dst;
+    }
+    {
+      Scope sc(h, "other", 2.0 * k * static_cast<double>(k) * n);
+      // R = Rbar [I_k T]
+      RS_CUDA(h, copy_2d(h->st, bufs[which], L.kp, R, ldr, k, k));
+      if (n > k)
+        RS_CUDA(h, small_gemm(h->st, k, static_cast<int>(n - k), k, bufs[which], 1, L.kp, h->T, 1, L.kp,
+                              R + static_cast<long long>(k) * ldr, 1, ldr, false));
+    }
+    return sync_and_check(h);
+  };
+  // CholQR2; on breakdown (kappa(A P_1)^2 u > 1, e.g. an adaptive l past the numerical rank)
+  // shifted CholQR with 2, then 4 shifted passes ahead of the two plain ones (R20)
+  s = run(2, 0);
+  for (int nshift = 2; s == RS_ERR_NOT_SPD && nshift <= 4; nshift += 2) {
+    RS_CUDA(h, cudaMemsetAsync(h->info, 0, 16, h->st));
+    s = run(nshift + 2, nshift);
   }
-  {
-    Scope sc(h, "other", 2.0 * k * static_cast<double>(k) * n);
-    // Rbar = R2 R1 ; R = Rbar [I_k T]
-    RS_CUDA(h, small_gemm(h->st, k, k, k, h->R2, 1, L.kp, h->R1, 1, L.kp, h->Rbar, 1, L.kp, false));
-    RS_CUDA(h, copy_2d(h->st, h->Rbar, L.kp, R, ldr, k, k));
-    if (n > k)
-      RS_CUDA(h, small_gemm(h->st, k, static_cast<int>(n - k), k, h->Rbar, 1, L.kp, h->T, 1, L.kp,
-                            R + static_cast<long long>(k) * ldr, 1, ldr, false));
-  }
-  s = sync_and_check(h);
   if (s != RS_OK) return s;
   h->state = ST_FACTORED;
   return RS_OK;
@@ -566,11 +601,11 @@ rs_status_t rs_lowrank_factor(rs_lowrank_t h, const double* A, int64_t lda, doub
 
 namespace {
 
-// Bn (rp x n, ld rp) := Bn - (Bn Bold^T) Bold, twice (BCGS2) -- replicated, no communication.
+// Bn (rp x n, ld rp) := Bn - (Bn Bold^T) Bold (one BCGS projection) -- replicated, no communication.
 rs_status_t borth_small(rs_lowrank_t h, const double* Bold, int ldo, int lold, double* Bn, int rp) {
   if (lold <= 0) return RS_OK;
   const long long n = h->n;
-  for (int pass = 0; pass < 2; ++pass) {
+  {
     const int splits = gemm_choose_splits(rp, lold, n, max_splits_for(h, static_cast<long long>(rp) * lold), h->sms);
     const int ns = gemm_nsplit(n, splits);
     {
@@ -587,12 +622,12 @@ rs_status_t borth_small(rs_lowrank_t h, const double* Bold, int ldo, int lold, d
   return RS_OK;
 }
 
-// Cn (rr rows at Cn, row-major, ld ldc, distributed over ranks) := Cn - (Cn Cold^T) Cold, twice.
+// Cn (rr rows at Cn, row-major, ld ldc, distributed over ranks) := Cn - (Cn Cold^T) Cold (one pass).
 rs_status_t borth_dist(rs_lowrank_t h, const double* Cold, int lold, double* Cn, int rr) {
   if (lold <= 0) return RS_OK;
   const Layout& L = h->L;
   const long long ml = h->m_local;
-  for (int pass = 0; pass < 2; ++pass) {
+  {
     const int splits = gemm_choose_splits(rr, lold, ml, max_splits_for(h, static_cast<long long>(rr) * lold), h->sms);
     const int ns = gemm_nsplit(ml, splits);
     Scope sc(h, "borth", 4.0 * rr * lold * static_cast<double>(ml));
@@ -616,6 +651,59 @@ rs_status_t borth_dist(rs_lowrank_t h, const double* Cold, int lold, double* Cn,
       out.mode = 1;  // Cn -= W Cold
       RS_CUDA(h, gemm_mc(h->st, rr, static_cast<int>(ml), lold, Wv, Ov, out, 1));
     }
+  }
+  return RS_OK;
+}
+
+// BOrth + QR of a replicated block (R17): twice { project against B_{1:l}; block CholQR }.  The
+// first CholQR is the shifted CholQR3 (the projected block may be ill-conditioned), the second
+// acts on a block that is orthonormal to O(kappa u), where CholQR2 is exact to O(u).
+rs_status_t borth_qr_small(rs_lowrank_t h, int lold, double* Bn, int rr) {
+  rs_status_t s;
+  if (lold <= 0) return cholqr2_block(h, Bn, rr, rr, Bn, true);
+  for (int pass = 0; pass < 2; ++pass) {
+    if ((s = borth_small(h, h->B, h->L.lp, lold, Bn, rr)) != RS_OK) return s;
+    if ((s = cholqr2_block(h, Bn, rr, rr, Bn, pass == 0)) != RS_OK) return s;
+  }
+  return RS_OK;
+}
+
+// Distributed CholQR of Cn (rr rows of C, row-major, ld ldc): npass passes, the first shifted
+// when `shifted`; the result ends in Cn (npass even).
+rs_status_t cholqr_dist(rs_lowrank_t h, double* Cn, int rr, int npass, bool shifted) {
+  const Layout& L = h->L;
+  const long long ml = h->m_local;
+  rs_status_t s;
+  for (int pass = 0; pass < npass; ++pass) {
+    const double* src = pass % 2 == 0 ? Cn : h->C1;
+    double* dst = pass % 2 == 0 ? h->C1 : Cn;
+    if ((s = gram_rows_kc(h, src, L.ldc, ml, rr, rr)) != RS_OK) return s;
+    if ((s = allreduce(h, h->G, static_cast<long long>(rr) * rr)) != RS_OK) return s;
+    {
+      Scope sc(h, "chol", rr * static_cast<double>(rr) * rr / 3.0);
+      if (shifted && pass == 0)
+        RS_CUDA(h, shift_diag(h->st, h->G, rr, rr,
+                              11.0 * (static_cast<double>(h->m_global) * rr + rr * (rr + 1.0)) * 0x1p-53));
+      RS_CUDA(h, chol_inv(h->st, h->G, rr, rr, rr, h->Rf, rr, h->Linv, rr, h->cholw, h->info, RS_ERR_NOT_SPD));
+    }
+    if (ml > 0) {
+      Scope sc(h, "apply", 2.0 * rr * static_cast<double>(rr) * ml);
+      View2D Lv{h->Linv, rr, rr, rr};
+      View2D Cv{src, ml, rr, L.ldc};
+      GemmOutDesc out{dst, L.ldc, 1, 0, rr, static_cast<int>(ml)};
+      RS_CUDA(h, gemm_mc(h->st, rr, static_cast<int>(ml), rr, Lv, Cv, out, 1));
+    }
+  }
+  return RS_OK;
+}
+
+// BOrth + QR of a distributed C block (R17), as borth_qr_small.
+rs_status_t borth_qr_dist(rs_lowrank_t h, int lold, double* Cn, int rr) {
+  rs_status_t s;
+  if (lold <= 0) return cholqr_dist(h, Cn, rr, 4, true);
+  for (int pass = 0; pass < 2; ++pass) {
+    if ((s = borth_dist(h, h->C, lold, Cn, rr)) != RS_OK) return s;
+    if ((s = cholqr_dist(h, Cn, rr, pass == 0 ? 4 : 2, pass == 0)) != RS_OK) return s;
   }
   return RS_OK;
 }
@@ -651,8 +739,7 @@ rs_status_t power_block(rs_lowrank_t h, const double* A, long long lda, int l, i
   double* Cn = h->C + static_cast<long long>(l) * L.ldc;
   rs_status_t s;
   for (int it = 0; it < q; ++it) {
-    if ((s = borth_small(h, h->B, L.lp, l, Bn, rr)) != RS_OK) return s;        // line 4
-    if ((s = cholqr2_block(h, Bn, rr, rr, Bn)) != RS_OK) return s;            // line 5
+    if ((s = borth_qr_small(h, l, Bn, rr)) != RS_OK) return s;                  // lines 4-5
     if (ml > 0) {                                                               // line 7: C := B A^T
       Scope sc(h, "gemm_power_c", 2.0 * rr * static_cast<double>(ml) * n);
       View2D Bv{Bn, rr, n, rr};
@@ -660,25 +747,7 @@ rs_status_t power_block(rs_lowrank_t h, const double* A, long long lda, int l, i
       GemmOutDesc out{Cn, L.ldc, 1, 0, rr, static_cast<int>(ml)};
       RS_CUDA(h, gemm_mc(h->st, rr, static_cast<int>(ml), n, Bv, Av, out, 1));
     }
-    if ((s = borth_dist(h, h->C, l, Cn, rr)) != RS_OK) return s;              // line 9
-    // line 10: distributed CholQR2 of Cn, result stored back into C rows [l, l+rr)
-    for (int pass = 0; pass < 2; ++pass) {
-      const double* src = pass == 0 ? Cn : h->C1;
-      double* dst = pass == 0 ? h->C1 : Cn;
-      if ((s = gram_rows_kc(h, src, L.ldc, ml, rr, rr)) != RS_OK) return s;
-      if ((s = allreduce(h, h->G, static_cast<long long>(rr) * rr)) != RS_OK) return s;
-      {
-        Scope sc(h, "chol", rr * static_cast<double>(rr) * rr / 3.0);
-        RS_CUDA(h, chol_inv(h->st, h->G, rr, rr, rr, h->Rf, rr, h->Linv, rr, h->cholw, h->info, RS_ERR_NOT_SPD));
-      }
-      if (ml > 0) {
-        Scope sc(h, "apply", 2.0 * rr * static_cast<double>(rr) * ml);
-        View2D Lv{h->Linv, rr, rr, rr};
-        View2D Cv{src, ml, rr, L.ldc};
-        GemmOutDesc out{dst, L.ldc, 1, 0, rr, static_cast<int>(ml)};
-        RS_CUDA(h, gemm_mc(h->st, rr, static_cast<int>(ml), rr, Lv, Cv, out, 1));
-      }
-    }
+    if ((s = borth_qr_dist(h, l, Cn, rr)) != RS_OK) return s;                   // lines 9-10
     // line 12: B := C A
     if (ml > 0) {
       const int splits = gemm_choose_splits(rr, static_cast<int>(n), ml, max_splits_for(h, cnt), h->sms);
@@ -731,8 +800,7 @@ rs_status_t rs_lowrank_sample_adaptive(rs_lowrank_t h, const double* A, int64_t 
   bool converged = false;
   for (;;) {
     if ((s = power_block(h, A, lda, l, rr, q, Bn)) != RS_OK) return s;      // line 7
-    if ((s = borth_small(h, h->B, L.lp, l, Bn, rr)) != RS_OK) return s;      // line 8 (R17)
-    if ((s = cholqr2_block(h, Bn, rr, rr, Bn)) != RS_OK) return s;
+    if ((s = borth_qr_small(h, l, Bn, rr)) != RS_OK) return s;                // line 8 (R17)
     RS_CUDA(h, copy_2d(h->st, Bn, rr, h->B + l, L.lp, rr, n));
     l += rr;                                                                  // line 9
     if (l + rr > L.ell) break;

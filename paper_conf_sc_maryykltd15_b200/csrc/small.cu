@@ -275,3 +275,33 @@ cudaError_t rows_maxnorm(cudaStream_t st, const double* X, long long ld, int row
 }
 
 }  // namespace rs
+
+namespace rs {
+
+// Shift for shifted CholeskyQR (breakdown-free first pass for ill-conditioned blocks):
+// G[i][i] += c * trace(G).  One CTA.
+__global__ void shift_diag_kernel(double* G, int ldg, int n, double c) {
+  __shared__ double red[32];
+  double s = 0.0;
+  for (int i = threadIdx.x; i < n; i += blockDim.x) s += G[i + static_cast<long long>(i) * ldg];
+#pragma unroll
+  for (int o = 16; o > 0; o >>= 1) s += __shfl_xor_sync(0xffffffffu, s, o);
+  if ((threadIdx.x & 31) == 0) red[threadIdx.x >> 5] = s;
+  __syncthreads();
+  __shared__ double tr;
+  if (threadIdx.x == 0) {
+    double t = 0.0;
+    for (int w = 0; w < static_cast<int>(blockDim.x >> 5); ++w) t += red[w];
+    tr = t;
+  }
+  __syncthreads();
+  for (int i = threadIdx.x; i < n; i += blockDim.x) G[i + static_cast<long long>(i) * ldg] += c * tr;
+}
+
+cudaError_t shift_diag(cudaStream_t st, double* G, int ldg, int n, double c) {
+  shift_diag_kernel<<<1, 256, 0, st>>>(G, ldg, n, c);
+  count_launch();
+  return cudaGetLastError();
+}
+
+}  // namespace rs

@@ -24,6 +24,30 @@ def test_bcgs2_makes_rows_orthogonal():
     np.testing.assert_array_equal(AD.bcgs2(np.zeros((0, 40)), Y), Y)
 
 
+def test_borth_qr_equals_qr_of_the_projection():
+    """R17: in exact arithmetic the two-pass form is QR(Y - Y X^T X); the rows are orthonormal and
+    orthogonal to X, and the positive-diagonal LQ factor ties the result to one basis."""
+    rng = np.random.default_rng(1)
+    X, _ = rows_orth(rng.standard_normal((6, 50)))
+    Y = rng.standard_normal((4, 50))
+    Z = AD.borth_qr(X, Y)
+    np.testing.assert_allclose(Z @ Z.T, np.eye(4), atol=1e-14)
+    assert np.abs(Z @ X.T).max() <= 1e-14
+    P = np.eye(50) - X.T @ X                      # textbook projector, then one Householder QR
+    Zt, _ = rows_orth(Y @ P)
+    np.testing.assert_allclose(Z, Zt, atol=1e-13)
+    np.testing.assert_allclose(AD.borth_qr(np.zeros((0, 50)), Y), rows_orth(Y)[0], atol=0)
+
+
+def test_basis_stays_orthonormal_past_the_numerical_rank():
+    """Exponent matrix (sigma_i = 10^(-i/10)) sampled to l = 256 > numerical rank ~160 with
+    l_inc = 32: every block past the rank is rounding noise, yet B B^T = I to O(u) (R17)."""
+    A, _ = make_matrix(1500, 600, "exp-paper", 50, seed=8)
+    res = AD.adaptive_sample(A, eps=0.0, ell_inc=32, q=0, seed=3, ell_max=256)
+    assert res.ell == 256
+    assert np.abs(res.B @ res.B.T - np.eye(256)).max() <= 1e-13
+
+
 def test_single_round_q0_equals_fixed_rank_orthonormal_sample():
     """One round with l_inc = l: B = QR(Omega[0:l] A), the fixed-rank sample (R16)."""
     A, _ = make_matrix(300, 80, "exp-paper", 10, seed=1)
