@@ -138,6 +138,12 @@ RS_API rs_status_t rs_lowrank_omega(rs_lowrank_t h, int64_t j0, int64_t ncols, d
 /* info[0] = status code of the first device-detected failure (0 if none), info[1] = 1-based
  * failing Cholesky column / QRCP step.  Synchronises.                                        */
 RS_API rs_status_t rs_lowrank_get_info(rs_lowrank_t h, int64_t* info);
+/* CholQR breakdown fallbacks taken (R20), host-side, no sync:
+ *  counts[0] = power iterations since the last sample redone with shifted CholQR on B and C
+ *              (2 shifted + 2 plain passes each) after the plain CholQR2 broke down;
+ *  counts[1] = shifted passes the last factor call put ahead of its two plain CholQR passes
+ *              (0 = plain CholQR2 succeeded, 2 or 4 = shifted CholQR4 / CholQR6).            */
+RS_API rs_status_t rs_lowrank_get_fallbacks(rs_lowrank_t h, int32_t* counts);
 /* Per-kernel-class device time (ms, CUDA events on the handle's stream) accumulated while
  * profiling is enabled.  names: "gemm_sample", "gemm_power_c", "gemm_power_b", "gram",
  * "apply", "chol", "qrcp", "factor", "reduce", "comm", "other".                              */

@@ -98,6 +98,8 @@ struct rs_lowrank_s {
   int k, p, ell;
   int k0;                // k at create (fixed-rank runs); adaptive runs set k = ell = l found
   bool adaptive = false;
+  int robust_iters = 0;   // power iterations redone with shifted CholQR since the last sample
+  int factor_shifts = 0;  // shifted CholQR passes the last factor needed (0: plain CholQR2)
   uint64_t seed;
   cudaStream_t st;
   ncclComm_t comm;
@@ -226,11 +228,38 @@ rs_status_t gram_rows_kc(rs_lowrank_t h, const double* X, long long ldx, long lo
   return RS_OK;
 }
 
-// CholQR2 of a replicated short-wide block X (rp x n, column-major, ld rp; rows >= rr are zero)
-// into Y: G = X X^T, R^T R = G, Y = R^{-T} X, twice.
-// shifted = true: shifted CholeskyQR3 (a first pass on X X^T + s I with
-// s = 11 (n rp + rp (rp+1)) u ||X||_F^2, then CholQR2) -- breakdown-free for kappa(X) < ~1/u;
+// One CholQR pass on a replicated short-wide block X (rp x n, column-major, ld rp; rows >= rr are
+// zero): G = X X^T (+ s I when shift), R^T R = G, Y = R^{-T} X.  The shift
+// s = 11 (n rr + rr (rr+1)) u ||X||_F^2 is shifted CholeskyQR's: breakdown-free for kappa(X) < ~1/u,
 // the remedy for "unstable for an ill-conditioned matrix" the paper lists.
+rs_status_t cholqr_small_pass(rs_lowrank_t h, const double* src, int rr, int rp, double* dst, bool shift) {
+  const int splits = gemm_choose_splits(rp, rp, h->n, max_splits_for(h, static_cast<long long>(rp) * rp), h->sms);
+  const int ns = gemm_nsplit(h->n, splits);
+  {
+    Scope sc(h, "gram", 2.0 * rp * rp * static_cast<double>(h->n));
+    View2D Xv{src, rp, h->n, rp};
+    GemmOutDesc out{h->part, 1, rp, static_cast<long long>(rp) * rp, rp, rp};
+    RS_CUDA(h, gemm_mc(h->st, rp, rp, h->n, Xv, Xv, out, splits));
+  }
+  {
+    Scope sc(h, "reduce", 0.0);
+    RS_CUDA(h, splitk_reduce(h->st, h->G, h->part, ns, static_cast<long long>(rp) * rp,
+                             static_cast<long long>(rp) * rp));
+  }
+  {
+    Scope sc(h, "chol", rr * static_cast<double>(rr) * rr / 3.0);
+    if (shift)
+      RS_CUDA(h, shift_diag(h->st, h->G, rp, rr, 11.0 * (static_cast<double>(h->n) * rr + rr * (rr + 1.0)) * 0x1p-53));
+    RS_CUDA(h, chol_inv(h->st, h->G, rp, rr, rp, h->Rf, rp, h->Linv, rp, h->cholw, h->info, RS_ERR_NOT_SPD));
+  }
+  {
+    Scope sc(h, "apply", 2.0 * rr * rr * static_cast<double>(h->n));
+    RS_CUDA(h, small_gemm(h->st, rp, static_cast<int>(h->n), rp, h->Linv, 1, rp, src, 1, rp, dst, 1, rp, false));
+  }
+  return RS_OK;
+}
+
+// CholQR2 of X into Y (shifted = false), or shifted CholQR3 (one shifted pass, then CholQR2).
 rs_status_t cholqr2_block(rs_lowrank_t h, const double* X, int rr, int rp, double* Y, bool shifted = false) {
   const double* src = X;
   const int npass = shifted ? 3 : 2;
@@ -238,30 +267,38 @@ rs_status_t cholqr2_block(rs_lowrank_t h, const double* X, int rr, int rp, doubl
     // X -> B1 (-> Rho) -> Y: Y may alias X; Rho (k x n) is free outside pivot and holds rp x n
     // whenever shifted passes are used (adaptive runs, p = 0)
     double* dst = pass + 1 < npass ? (pass == 0 ? h->B1 : h->Rho) : Y;
-    const int splits = gemm_choose_splits(rp, rp, h->n, max_splits_for(h, static_cast<long long>(rp) * rp), h->sms);
-    const int ns = gemm_nsplit(h->n, splits);
-    {
-      Scope sc(h, "gram", 2.0 * rp * rp * static_cast<double>(h->n));
-      View2D Xv{src, rp, h->n, rp};
-      GemmOutDesc out{h->part, 1, rp, static_cast<long long>(rp) * rp, rp, rp};
-      RS_CUDA(h, gemm_mc(h->st, rp, rp, h->n, Xv, Xv, out, splits));
-    }
-    {
-      Scope sc(h, "reduce", 0.0);
-      RS_CUDA(h, splitk_reduce(h->st, h->G, h->part, ns, static_cast<long long>(rp) * rp,
-                               static_cast<long long>(rp) * rp));
-    }
+    rs_status_t s = cholqr_small_pass(h, src, rr, rp, dst, shifted && pass == 0);
+    if (s != RS_OK) return s;
+    src = dst;
+  }
+  return RS_OK;
+}
+
+// Distributed CholQR of the rows [Cn, Cn + rp) of C (row-major, ld ldc; rows >= rr are zero):
+// npass passes (even: the result ends in Cn, C1 is the ping-pong buffer), the first nshift shifted.
+rs_status_t cholqr_dist(rs_lowrank_t h, double* Cn, int rr, int rp, int npass, int nshift) {
+  const Layout& L = h->L;
+  const long long ml = h->m_local;
+  rs_status_t s;
+  for (int pass = 0; pass < npass; ++pass) {
+    const double* src = pass % 2 == 0 ? Cn : h->C1;
+    double* dst = pass % 2 == 0 ? h->C1 : Cn;
+    if ((s = gram_rows_kc(h, src, L.ldc, ml, rp, rp)) != RS_OK) return s;
+    if ((s = allreduce(h, h->G, static_cast<long long>(rp) * rp)) != RS_OK) return s;
     {
       Scope sc(h, "chol", rr * static_cast<double>(rr) * rr / 3.0);
-      if (shifted && pass == 0)
-        RS_CUDA(h, shift_diag(h->st, h->G, rp, rr, 11.0 * (static_cast<double>(h->n) * rr + rr * (rr + 1.0)) * 0x1p-53));
+      if (pass < nshift)
+        RS_CUDA(h, shift_diag(h->st, h->G, rp, rr,
+                              11.0 * (static_cast<double>(h->m_global) * rr + rr * (rr + 1.0)) * 0x1p-53));
       RS_CUDA(h, chol_inv(h->st, h->G, rp, rr, rp, h->Rf, rp, h->Linv, rp, h->cholw, h->info, RS_ERR_NOT_SPD));
     }
-    {
-      Scope sc(h, "apply", 2.0 * rr * rr * static_cast<double>(h->n));
-      RS_CUDA(h, small_gemm(h->st, rp, static_cast<int>(h->n), rp, h->Linv, 1, rp, src, 1, rp, dst, 1, rp, false));
+    if (ml > 0) {
+      Scope sc(h, "apply", 2.0 * rr * static_cast<double>(rr) * ml);
+      View2D Lv{h->Linv, rp, rp, rp};
+      View2D Cv{src, ml, rp, L.ldc};
+      GemmOutDesc out{dst, L.ldc, 1, 0, rp, static_cast<int>(ml)};
+      RS_CUDA(h, gemm_mc(h->st, rp, static_cast<int>(ml), rp, Lv, Cv, out, 1));
     }
-    src = dst;
   }
   return RS_OK;
 }
@@ -401,6 +438,7 @@ rs_status_t rs_lowrank_sample(rs_lowrank_t h, const double* A, int64_t lda) {
   if (s != RS_OK) return s;
   h->state = ST_SAMPLED;
   h->powers = 0;
+  h->robust_iters = 0;
   h->ell = L.ell;
   h->k = h->k0;
   h->adaptive = false;
@@ -420,11 +458,28 @@ rs_status_t rs_lowrank_power_iterate(rs_lowrank_t h, const double* A, int64_t ld
   }
   const long long ml = h->m_local, n = h->n;
   const long long lxn = static_cast<long long>(L.lp) * n;
-  for (int it = 0; it < q; ++it) {
-    // line 5: B := QR(B)  (replicated CholQR2)
-    rs_status_t s = cholqr2_rows_small(h, h->B, h->Bt);
-    if (s != RS_OK) return s;
-    // line 7: C := B A^T   (C row-major lp x ldc: C[i, j] at i*ldc + j)
+  // line 12: dst := Csrc A summed over ranks
+  auto gemm_b = [&](const double* Csrc, double* dst) -> rs_status_t {
+    if (ml > 0) {
+      const int splits = gemm_choose_splits(L.lp, static_cast<int>(n), ml, max_splits_for(h, lxn), h->sms);
+      const int ns = gemm_nsplit(ml, splits);
+      {
+        Scope sc(h, "gemm_power_b", 2.0 * h->ell * static_cast<double>(ml) * n);
+        View2D Cv{Csrc, ml, L.lp, L.ldc};
+        View2D Av{A, ml, n, lda};
+        GemmOutDesc out{h->part, 1, L.lp, lxn, L.lp, static_cast<int>(n)};
+        PhiloxDesc nophx{false, 0, 0, 0, 0};
+        RS_CUDA(h, gemm_kc(h->st, L.lp, static_cast<int>(n), ml, Cv, Av, nophx, out, splits));
+      }
+      Scope sc(h, "reduce", 0.0);
+      RS_CUDA(h, splitk_reduce(h->st, dst, h->part, ns, lxn, lxn));
+    } else {
+      RS_CUDA(h, cudaMemsetAsync(dst, 0, lxn * 8, h->st));
+    }
+    return allreduce(h, dst, lxn);
+  };
+  // line 7: C := Bt A^T   (C row-major lp x ldc: C[i, j] at i*ldc + j)
+  auto gemm_c = [&]() -> rs_status_t {
     if (ml > 0) {
       Scope sc(h, "gemm_power_c", 2.0 * h->ell * static_cast<double>(ml) * n);
       View2D Bv{h->Bt, L.lp, n, L.lp};
@@ -432,6 +487,13 @@ rs_status_t rs_lowrank_power_iterate(rs_lowrank_t h, const double* A, int64_t ld
       GemmOutDesc out{h->C, L.ldc, 1, 0, L.lp, static_cast<int>(ml)};
       RS_CUDA(h, gemm_mc(h->st, L.lp, static_cast<int>(ml), n, Bv, Av, out, 1));
     }
+    return RS_OK;
+  };
+  for (int it = 0; it < q; ++it) {
+    // line 5: B := QR(B)  (replicated CholQR2)
+    rs_status_t s = cholqr2_rows_small(h, h->B, h->Bt);
+    if (s != RS_OK) return s;
+    if ((s = gemm_c()) != RS_OK) return s;
     // line 10: C := QR(C)  (distributed CholQR2; the second R^{-T} is applied to B below)
     s = gram_rows_kc(h, h->C, L.ldc, ml, L.lp, L.lp);
     if (s != RS_OK) return s;
@@ -457,25 +519,26 @@ rs_status_t rs_lowrank_power_iterate(rs_lowrank_t h, const double* A, int64_t ld
       RS_CUDA(h, chol_inv(h->st, h->G, L.lp, L.ell, L.lp, h->Rf, L.lp, h->Linv, L.lp, h->cholw, h->info, RS_ERR_NOT_SPD));
     }
     // line 12: B := C A   (B1 = C1 A summed over ranks; then B = R2^{-T} B1, exact re-association)
-    if (ml > 0) {
-      const int splits = gemm_choose_splits(L.lp, static_cast<int>(n), ml, max_splits_for(h, lxn), h->sms);
-      const int ns = gemm_nsplit(ml, splits);
-      {
-        Scope sc(h, "gemm_power_b", 2.0 * h->ell * static_cast<double>(ml) * n);
-        View2D Cv{h->C1, ml, L.lp, L.ldc};
-        View2D Av{A, ml, n, lda};
-        GemmOutDesc out{h->part, 1, L.lp, lxn, L.lp, static_cast<int>(n)};
-        PhiloxDesc nophx{false, 0, 0, 0, 0};
-        RS_CUDA(h, gemm_kc(h->st, L.lp, static_cast<int>(n), ml, Cv, Av, nophx, out, splits));
+    if ((s = gemm_b(h->C1, h->B1)) != RS_OK) return s;
+    // B is still this iteration's input: on a CholQR breakdown (kappa^2 u > 1) redo the
+    // iteration with shifted CholQR (2 shifted + 2 plain passes on B and on C, R20).  The Gram
+    // matrices are replicated, so every rank takes the same branch.
+    int info[2] = {0, 0};
+    RS_CUDA(h, cudaMemcpyAsync(info, h->info, sizeof(info), cudaMemcpyDeviceToHost, h->st));
+    RS_CUDA(h, cudaStreamSynchronize(h->st));
+    if (info[0] == RS_ERR_NOT_SPD) {
+      RS_CUDA(h, cudaMemsetAsync(h->info, 0, 16, h->st));
+      const double* src = h->B;
+      for (int pass = 0; pass < 4; ++pass) {  // B -> B1 -> Bt -> B1 -> Bt
+        double* dst = pass % 2 == 0 ? h->B1 : h->Bt;
+        if ((s = cholqr_small_pass(h, src, L.ell, L.lp, dst, pass < 2)) != RS_OK) return s;
+        src = dst;
       }
-      Scope sc(h, "reduce", 0.0);
-      RS_CUDA(h, splitk_reduce(h->st, h->B1, h->part, ns, lxn, lxn));
+      if ((s = gemm_c()) != RS_OK) return s;
+      if ((s = cholqr_dist(h, h->C, L.ell, L.lp, 4, 2)) != RS_OK) return s;
+      if ((s = gemm_b(h->C, h->B)) != RS_OK) return s;
+      h->robust_iters++;
     } else {
-      RS_CUDA(h, cudaMemsetAsync(h->B1, 0, lxn * 8, h->st));
-    }
-    s = allreduce(h, h->B1, lxn);
-    if (s != RS_OK) return s;
-    {
       Scope sc(h, "apply", 2.0 * L.ell * static_cast<double>(L.ell) * n);
       RS_CUDA(h, small_gemm(h->st, L.lp, static_cast<int>(n), L.lp, h->Linv, 1, L.lp, h->B1, 1, L.lp, h->B, 1, L.lp, false));
     }
@@ -585,9 +648,11 @@ rs_status_t rs_lowrank_factor(rs_lowrank_t h, const double* A, int64_t lda, doub
   // CholQR2; on breakdown (kappa(A P_1)^2 u > 1, e.g. an adaptive l past the numerical rank)
   // shifted CholQR with 2, then 4 shifted passes ahead of the two plain ones (R20)
   s = run(2, 0);
+  h->factor_shifts = 0;
   for (int nshift = 2; s == RS_ERR_NOT_SPD && nshift <= 4; nshift += 2) {
     RS_CUDA(h, cudaMemsetAsync(h->info, 0, 16, h->st));
     s = run(nshift + 2, nshift);
+    h->factor_shifts = nshift;
   }
   if (s != RS_OK) return s;
   h->state = ST_FACTORED;
@@ -668,42 +733,13 @@ rs_status_t borth_qr_small(rs_lowrank_t h, int lold, double* Bn, int rr) {
   return RS_OK;
 }
 
-// Distributed CholQR of Cn (rr rows of C, row-major, ld ldc): npass passes, the first shifted
-// when `shifted`; the result ends in Cn (npass even).
-rs_status_t cholqr_dist(rs_lowrank_t h, double* Cn, int rr, int npass, bool shifted) {
-  const Layout& L = h->L;
-  const long long ml = h->m_local;
-  rs_status_t s;
-  for (int pass = 0; pass < npass; ++pass) {
-    const double* src = pass % 2 == 0 ? Cn : h->C1;
-    double* dst = pass % 2 == 0 ? h->C1 : Cn;
-    if ((s = gram_rows_kc(h, src, L.ldc, ml, rr, rr)) != RS_OK) return s;
-    if ((s = allreduce(h, h->G, static_cast<long long>(rr) * rr)) != RS_OK) return s;
-    {
-      Scope sc(h, "chol", rr * static_cast<double>(rr) * rr / 3.0);
-      if (shifted && pass == 0)
-        RS_CUDA(h, shift_diag(h->st, h->G, rr, rr,
-                              11.0 * (static_cast<double>(h->m_global) * rr + rr * (rr + 1.0)) * 0x1p-53));
-      RS_CUDA(h, chol_inv(h->st, h->G, rr, rr, rr, h->Rf, rr, h->Linv, rr, h->cholw, h->info, RS_ERR_NOT_SPD));
-    }
-    if (ml > 0) {
-      Scope sc(h, "apply", 2.0 * rr * static_cast<double>(rr) * ml);
-      View2D Lv{h->Linv, rr, rr, rr};
-      View2D Cv{src, ml, rr, L.ldc};
-      GemmOutDesc out{dst, L.ldc, 1, 0, rr, static_cast<int>(ml)};
-      RS_CUDA(h, gemm_mc(h->st, rr, static_cast<int>(ml), rr, Lv, Cv, out, 1));
-    }
-  }
-  return RS_OK;
-}
-
 // BOrth + QR of a distributed C block (R17), as borth_qr_small.
 rs_status_t borth_qr_dist(rs_lowrank_t h, int lold, double* Cn, int rr) {
   rs_status_t s;
-  if (lold <= 0) return cholqr_dist(h, Cn, rr, 4, true);
+  if (lold <= 0) return cholqr_dist(h, Cn, rr, rr, 4, 1);
   for (int pass = 0; pass < 2; ++pass) {
     if ((s = borth_dist(h, h->C, lold, Cn, rr)) != RS_OK) return s;
-    if ((s = cholqr_dist(h, Cn, rr, pass == 0 ? 4 : 2, pass == 0)) != RS_OK) return s;
+    if ((s = cholqr_dist(h, Cn, rr, rr, pass == 0 ? 4 : 2, pass == 0 ? 1 : 0)) != RS_OK) return s;
   }
   return RS_OK;
 }
@@ -921,6 +957,13 @@ rs_status_t rs_lowrank_get_info(rs_lowrank_t h, int64_t* info) {
   RS_CUDA(h, cudaMemcpy(v, h->info, sizeof(v), cudaMemcpyDeviceToHost));
   info[0] = v[0];
   info[1] = v[1];
+  return RS_OK;
+}
+
+rs_status_t rs_lowrank_get_fallbacks(rs_lowrank_t h, int32_t* counts) {
+  if (!h || !counts) return RS_ERR_INVALID_ARG;
+  counts[0] = h->robust_iters;
+  counts[1] = h->factor_shifts;
   return RS_OK;
 }
 

@@ -29,7 +29,7 @@ ABI_FUNCTIONS = (
     "rs_lowrank_pivot", "rs_lowrank_factor", "rs_lowrank_run_host", "rs_lowrank_sample_adaptive",
     "rs_lowrank_destroy",
     "rs_lowrank_get_sample", "rs_lowrank_set_sample", "rs_lowrank_get_pivot_data", "rs_lowrank_omega",
-    "rs_lowrank_get_info", "rs_lowrank_set_profiling", "rs_lowrank_get_profile", "rs_lowrank_reset_profile",
+    "rs_lowrank_get_info", "rs_lowrank_get_fallbacks", "rs_lowrank_set_profiling", "rs_lowrank_get_profile", "rs_lowrank_reset_profile",
     "rs_lowrank_kernel_launches",
     "rs_lowrank_last_error", "rs_comm_get_unique_id", "rs_comm_init", "rs_comm_destroy",
 )
@@ -72,6 +72,7 @@ def load_library(path: str = LIB_PATH):
         "rs_lowrank_get_pivot_data": (ctypes.c_int, [P, P, I64, P, I64, D]),
         "rs_lowrank_omega": (ctypes.c_int, [P, I64, I64, P, I64]),
         "rs_lowrank_get_info": (ctypes.c_int, [P, ctypes.POINTER(I64)]),
+        "rs_lowrank_get_fallbacks": (ctypes.c_int, [P, ctypes.POINTER(I32)]),
         "rs_lowrank_set_profiling": (ctypes.c_int, [P, I32]),
         "rs_lowrank_get_profile": (ctypes.c_int, [P, ctypes.c_char_p, D, ctypes.POINTER(I64), D]),
         "rs_lowrank_reset_profile": (ctypes.c_int, [P]),
@@ -260,6 +261,13 @@ def omega(h: Handle, j0: int, ncols: int) -> torch.Tensor:
 def get_info(h: Handle):
     arr = (ctypes.c_int64 * 2)()
     _check(load_library().rs_lowrank_get_info(h.ptr, arr), h.ptr)
+    return int(arr[0]), int(arr[1])
+
+
+def get_fallbacks(h: Handle):
+    """(power iterations redone with shifted CholQR, shifted passes of the last factor)."""
+    arr = (ctypes.c_int32 * 2)()
+    _check(load_library().rs_lowrank_get_fallbacks(h.ptr, arr), h.ptr)
     return int(arr[0]), int(arr[1])
 
 
