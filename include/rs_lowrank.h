@@ -155,6 +155,27 @@ RS_API rs_status_t rs_lowrank_reset_profile(rs_lowrank_t h);
 RS_API int64_t rs_lowrank_kernel_launches(void);
 RS_API const char* rs_lowrank_last_error(rs_lowrank_t h);
 
+/* ---- the paper's deterministic baseline: truncated QP3 of A itself (one GPU) ----
+ * Householder QR with column pivoting stopped after k columns (Sec. 2; "QP3" of
+ * Figs. 7, 10-14), blocked like LAPACK dgeqp3/dlaqps: panels of 32 columns, delayed trailing
+ * updates, downdated column norms with LAPACK's cancellation test (a failing column's norm is
+ * recomputed exactly on the device).  Pivot rule: largest residual column norm, ties -> lowest
+ * original index; perm in LAPACK swap order.
+ *  A (device, m x n, lda >= m even, 16-byte aligned) is overwritten LAPACK-style: rows 0..k-1
+ *    hold R (upper trapezoidal, k x n, columns in perm order), the columns 0..k-1 below the
+ *    diagonal hold the Householder vectors (unit leading entry implicit); the trailing block
+ *    A(k:m, k:n) holds R22 if residual_host != NULL, else it is only partly updated.
+ *  perm (device int64[n]), tau (device double[k]): outputs; caller-owned.
+ *  residual_host (may be NULL): receives ||R22||_F (the error of Fig. 6's "QP3" column is
+ *    ||R22||_F / ||A||_F); requesting it adds the last panel's trailing update and synchronises.
+ *  workspace: device, 256-byte aligned, >= rs_qp3_workspace_bytes(m, n, k).
+ *  cuda_stream: cudaStream_t (NULL = legacy default stream).  Enqueues only (no synchronisation)
+ *    unless residual_host != NULL.  Errors: RS_ERR_INVALID_ARG, RS_ERR_WORKSPACE, RS_ERR_CUDA. */
+RS_API size_t rs_qp3_workspace_bytes(int64_t m, int64_t n, int32_t k);
+RS_API rs_status_t rs_qp3_truncated(int64_t m, int64_t n, int32_t k, double* A, int64_t lda, int64_t* perm,
+                                    double* tau, double* residual_host, void* workspace, size_t workspace_bytes,
+                                    void* cuda_stream);
+
 /* ---- NCCL plumbing (the harness exchanges the id with torch.distributed) ---- */
 RS_API rs_status_t rs_comm_get_unique_id(char id_out[128]);
 RS_API rs_status_t rs_comm_init(void** comm, int32_t nranks, const char id[128], int32_t rank);

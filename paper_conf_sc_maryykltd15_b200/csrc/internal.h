@@ -76,4 +76,9 @@ size_t qrcp_workspace_bytes(int ell, long long n);
 cudaError_t qrcp_truncated(cudaStream_t st, const double* B, int ldb, int ell, long long n, int k, void* work,
                            int64_t* perm, double* Rhat_orig, int ldr, double* gaps, int* info, int num_sms);
 
+// truncated QP3 of the full A (qp3.cu): the paper's deterministic baseline
+size_t qp3_workspace_bytes(long long m, long long n);
+cudaError_t qp3_truncated_large(cudaStream_t st, double* A, long long lda, long long m, long long n, int k,
+                                void* work, int64_t* perm, double* tau, bool want_residual, double* residual);
+
 }  // namespace rs

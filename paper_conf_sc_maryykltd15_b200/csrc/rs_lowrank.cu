@@ -993,6 +993,24 @@ rs_status_t rs_lowrank_reset_profile(rs_lowrank_t h) {
 
 int64_t rs_lowrank_kernel_launches(void) { return rs::launch_count(); }
 
+size_t rs_qp3_workspace_bytes(int64_t m, int64_t n, int32_t k) {
+  (void)k;
+  return m > 0 && n > 0 ? qp3_workspace_bytes(m, n) : 0;
+}
+
+rs_status_t rs_qp3_truncated(int64_t m, int64_t n, int32_t k, double* A, int64_t lda, int64_t* perm, double* tau,
+                             double* residual_host, void* workspace, size_t workspace_bytes, void* cuda_stream) {
+  if (m < 1 || n < 1 || k < 1 || k > std::min<int64_t>(m, n)) return RS_ERR_INVALID_ARG;
+  if (!A || !perm || !tau || !workspace) return RS_ERR_INVALID_ARG;
+  if (reinterpret_cast<uintptr_t>(A) % 16 != 0 || lda < m || lda % 2 != 0) return RS_ERR_INVALID_ARG;
+  if (workspace_bytes < qp3_workspace_bytes(m, n)) return RS_ERR_WORKSPACE;
+  if (reinterpret_cast<uintptr_t>(workspace) % 256 != 0) return RS_ERR_INVALID_ARG;
+  cudaStream_t st = static_cast<cudaStream_t>(cuda_stream);
+  const cudaError_t e = qp3_truncated_large(st, A, lda, m, n, k, workspace, perm, tau, residual_host != nullptr,
+                                            residual_host);
+  return e == cudaSuccess ? RS_OK : RS_ERR_CUDA;
+}
+
 const char* rs_lowrank_last_error(rs_lowrank_t h) { return h ? h->err.c_str() : "null handle"; }
 
 rs_status_t rs_comm_get_unique_id(char id_out[128]) {

@@ -30,7 +30,7 @@ ABI_FUNCTIONS = (
     "rs_lowrank_destroy",
     "rs_lowrank_get_sample", "rs_lowrank_set_sample", "rs_lowrank_get_pivot_data", "rs_lowrank_omega",
     "rs_lowrank_get_info", "rs_lowrank_get_fallbacks", "rs_lowrank_set_profiling", "rs_lowrank_get_profile", "rs_lowrank_reset_profile",
-    "rs_lowrank_kernel_launches",
+    "rs_lowrank_kernel_launches", "rs_qp3_workspace_bytes", "rs_qp3_truncated",
     "rs_lowrank_last_error", "rs_comm_get_unique_id", "rs_comm_init", "rs_comm_destroy",
 )
 
@@ -77,6 +77,8 @@ def load_library(path: str = LIB_PATH):
         "rs_lowrank_get_profile": (ctypes.c_int, [P, ctypes.c_char_p, D, ctypes.POINTER(I64), D]),
         "rs_lowrank_reset_profile": (ctypes.c_int, [P]),
         "rs_lowrank_kernel_launches": (I64, []),
+        "rs_qp3_workspace_bytes": (SZ, [I64, I64, I32]),
+        "rs_qp3_truncated": (ctypes.c_int, [I64, I64, I32, P, I64, P, P, D, P, SZ, P]),
         "rs_lowrank_last_error": (ctypes.c_char_p, [P]),
         "rs_comm_get_unique_id": (ctypes.c_int, [ctypes.c_char_p]),
         "rs_comm_init": (ctypes.c_int, [ctypes.POINTER(P), I32, ctypes.c_char_p, I32]),
@@ -297,6 +299,39 @@ def reset_profile(h: Handle):
 
 def kernel_launches() -> int:
     return int(load_library().rs_lowrank_kernel_launches())
+
+
+class Qp3:
+    """Workspace for the truncated QP3 baseline of an m x n matrix (rs_qp3_truncated)."""
+
+    def __init__(self, m: int, n: int, k: int, device=None):
+        device = torch.device("cuda", torch.cuda.current_device()) if device is None else torch.device(device)
+        self.m, self.n, self.k = m, n, k
+        nbytes = int(load_library().rs_qp3_workspace_bytes(m, n, k))
+        if nbytes == 0:
+            raise RSError(1, "invalid sizes")
+        self.workspace = torch.empty(nbytes, dtype=torch.uint8, device=device)
+        self.perm = torch.empty(n, dtype=torch.int64, device=device)
+        self.tau = torch.empty(max(k, 1), dtype=torch.float64, device=device)
+
+    def run(self, A: torch.Tensor, *, residual: bool = False, stream=None):
+        """Overwrites A (LAPACK layout: R in rows < k, reflectors below).  Returns ||R22||_F when
+        residual=True (synchronises), else None."""
+        res = ctypes.c_double(-1.0)
+        code = load_library().rs_qp3_truncated(
+            self.m, self.n, self.k, A.data_ptr(), colmajor_ld(A, "A"), self.perm.data_ptr(), self.tau.data_ptr(),
+            ctypes.byref(res) if residual else None, self.workspace.data_ptr(), self.workspace.numel(),
+            _stream_ptr(stream))
+        _check(code)
+        return res.value if residual else None
+
+
+def qp3_truncated(A: torch.Tensor, k: int, *, residual: bool = False):
+    """Truncated QP3 of A (overwritten).  Returns (perm, tau, ||R22||_F or None)."""
+    m, n = A.shape
+    q = Qp3(m, n, k, device=A.device)
+    res = q.run(A, residual=residual)
+    return q.perm, q.tau, res
 
 
 def last_error(h: Handle) -> str:
