@@ -7,7 +7,7 @@
 //
 // B200 design (memory-bound: every step streams the trailing matrix once through the GEMV that
 // forms F(:, j), "about half of its flops using BLAS-2"):
-//  * per step six small kernels and no host synchronisation -- the pivot index, the reflector and
+//  * per step four kernels and no host synchronisation -- the pivot index, the reflector and
 //    the list of norms to recompute live in device memory;
 //  * the trailing GEMV reads A column-major with 16-byte loads, the reflector staged in shared
 //    memory, deterministic two-stage reduction;
@@ -17,6 +17,7 @@
 //    recomputed" without ending the panel early;
 //  * the per-panel trailing update (rank NB, ~4 flop/byte: HBM-bound) is a DFMA tile kernel that
 //    also recomputes every trailing column norm exactly while the tile is in registers.
+#include <algorithm>
 #include <cmath>
 
 #include "common.cuh"
@@ -32,19 +33,20 @@ constexpr int QP3_GV_CPW = 2;          // GEMV: columns per warp
 constexpr int QP3_GV_COLS = 8 * QP3_GV_CPW;
 constexpr int QP3_UP_ROWS = 128;       // trailing update: rows per sub-tile (4 per lane)
 constexpr int QP3_UP_SUB = 8;          // sub-tiles per CTA (1024 rows)
-constexpr int QP3_UP_COLS = 64;        // columns per CTA (8 per warp)
+constexpr int QP3_UP_COLS = 32;        // columns per CTA (4 per warp)
 
 struct Qp3Scalars {
   double beta, tau, scale, res;
   long long pvt;
-  int nflag, pad;
+  int nflag;
+  unsigned int done;  // CTAs of the pivot kernel that finished (last one forms the reflector)
 };
 
 struct Qp3Work {
   Qp3Scalars* sc;
   double* vn1;     // n
   double* vn2;     // n
-  double* F;       // n x NB (ld n)
+  double* F;       // n x NB, row-major: F(c, t) at F[c * NB + t]
   double* parts_a; // QP3_A_CTAS
   double* parts;   // nch x n (GEMV / trailing-update partial sums)
   int* flags;      // n
@@ -109,16 +111,27 @@ __global__ void __launch_bounds__(QP3_T) qp3_init_kernel(const double* __restric
                                                          Qp3Scalars* sc) {
   const long long c = static_cast<long long>(blockIdx.x) * 8 + (threadIdx.x >> 5);
   const int lane = threadIdx.x & 31;
-  if (blockIdx.x == 0 && threadIdx.x == 0) sc->nflag = 0;
+  if (blockIdx.x == 0 && threadIdx.x == 0) {
+    sc->nflag = 0;
+    sc->done = 0;
+  }
   if (c >= n) return;
   const double* col = A + c * lda;
-  double s = 0.0;
+  double s = 0.0, s4[4] = {0.0, 0.0, 0.0, 0.0};
   const long long m2 = m & ~1LL;
-  for (long long i = 2 * lane; i < m2; i += 64) {
-    const double2 x = *reinterpret_cast<const double2*>(col + i);
-    s = fma(x.x, x.x, s);
-    s = fma(x.y, x.y, s);
+  long long i = 2 * lane;
+  for (; i + 192 < m2; i += 256) {  // four independent 16-byte loads in flight per lane
+    double2 x[4];
+#pragma unroll
+    for (int u = 0; u < 4; ++u) x[u] = *reinterpret_cast<const double2*>(col + i + 64 * u);
+#pragma unroll
+    for (int u = 0; u < 4; ++u) s4[u] = fma(x[u].y, x[u].y, fma(x[u].x, x[u].x, s4[u]));
   }
+  for (; i < m2; i += 64) {
+    const double2 x = *reinterpret_cast<const double2*>(col + i);
+    s = fma(x.y, x.y, fma(x.x, x.x, s));
+  }
+  s += (s4[0] + s4[1]) + (s4[2] + s4[3]);
   if ((m & 1) && lane == 0) s = fma(col[m - 1], col[m - 1], s);
   s = warp_sum(s);
   if (lane == 0) {
@@ -128,14 +141,14 @@ __global__ void __launch_bounds__(QP3_T) qp3_init_kernel(const double* __restric
   }
 }
 
-// ---- step (a): pivot choice, column swap, delayed update of the pivot column ----------------
+// ---- steps (a)+(b): pivot choice, column swap, delayed update of the pivot column, reflector -----
 // A(rk:m, j) := A(rk:m, pvt) - A(rk:m, j0:j) F(pvt, 0:kk)^T, A(:, pvt) := old A(:, j);
-// parts_a[cta] = partial sum of squares of the new A(rk+1:m, j).
+// parts_a[cta] = partial sum of squares of the new A(rk+1:m, j); the last CTA to finish sums the
+// partials in index order, forms the dlarfg reflector and swaps perm / vn / F rows.
 __global__ void __launch_bounds__(QP3_T) qp3_pivot_kernel(double* __restrict__ A, long long lda, long long m,
                                                           long long n, long long j, long long j0, int kk,
-                                                          const double* __restrict__ vn1, const int64_t* perm,
-                                                          const double* __restrict__ F, double* parts_a,
-                                                          Qp3Scalars* sc) {
+                                                          double* vn1, double* vn2, int64_t* perm, double* F,
+                                                          double* parts_a, double* tau_out, Qp3Scalars* sc) {
   __shared__ double s_best[QP3_T / 32];
   __shared__ long long s_idx[QP3_T / 32], s_org[QP3_T / 32];
   __shared__ double s_f[QP3_NB];
@@ -144,7 +157,25 @@ __global__ void __launch_bounds__(QP3_T) qp3_pivot_kernel(double* __restrict__ A
   // largest residual norm, ties -> lowest original column index (reading R5 / oracle rule)
   double best = -1.0;
   long long bi = -1, bo = 0;
-  for (long long c = j + threadIdx.x; c < n; c += blockDim.x) {
+  long long c = j + threadIdx.x;
+  for (; c + 7 * blockDim.x < n; c += 8 * blockDim.x) {  // eight independent loads in flight
+    double v[8];
+    long long o[8];
+#pragma unroll
+    for (int u = 0; u < 8; ++u) {
+      v[u] = vn1[c + u * blockDim.x];
+      o[u] = perm[c + u * blockDim.x];
+    }
+#pragma unroll
+    for (int u = 0; u < 8; ++u) {
+      if (v[u] > best || (v[u] == best && o[u] < bo)) {
+        best = v[u];
+        bi = c + u * blockDim.x;
+        bo = o[u];
+      }
+    }
+  }
+  for (; c < n; c += blockDim.x) {
     const double v = vn1[c];
     const long long o = perm[c];
     if (v > best || (v == best && o < bo)) {
@@ -186,7 +217,7 @@ __global__ void __launch_bounds__(QP3_T) qp3_pivot_kernel(double* __restrict__ A
   }
   __syncthreads();
   const long long pvt = s_pvt;
-  if (threadIdx.x < kk) s_f[threadIdx.x] = F[pvt + static_cast<long long>(threadIdx.x) * n];
+  if (threadIdx.x < kk) s_f[threadIdx.x] = F[pvt * QP3_NB + threadIdx.x];
   __syncthreads();
   const long long rk = j;
   double ss = 0.0;
@@ -197,28 +228,28 @@ __global__ void __launch_bounds__(QP3_T) qp3_pivot_kernel(double* __restrict__ A
     double a = colp[i];
     if (pvt != j) colp[i] = colj[i];
     if (i >= rk) {
+#pragma unroll 8
       for (int t = 0; t < kk; ++t) a = fma(-A[i + (j0 + t) * lda], s_f[t], a);
       if (i > rk) ss = fma(a, a, ss);
     }
     colj[i] = a;
   }
   ss = block_sum(ss, red);
-  if (threadIdx.x == 0) parts_a[blockIdx.x] = ss;
-}
-
-// ---- step (b): reflector (dlarfg) and bookkeeping --------------------------------------------
-__global__ void __launch_bounds__(1024) qp3_reflector_kernel(const double* __restrict__ A, long long lda,
-                                                              long long n, long long j, int kk, int nparts,
-                                                              const double* __restrict__ parts_a, double* vn1,
-                                                              double* vn2, int64_t* perm, double* F, double* tau_out,
-                                                              Qp3Scalars* sc) {
-  __shared__ double red[32];
-  double v = 0.0;
-  for (int i = threadIdx.x; i < nparts; i += blockDim.x) v += parts_a[i];
-  const double xnorm2 = block_sum(v, red);
-  const long long pvt = sc->pvt;
+  __shared__ bool s_last;
   if (threadIdx.x == 0) {
-    const double alpha = A[j + j * lda];
+    parts_a[blockIdx.x] = ss;
+    __threadfence();
+    s_last = atomicAdd(&sc->done, 1u) == gridDim.x - 1;
+  }
+  __syncthreads();
+  if (!s_last) return;
+  // ---- step (b), last CTA: reflector (dlarfg) and bookkeeping ----
+  __threadfence();
+  double v = 0.0;
+  for (int i = threadIdx.x; i < static_cast<int>(gridDim.x); i += blockDim.x) v += __ldcg(parts_a + i);
+  const double xnorm2 = block_sum(v, red);
+  if (threadIdx.x == 0) {
+    const double alpha = __ldcg(colj + rk);
     const double xnorm = sqrt(xnorm2);
     double beta = alpha, tau = 0.0, scale = 0.0;
     if (xnorm != 0.0) {
@@ -231,6 +262,7 @@ __global__ void __launch_bounds__(1024) qp3_reflector_kernel(const double* __res
     sc->tau = tau;
     sc->scale = scale;
     sc->nflag = 0;
+    sc->done = 0;
     tau_out[j] = tau;
     if (pvt != j) {
       const int64_t tp = perm[j];
@@ -242,66 +274,76 @@ __global__ void __launch_bounds__(1024) qp3_reflector_kernel(const double* __res
   }
   if (pvt != j && threadIdx.x < kk) {  // swap rows j and pvt of F(:, 0:kk)
     const long long t = threadIdx.x;
-    const double a = F[j + t * n];
-    F[j + t * n] = F[pvt + t * n];
-    F[pvt + t * n] = a;
+    const double a = F[j * QP3_NB + t];
+    F[j * QP3_NB + t] = F[pvt * QP3_NB + t];
+    F[pvt * QP3_NB + t] = a;
   }
 }
 
 // ---- step (c): z(c) = A(rk:m, c)^T v, c in [j0, n), v = (1, scale * A(rk+1:m, j)) ------------
+// CTA (x, y): 16 columns x rows [rs + y * rows_per_cta, ...), in sub-chunks of QP3_GV_ROWS whose
+// reflector slice is staged in shared memory; one partial sum per (y, column).
 __global__ void __launch_bounds__(QP3_T) qp3_gemv_kernel(const double* __restrict__ A, long long lda, long long m,
                                                          long long n, long long j, long long j0,
-                                                         const Qp3Scalars* __restrict__ sc, double* parts) {
+                                                         long long rows_per_cta, const Qp3Scalars* __restrict__ sc,
+                                                         double* parts) {
   __shared__ __align__(16) double sv[QP3_GV_ROWS];
   const long long rk = j;
-  const long long rs = (rk & ~1LL) + static_cast<long long>(blockIdx.y) * QP3_GV_ROWS;
-  const long long re = rs + QP3_GV_ROWS < m ? rs + QP3_GV_ROWS : m;
+  const long long rbeg = (rk & ~1LL) + static_cast<long long>(blockIdx.y) * rows_per_cta;
+  const long long rend = rbeg + rows_per_cta < m ? rbeg + rows_per_cta : m;
   const double scale = sc->scale;
   const double* colj = A + j * lda;
-  for (int r = threadIdx.x; r < QP3_GV_ROWS; r += blockDim.x) {
-    const long long i = rs + r;
-    double v = 0.0;
-    if (i < re && i >= rk) v = i == rk ? 1.0 : colj[i] * scale;
-    sv[r] = v;
-  }
-  __syncthreads();
   const int warp = threadIdx.x >> 5, lane = threadIdx.x & 31;
   const long long c0 = j0 + static_cast<long long>(blockIdx.x) * QP3_GV_COLS + warp * QP3_GV_CPW;
-  if (c0 >= n) return;  // no block-level synchronisation below
-  const long long nrow = re - rs;  // >= 0
-  const long long npair = nrow >> 1;
+  const bool active = c0 < n;
   double acc[QP3_GV_CPW];
 #pragma unroll
   for (int q = 0; q < QP3_GV_CPW; ++q) acc[q] = 0.0;
-  const double* cols[QP3_GV_CPW];
+  for (long long rs = rbeg; rs < rend; rs += QP3_GV_ROWS) {
+    const long long re = rs + QP3_GV_ROWS < rend ? rs + QP3_GV_ROWS : rend;
+    __syncthreads();
+    for (int r = threadIdx.x; r < QP3_GV_ROWS; r += blockDim.x) {
+      const long long i = rs + r;
+      double v = 0.0;
+      if (i < re && i >= rk) v = i == rk ? 1.0 : colj[i] * scale;
+      sv[r] = v;
+    }
+    __syncthreads();
+    if (!active) continue;
+    const long long nrow = re - rs;
+    const long long npair = nrow >> 1;
+    const double* cols[QP3_GV_CPW];
 #pragma unroll
-  for (int q = 0; q < QP3_GV_CPW; ++q) cols[q] = A + (c0 + q < n ? c0 + q : c0) * lda + rs;
-  long long p = lane;
-  for (; p + 96 < npair; p += 128) {
-    double2 x[4][QP3_GV_CPW];
+    for (int q = 0; q < QP3_GV_CPW; ++q) cols[q] = A + (c0 + q < n ? c0 + q : c0) * lda + rs;
+    long long p = lane;
+    for (; p + 96 < npair; p += 128) {
+      double2 x[4][QP3_GV_CPW];
 #pragma unroll
-    for (int u = 0; u < 4; ++u)
+      for (int u = 0; u < 4; ++u)
 #pragma unroll
-      for (int q = 0; q < QP3_GV_CPW; ++q) x[u][q] = *reinterpret_cast<const double2*>(cols[q] + 2 * (p + 32 * u));
+        for (int q = 0; q < QP3_GV_CPW; ++q)
+          x[u][q] = *reinterpret_cast<const double2*>(cols[q] + 2 * (p + 32 * u));
 #pragma unroll
-    for (int u = 0; u < 4; ++u) {
-      const double2 v = *reinterpret_cast<const double2*>(sv + 2 * (p + 32 * u));
+      for (int u = 0; u < 4; ++u) {
+        const double2 v = *reinterpret_cast<const double2*>(sv + 2 * (p + 32 * u));
 #pragma unroll
-      for (int q = 0; q < QP3_GV_CPW; ++q) acc[q] = fma(x[u][q].y, v.y, fma(x[u][q].x, v.x, acc[q]));
+        for (int q = 0; q < QP3_GV_CPW; ++q) acc[q] = fma(x[u][q].y, v.y, fma(x[u][q].x, v.x, acc[q]));
+      }
+    }
+    for (; p < npair; p += 32) {
+      const double2 v = *reinterpret_cast<const double2*>(sv + 2 * p);
+#pragma unroll
+      for (int q = 0; q < QP3_GV_CPW; ++q) {
+        const double2 x = *reinterpret_cast<const double2*>(cols[q] + 2 * p);
+        acc[q] = fma(x.y, v.y, fma(x.x, v.x, acc[q]));
+      }
+    }
+    if ((nrow & 1) && lane == 0) {
+#pragma unroll
+      for (int q = 0; q < QP3_GV_CPW; ++q) acc[q] = fma(cols[q][nrow - 1], sv[nrow - 1], acc[q]);
     }
   }
-  for (; p < npair; p += 32) {
-    const double2 v = *reinterpret_cast<const double2*>(sv + 2 * p);
-#pragma unroll
-    for (int q = 0; q < QP3_GV_CPW; ++q) {
-      const double2 x = *reinterpret_cast<const double2*>(cols[q] + 2 * p);
-      acc[q] = fma(x.y, v.y, fma(x.x, v.x, acc[q]));
-    }
-  }
-  if ((nrow & 1) && lane == 0) {
-#pragma unroll
-    for (int q = 0; q < QP3_GV_CPW; ++q) acc[q] = fma(cols[q][nrow - 1], sv[nrow - 1], acc[q]);
-  }
+  if (!active) return;
 #pragma unroll
   for (int q = 0; q < QP3_GV_CPW; ++q) {
     const double s = warp_sum(acc[q]);
@@ -309,30 +351,67 @@ __global__ void __launch_bounds__(QP3_T) qp3_gemv_kernel(const double* __restric
   }
 }
 
-// ---- step (d): F(:, kk); scale the reflector into A(rk+1:m, j), A(rk, j) := beta -------------
-//   F(c, kk) = [c > j] tau z(c) - tau sum_t F(c, t) z(j0 + t)   (c in [j0, n))
-__global__ void __launch_bounds__(QP3_T) qp3_fcol_kernel(double* __restrict__ A, long long lda, long long m,
-                                                         long long n, long long j, long long j0, int kk, int nch,
-                                                         const double* __restrict__ parts, double* F,
-                                                         const Qp3Scalars* __restrict__ sc) {
+// ---- steps (d)+(e), one warp per column c in [j0, n):
+//   F(c, kk) = [c > j] tau z(c) - tau sum_t F(c, t) z(j0 + t)                       (F column kk)
+//   c > j:  A(rk, c) -= sum_{t<kk} A(rk, j0+t) F(c, t) + F(c, kk);  downdate vn1(c)   (row rk)
+// plus the reflector scaled into A(rk+1:m, j) and A(rk, j) := beta.  Lane t holds F(c, t) (one
+// 256-byte row of F); the z partial sums are split over lanes; fixed-tree warp sums.
+__global__ void __launch_bounds__(QP3_T) qp3_fcol_row_kernel(double* __restrict__ A, long long lda, long long m,
+                                                             long long n, long long j, long long j0, int kk, int nch,
+                                                             const double* __restrict__ parts, double* F, double* vn1,
+                                                             double* vn2, int* flags, Qp3Scalars* sc, int downdate) {
+  __shared__ double s_aux8[QP3_NB][8];
   __shared__ double s_aux[QP3_NB];
+  __shared__ double s_r[QP3_NB];
+  const long long rk = j;
   const double tau = sc->tau;
-  if (threadIdx.x < kk) {
+  {  // aux(t) = -tau z(j0 + t), t < kk: thread (t, g) sums partials q = g, g+8, ...
+    const int t = threadIdx.x >> 3, g = threadIdx.x & 7;
     double z = 0.0;
-    for (int q = 0; q < nch; ++q) z += parts[static_cast<long long>(q) * n + j0 + threadIdx.x];
-    s_aux[threadIdx.x] = -tau * z;
+    if (t < kk)
+      for (int q = g; q < nch; q += 8) z += parts[static_cast<long long>(q) * n + j0 + t];
+    s_aux8[t][g] = z;
+    if (threadIdx.x < kk) s_r[threadIdx.x] = A[rk + (j0 + threadIdx.x) * lda];
   }
   __syncthreads();
-  const long long c = j0 + static_cast<long long>(blockIdx.x) * blockDim.x + threadIdx.x;
+  if (threadIdx.x < kk) {
+    const double* z8 = s_aux8[threadIdx.x];
+    s_aux[threadIdx.x] = -tau * (((z8[0] + z8[1]) + (z8[2] + z8[3])) + ((z8[4] + z8[5]) + (z8[6] + z8[7])));
+  }
+  __syncthreads();
+  const int warp = threadIdx.x >> 5, lane = threadIdx.x & 31;
+  const long long c = j0 + static_cast<long long>(blockIdx.x) * (QP3_T / 32) + warp;
   if (c < n) {
-    double f = 0.0;
-    if (c > j) {
-      double z = 0.0;
-      for (int q = 0; q < nch; ++q) z += parts[static_cast<long long>(q) * n + c];
-      f = tau * z;
+    double z = 0.0;
+    if (c > j)
+      for (int q = lane; q < nch; q += 32) z += parts[static_cast<long long>(q) * n + c];
+    const double fct = lane < kk ? F[c * QP3_NB + lane] : 0.0;
+    double fsum = lane < kk ? fct * s_aux[lane] : 0.0;
+    double asum = lane < kk ? s_r[lane] * fct : 0.0;
+    z = warp_sum(z);
+    fsum = warp_sum(fsum);
+    asum = warp_sum(asum);
+    if (lane == 0) {
+      const double f = (c > j ? tau * z : 0.0) + fsum;
+      F[c * QP3_NB + kk] = f;
+      if (c > j) {
+        const double a = A[rk + c * lda] - asum - f;  // v(rk) = 1
+        A[rk + c * lda] = a;
+        const double v1 = vn1[c];
+        if (downdate && v1 != 0.0) {  // LAPACK dlaqps: tol3z = sqrt(eps)
+          double temp = fabs(a) / v1;
+          temp = fmax(0.0, (1.0 + temp) * (1.0 - temp));
+          const double r = v1 / vn2[c];
+          const double temp2 = temp * r * r;
+          if (temp2 <= 1.0536712127723509e-08) {
+            const int slot = atomicAdd(&sc->nflag, 1);
+            flags[slot] = static_cast<int>(c);
+          } else {
+            vn1[c] = v1 * sqrt(temp);
+          }
+        }
+      }
     }
-    for (int t = 0; t < kk; ++t) f = fma(F[c + static_cast<long long>(t) * n], s_aux[t], f);
-    F[c + static_cast<long long>(kk) * n] = f;
   }
   const double scale = sc->scale;
   double* colj = A + j * lda;
@@ -340,37 +419,6 @@ __global__ void __launch_bounds__(QP3_T) qp3_fcol_kernel(double* __restrict__ A,
        i += static_cast<long long>(gridDim.x) * blockDim.x)
     colj[i] *= scale;
   if (blockIdx.x == 0 && threadIdx.x == 0) colj[j] = sc->beta;
-}
-
-// ---- step (e): current row A(rk, j+1:n) -= A(rk, j0:j+1) F(j+1:n, 0:kk+1)^T; norm downdate ---
-__global__ void __launch_bounds__(QP3_T) qp3_row_kernel(double* __restrict__ A, long long lda, long long m,
-                                                        long long n, long long j, long long j0, int kk,
-                                                        const double* __restrict__ F, double* vn1, double* vn2,
-                                                        int* flags, Qp3Scalars* sc, int downdate) {
-  __shared__ double s_r[QP3_NB];
-  const long long rk = j;
-  if (threadIdx.x < kk) s_r[threadIdx.x] = A[rk + (j0 + threadIdx.x) * lda];
-  if (threadIdx.x == kk) s_r[kk] = 1.0;  // v(rk) = 1 (A(rk, j) already holds beta)
-  __syncthreads();
-  const long long c = j + 1 + static_cast<long long>(blockIdx.x) * blockDim.x + threadIdx.x;
-  if (c >= n) return;
-  double a = A[rk + c * lda];
-  for (int t = 0; t <= kk; ++t) a = fma(-s_r[t], F[c + static_cast<long long>(t) * n], a);
-  A[rk + c * lda] = a;
-  if (!downdate) return;
-  const double v1 = vn1[c];
-  if (v1 != 0.0) {  // LAPACK dlaqps: tol3z = sqrt(eps)
-    double temp = fabs(a) / v1;
-    temp = fmax(0.0, (1.0 + temp) * (1.0 - temp));
-    const double r = v1 / vn2[c];
-    const double temp2 = temp * r * r;
-    if (temp2 <= 1.0536712127723509e-08) {
-      const int slot = atomicAdd(&sc->nflag, 1);
-      flags[slot] = static_cast<int>(c);
-    } else {
-      vn1[c] = v1 * sqrt(temp);
-    }
-  }
 }
 
 // ---- step (f): exact norms of flagged columns from the delayed update ------------------------
@@ -384,7 +432,7 @@ __global__ void __launch_bounds__(QP3_T) qp3_recompute_kernel(const double* __re
   for (int f = blockIdx.x; f < nflag; f += gridDim.x) {
     const long long c = flags[f];
     __syncthreads();
-    if (threadIdx.x <= kk) s_f[threadIdx.x] = F[c + static_cast<long long>(threadIdx.x) * n];
+    if (threadIdx.x <= kk) s_f[threadIdx.x] = F[c * QP3_NB + threadIdx.x];
     __syncthreads();
     double ss = 0.0;
     for (long long i = j + 1 + threadIdx.x; i < m; i += blockDim.x) {
@@ -401,26 +449,43 @@ __global__ void __launch_bounds__(QP3_T) qp3_recompute_kernel(const double* __re
 }
 
 // ---- panel end: A(r0:m, c0:n) -= A(r0:m, j0:j0+kb) F(c0:n, 0:kb)^T, fused exact column norms --
-__global__ void __launch_bounds__(QP3_T) qp3_trailing_kernel(double* __restrict__ A, long long lda, long long m,
-                                                             long long n, long long j0, int kb, long long r0,
-                                                             long long c0, const double* __restrict__ F,
-                                                             double* parts) {
+// CTA: 32 columns (4 per warp) x 1024 rows in sub-tiles of 128 (two row pairs per lane).  The thread's
+// 4 x 4 block of A is loaded before the panel slice is staged, so the HBM reads overlap the
+// shared-memory staging; F(tile, :) and the panel slice are broadcast / conflict-free LDS.128.
+__global__ void __launch_bounds__(QP3_T, 2) qp3_trailing_kernel(double* __restrict__ A, long long lda, long long m,
+                                                                long long n, long long j0, int kb, long long r0,
+                                                                long long c0, const double* __restrict__ F,
+                                                                double* parts) {
   __shared__ __align__(16) double Ls[QP3_NB][QP3_UP_ROWS];
   __shared__ __align__(16) double Fs[QP3_NB][QP3_UP_COLS];
   const int warp = threadIdx.x >> 5, lane = threadIdx.x & 31;
   const long long cb = c0 + static_cast<long long>(blockIdx.x) * QP3_UP_COLS;
   for (int e = threadIdx.x; e < QP3_NB * QP3_UP_COLS; e += blockDim.x) {
     const int t = e / QP3_UP_COLS, cc = e % QP3_UP_COLS;
-    Fs[t][cc] = (t < kb && cb + cc < n) ? F[cb + cc + static_cast<long long>(t) * n] : 0.0;
+    Fs[t][cc] = (t < kb && cb + cc < n) ? F[(cb + cc) * QP3_NB + t] : 0.0;
   }
-  const long long cw = cb + warp * 8;  // this warp's 8 columns
-  double ssq[8];
-#pragma unroll
-  for (int q = 0; q < 8; ++q) ssq[q] = 0.0;
+  const long long cw = cb + warp * 4;  // this warp's 4 columns
+  double ssq[4] = {0.0, 0.0, 0.0, 0.0};
   const long long rbase = (r0 & ~1LL) + static_cast<long long>(blockIdx.y) * (QP3_UP_ROWS * QP3_UP_SUB);
   for (int sub = 0; sub < QP3_UP_SUB; ++sub) {
     const long long rs = rbase + sub * QP3_UP_ROWS;
     if (rs >= m) break;
+    // lane rows: pair h = 0, 1 at rs + 64 h + 2 lane (+0, +1): conflict-free LDS.128 of the slice
+    long long ih[2];
+    bool full[2];
+#pragma unroll
+    for (int hh = 0; hh < 2; ++hh) {
+      ih[hh] = rs + 64 * hh + 2 * lane;
+      full[hh] = ih[hh] + 1 < m;
+    }
+    double2 a[4][2];
+#pragma unroll
+    for (int q = 0; q < 4; ++q)
+#pragma unroll
+      for (int hh = 0; hh < 2; ++hh) {
+        a[q][hh] = make_double2(0.0, 0.0);
+        if (full[hh] && cw + q < n) a[q][hh] = *reinterpret_cast<const double2*>(A + (cw + q) * lda + ih[hh]);
+      }
     __syncthreads();
     for (int e = threadIdx.x; e < QP3_NB * (QP3_UP_ROWS / 2); e += blockDim.x) {
       const int t = e / (QP3_UP_ROWS / 2), rp = e % (QP3_UP_ROWS / 2);
@@ -439,61 +504,51 @@ __global__ void __launch_bounds__(QP3_T) qp3_trailing_kernel(double* __restrict_
       *reinterpret_cast<double2*>(&Ls[t][2 * rp]) = x;
     }
     __syncthreads();
-    const long long i0 = rs + 4 * lane;  // rows i0 .. i0+3
-    if (i0 >= m) continue;
-    double acc[8][4];
+    if (ih[0] >= m) continue;
+    double acc[4][4];  // [column][row: pair 0 (.x, .y), pair 1 (.x, .y)]
 #pragma unroll
-    for (int q = 0; q < 8; ++q)
+    for (int q = 0; q < 4; ++q)
 #pragma unroll
       for (int r = 0; r < 4; ++r) acc[q][r] = 0.0;
-#pragma unroll 4
+#pragma unroll 8
     for (int t = 0; t < QP3_NB; ++t) {
       if (t >= kb) break;
-      const double2 l01 = *reinterpret_cast<const double2*>(&Ls[t][4 * lane]);
-      const double2 l23 = *reinterpret_cast<const double2*>(&Ls[t][4 * lane + 2]);
-      const double2 f01 = *reinterpret_cast<const double2*>(&Fs[t][warp * 8]);
-      const double2 f23 = *reinterpret_cast<const double2*>(&Fs[t][warp * 8 + 2]);
-      const double2 f45 = *reinterpret_cast<const double2*>(&Fs[t][warp * 8 + 4]);
-      const double2 f67 = *reinterpret_cast<const double2*>(&Fs[t][warp * 8 + 6]);
+      const double2 l01 = *reinterpret_cast<const double2*>(&Ls[t][2 * lane]);
+      const double2 l23 = *reinterpret_cast<const double2*>(&Ls[t][64 + 2 * lane]);
+      const double2 f01 = *reinterpret_cast<const double2*>(&Fs[t][warp * 4]);
+      const double2 f23 = *reinterpret_cast<const double2*>(&Fs[t][warp * 4 + 2]);
       const double l[4] = {l01.x, l01.y, l23.x, l23.y};
-      const double f[8] = {f01.x, f01.y, f23.x, f23.y, f45.x, f45.y, f67.x, f67.y};
+      const double f[4] = {f01.x, f01.y, f23.x, f23.y};
 #pragma unroll
-      for (int q = 0; q < 8; ++q)
+      for (int q = 0; q < 4; ++q)
 #pragma unroll
         for (int r = 0; r < 4; ++r) acc[q][r] = fma(l[r], f[q], acc[q][r]);
     }
 #pragma unroll
-    for (int q = 0; q < 8; ++q) {
+    for (int q = 0; q < 4; ++q) {
       const long long c = cw + q;
       if (c >= n) continue;
       double* col = A + c * lda;
-      if (i0 + 3 < m) {
-        double2 a01 = *reinterpret_cast<const double2*>(col + i0);
-        double2 a23 = *reinterpret_cast<const double2*>(col + i0 + 2);
-        if (i0 >= r0) a01.x -= acc[q][0];
-        if (i0 + 1 >= r0) a01.y -= acc[q][1];
-        a23.x -= acc[q][2];  // i0 + 2 >= r0 whenever i0 + 1 >= r0 - 1; rows < r0 have acc = 0
-        a23.y -= acc[q][3];
-        *reinterpret_cast<double2*>(col + i0) = a01;
-        *reinterpret_cast<double2*>(col + i0 + 2) = a23;
-        if (i0 >= r0) ssq[q] = fma(a01.x, a01.x, ssq[q]);
-        if (i0 + 1 >= r0) ssq[q] = fma(a01.y, a01.y, ssq[q]);
-        if (i0 + 2 >= r0) ssq[q] = fma(a23.x, a23.x, ssq[q]);
-        if (i0 + 3 >= r0) ssq[q] = fma(a23.y, a23.y, ssq[q]);
-      } else {
-        for (int r = 0; r < 4; ++r) {
-          const long long i = i0 + r;
-          if (i >= m) break;
-          if (i < r0) continue;
-          const double a = col[i] - acc[q][r];
-          col[i] = a;
-          ssq[q] = fma(a, a, ssq[q]);
+#pragma unroll
+      for (int hh = 0; hh < 2; ++hh) {
+        const long long i = ih[hh];
+        if (full[hh]) {  // rows < r0 have acc = 0 (masked slice): the store leaves them unchanged
+          double2 v = a[q][hh];
+          v.x -= acc[q][2 * hh];
+          v.y -= acc[q][2 * hh + 1];
+          *reinterpret_cast<double2*>(col + i) = v;
+          if (i >= r0) ssq[q] = fma(v.x, v.x, ssq[q]);
+          ssq[q] = fma(v.y, v.y, ssq[q]);  // i + 1 >= r0 always (r0 - rbase <= 1)
+        } else if (i < m && i >= r0) {
+          const double v = col[i] - acc[q][2 * hh];
+          col[i] = v;
+          ssq[q] = fma(v, v, ssq[q]);
         }
       }
     }
   }
 #pragma unroll
-  for (int q = 0; q < 8; ++q) {
+  for (int q = 0; q < 4; ++q) {
     const double s = warp_sum(ssq[q]);
     if (lane == 0 && cw + q < n) parts[static_cast<long long>(blockIdx.y) * n + cw + q] = s;
   }
@@ -535,29 +590,24 @@ cudaError_t qp3_truncated_large(cudaStream_t st, double* A, long long lda, long 
     const int kb = static_cast<int>(k - j0 < QP3_NB ? k - j0 : QP3_NB);
     for (int kk = 0; kk < kb; ++kk) {
       const long long j = j0 + kk;
-      qp3_pivot_kernel<<<QP3_A_CTAS, QP3_T, 0, st>>>(A, lda, m, n, j, j0, kk, w.vn1, perm, w.F, w.parts_a, w.sc);
-      QP3_LAUNCHED();
-      qp3_reflector_kernel<<<1, 1024, 0, st>>>(A, lda, n, j, kk, QP3_A_CTAS, w.parts_a, w.vn1, w.vn2, perm, w.F, tau,
-                                               w.sc);
+      qp3_pivot_kernel<<<QP3_A_CTAS, QP3_T, 0, st>>>(A, lda, m, n, j, j0, kk, w.vn1, w.vn2, perm, w.F, w.parts_a,
+                                                     tau, w.sc);
       QP3_LAUNCHED();
       const long long rows = m - (j & ~1LL);
-      const unsigned nchg = static_cast<unsigned>((rows + QP3_GV_ROWS - 1) / QP3_GV_ROWS);
-      const unsigned ncg = static_cast<unsigned>((n - j0 + QP3_GV_COLS - 1) / QP3_GV_COLS);
-      qp3_gemv_kernel<<<dim3(ncg, nchg), QP3_T, 0, st>>>(A, lda, m, n, j, j0, w.sc, w.parts);
+      const long long ncg = (n - j0 + QP3_GV_COLS - 1) / QP3_GV_COLS;
+      const long long rpc = QP3_GV_ROWS;
+      const unsigned nchg = static_cast<unsigned>((rows + rpc - 1) / rpc);
+      qp3_gemv_kernel<<<dim3(static_cast<unsigned>(ncg), nchg), QP3_T, 0, st>>>(A, lda, m, n, j, j0, rpc, w.sc,
+                                                                               w.parts);
       QP3_LAUNCHED();
-      const unsigned nfb = static_cast<unsigned>((n - j0 + QP3_T - 1) / QP3_T);
-      qp3_fcol_kernel<<<nfb < 64 ? 64 : nfb, QP3_T, 0, st>>>(A, lda, m, n, j, j0, kk, static_cast<int>(nchg), w.parts,
-                                                            w.F, w.sc);
+      const unsigned nfb = static_cast<unsigned>((n - j0 + QP3_T / 32 - 1) / (QP3_T / 32));
+      const int downdate = j + 1 < lastrk && j + 1 < k ? 1 : 0;  // norms are not needed after step k
+      qp3_fcol_row_kernel<<<nfb < 64 ? 64 : nfb, QP3_T, 0, st>>>(A, lda, m, n, j, j0, kk, static_cast<int>(nchg),
+                                                                w.parts, w.F, w.vn1, w.vn2, w.flags, w.sc, downdate);
       QP3_LAUNCHED();
-      if (j + 1 < n) {
-        const int downdate = j + 1 < lastrk && j + 1 < k ? 1 : 0;  // norms are not needed after step k
-        qp3_row_kernel<<<static_cast<unsigned>((n - j - 1 + QP3_T - 1) / QP3_T), QP3_T, 0, st>>>(
-            A, lda, m, n, j, j0, kk, w.F, w.vn1, w.vn2, w.flags, w.sc, downdate);
+      if (downdate) {
+        qp3_recompute_kernel<<<148, QP3_T, 0, st>>>(A, lda, m, n, j, j0, kk, w.F, w.vn1, w.vn2, w.flags, w.sc);
         QP3_LAUNCHED();
-        if (downdate) {
-          qp3_recompute_kernel<<<148, QP3_T, 0, st>>>(A, lda, m, n, j, j0, kk, w.F, w.vn1, w.vn2, w.flags, w.sc);
-          QP3_LAUNCHED();
-        }
       }
     }
     const long long r0 = j0 + kb, c0 = j0 + kb;

@@ -19,12 +19,15 @@ def main():
     ap.add_argument("--cfg", default="cfg2")
     ap.add_argument("--reps", type=int, default=3)
     ap.add_argument("--m", type=int, default=0)
+    ap.add_argument("--n", type=int, default=0)
     ap.add_argument("--k", type=int, default=0)
     ap.add_argument("--q", type=int, default=-1)
     args = ap.parse_args()
     c = dict(CONFIGS[args.cfg])
     if args.m:
         c["m"] = args.m
+    if args.n:
+        c["n"] = args.n
     if args.k:
         c["k"] = args.k
     if args.q >= 0:
