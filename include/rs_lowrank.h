@@ -109,17 +109,23 @@ RS_API rs_status_t rs_lowrank_run_host(rs_lowrank_t h, const double* A_host, int
                                 int64_t ldr, double* Q_dev, int64_t ld_qdev, double* R_dev, int64_t ld_rdev);
 
 /* Adaptive sample size for the fixed-accuracy problem (Fig. 3; Sec. 10):
- * grows l by l_inc (a multiple of 8) per round -- new rows of the same Omega (Philox rows
- * [l, l+l_inc)), q power iterations of the new block with block Gram-Schmidt (BCGS2) against
- * the previous blocks (Fig. 2(a) lines 4/9), BOrth + CholQR2 of the block -- until the estimate
- * eps~ = max_i ||b_i - b_i B^T B|| of the next block's rows is <= eps (bound (4)).
- * The handle must be created with k = l_max and p = 0.  On return B holds l orthonormal rows and
- * pivot/factor run with k = l.  history (host, may be NULL) receives up to history_len pairs
- * (l, eps~).  Returns RS_ERR_NOT_CONVERGED (B still valid, *ell_out = l_max) if l_max is reached.
- * Synchronises once per round (eps~ is read on the host).                                      */
+ * grows l block by block -- new rows of the same Omega (Philox rows [l, l + l_inc)), q power
+ * iterations of the new block, each BOrth + QR being block classical Gram-Schmidt in its two-pass
+ * form (project against the previous blocks, CholQR; project, CholQR again: DESIGN.md R17) --
+ * until the estimate eps~ = max_i ||b_i - b_i B^T B|| of the next block's rows is <= eps (bound
+ * (4)).  l_inc (a multiple of 8) is the first block size; inc_policy chooses
+ * f(l, l_inc) of line 11: RS_INC_STATIC keeps it (Figs. 16-18), RS_INC_INTERP extrapolates
+ * log10 eps~ linearly from the previous two estimates (Fig. 17 "adapt. linc"),
+ * rounded up to a multiple of 8.  The handle must be created with k = l_max and p = 0.  On
+ * return B holds l orthonormal rows and pivot/factor run with k = l.  history (host, may be NULL)
+ * receives up to history_len pairs (l, eps~).  Returns RS_ERR_NOT_CONVERGED (B still valid,
+ * *ell_out = l reached) when the next block would not fit in l_max.  Synchronises once per round
+ * (eps~ and the next increment are decided on the host).                                      */
+#define RS_INC_STATIC 0
+#define RS_INC_INTERP 1
 RS_API rs_status_t rs_lowrank_sample_adaptive(rs_lowrank_t h, const double* A, int64_t lda, double eps,
-                                              int32_t ell_inc, int32_t q, int32_t* ell_out, double* est_out,
-                                              double* history, int32_t history_len);
+                                              int32_t ell_inc, int32_t q, int32_t inc_policy, int32_t* ell_out,
+                                              double* est_out, double* history, int32_t history_len);
 
 RS_API rs_status_t rs_lowrank_destroy(rs_lowrank_t h);
 

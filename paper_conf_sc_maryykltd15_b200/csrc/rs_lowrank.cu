@@ -5,6 +5,7 @@
 
 #include <algorithm>
 #include <cstdarg>
+#include <cmath>
 #include <cstdio>
 #include <cstring>
 #include <map>
@@ -259,15 +260,17 @@ rs_status_t cholqr_small_pass(rs_lowrank_t h, const double* src, int rr, int rp,
   return RS_OK;
 }
 
-// CholQR2 of X into Y (shifted = false), or shifted CholQR3 (one shifted pass, then CholQR2).
-rs_status_t cholqr2_block(rs_lowrank_t h, const double* X, int rr, int rp, double* Y, bool shifted = false) {
+// CholQR of X into Y with nshift shifted passes followed by two plain ones: CholQR2 (nshift = 0),
+// shifted CholQR3 (nshift = 1), ...  Each shifted pass is breakdown-free and cuts kappa by about
+// 1 / sqrt(11 n rr u), so the plain passes see kappa^2 u < 1 (R20).
+rs_status_t cholqr2_block(rs_lowrank_t h, const double* X, int rr, int rp, double* Y, int nshift = 0) {
   const double* src = X;
-  const int npass = shifted ? 3 : 2;
+  const int npass = nshift + 2;
   for (int pass = 0; pass < npass; ++pass) {
-    // X -> B1 (-> Rho) -> Y: Y may alias X; Rho (k x n) is free outside pivot and holds rp x n
-    // whenever shifted passes are used (adaptive runs, p = 0)
-    double* dst = pass + 1 < npass ? (pass == 0 ? h->B1 : h->Rho) : Y;
-    rs_status_t s = cholqr_small_pass(h, src, rr, rp, dst, shifted && pass == 0);
+    // X -> B1 (-> Rho -> B1 ...) -> Y: Y may alias X; Rho (k x n) is free outside pivot and holds
+    // rp x n whenever shifted passes are used (adaptive runs, p = 0)
+    double* dst = pass + 1 < npass ? (pass % 2 == 0 ? h->B1 : h->Rho) : Y;
+    rs_status_t s = cholqr_small_pass(h, src, rr, rp, dst, pass < nshift);
     if (s != RS_OK) return s;
     src = dst;
   }
@@ -721,25 +724,26 @@ rs_status_t borth_dist(rs_lowrank_t h, const double* Cold, int lold, double* Cn,
 }
 
 // BOrth + QR of a replicated block (R17): twice { project against B_{1:l}; block CholQR }.  The
-// first CholQR is the shifted CholQR3 (the projected block may be ill-conditioned), the second
+// first CholQR has nshift shifted passes (the projected block may be ill-conditioned), the second
 // acts on a block that is orthonormal to O(kappa u), where CholQR2 is exact to O(u).
-rs_status_t borth_qr_small(rs_lowrank_t h, int lold, double* Bn, int rr) {
+rs_status_t borth_qr_small(rs_lowrank_t h, int lold, double* Bn, int rr, int nshift) {
   rs_status_t s;
-  if (lold <= 0) return cholqr2_block(h, Bn, rr, rr, Bn, true);
+  if (lold <= 0) return cholqr2_block(h, Bn, rr, rr, Bn, nshift);
   for (int pass = 0; pass < 2; ++pass) {
     if ((s = borth_small(h, h->B, h->L.lp, lold, Bn, rr)) != RS_OK) return s;
-    if ((s = cholqr2_block(h, Bn, rr, rr, Bn, pass == 0)) != RS_OK) return s;
+    if ((s = cholqr2_block(h, Bn, rr, rr, Bn, pass == 0 ? nshift : 0)) != RS_OK) return s;
   }
   return RS_OK;
 }
 
-// BOrth + QR of a distributed C block (R17), as borth_qr_small.
-rs_status_t borth_qr_dist(rs_lowrank_t h, int lold, double* Cn, int rr) {
+// BOrth + QR of a distributed C block (R17), as borth_qr_small (pass counts rounded up to even).
+rs_status_t borth_qr_dist(rs_lowrank_t h, int lold, double* Cn, int rr, int nshift) {
   rs_status_t s;
-  if (lold <= 0) return cholqr_dist(h, Cn, rr, rr, 4, 1);
+  const int npass = (nshift + 3) / 2 * 2;
+  if (lold <= 0) return cholqr_dist(h, Cn, rr, rr, npass, nshift);
   for (int pass = 0; pass < 2; ++pass) {
     if ((s = borth_dist(h, h->C, lold, Cn, rr)) != RS_OK) return s;
-    if ((s = cholqr_dist(h, Cn, rr, rr, pass == 0 ? 4 : 2, pass == 0 ? 1 : 0)) != RS_OK) return s;
+    if ((s = cholqr_dist(h, Cn, rr, rr, pass == 0 ? npass : 2, pass == 0 ? nshift : 0)) != RS_OK) return s;
   }
   return RS_OK;
 }
@@ -768,14 +772,15 @@ rs_status_t sample_block(rs_lowrank_t h, const double* A, long long lda, int row
 }
 
 // POWER (Fig. 2(a)) on the new block (rows [l, l+rr)) with BOrth against rows [0, l)
-rs_status_t power_block(rs_lowrank_t h, const double* A, long long lda, int l, int rr, int q, double* Bn) {
+rs_status_t power_block(rs_lowrank_t h, const double* A, long long lda, int l, int rr, int q, double* Bn,
+                        int nshift) {
   const Layout& L = h->L;
   const long long ml = h->m_local, n = h->n;
   const long long cnt = static_cast<long long>(rr) * n;
   double* Cn = h->C + static_cast<long long>(l) * L.ldc;
   rs_status_t s;
   for (int it = 0; it < q; ++it) {
-    if ((s = borth_qr_small(h, l, Bn, rr)) != RS_OK) return s;                  // lines 4-5
+    if ((s = borth_qr_small(h, l, Bn, rr, nshift)) != RS_OK) return s;          // lines 4-5
     if (ml > 0) {                                                               // line 7: C := B A^T
       Scope sc(h, "gemm_power_c", 2.0 * rr * static_cast<double>(ml) * n);
       View2D Bv{Bn, rr, n, rr};
@@ -783,7 +788,7 @@ rs_status_t power_block(rs_lowrank_t h, const double* A, long long lda, int l, i
       GemmOutDesc out{Cn, L.ldc, 1, 0, rr, static_cast<int>(ml)};
       RS_CUDA(h, gemm_mc(h->st, rr, static_cast<int>(ml), n, Bv, Av, out, 1));
     }
-    if ((s = borth_qr_dist(h, l, Cn, rr)) != RS_OK) return s;                   // lines 9-10
+    if ((s = borth_qr_dist(h, l, Cn, rr, nshift)) != RS_OK) return s;           // lines 9-10
     // line 12: B := C A
     if (ml > 0) {
       const int splits = gemm_choose_splits(rr, static_cast<int>(n), ml, max_splits_for(h, cnt), h->sms);
@@ -806,26 +811,44 @@ rs_status_t power_block(rs_lowrank_t h, const double* A, long long lda, int l, i
   return RS_OK;
 }
 
+// f(l, l_inc) of Fig. 3 line 11 (readings R19 / R19b): static, or the "simple linear
+// interpolation of the previous two steps": extrapolate log10 eps~ linearly in l to
+// where it reaches eps and round the increment up to a multiple of 8 (at least 8).
+int next_inc(int policy, const std::vector<std::pair<int, double>>& hv, int l, int inc, double eps) {
+  if (policy == RS_INC_STATIC || hv.size() < 2 || !(eps > 0.0)) return inc;
+  const double l1 = hv[hv.size() - 2].first, e1 = hv[hv.size() - 2].second;
+  const double l2 = hv.back().first, e2 = hv.back().second;
+  if (!(e1 > 0.0 && e2 > 0.0 && e2 < e1)) return inc;
+  const double slope = (std::log10(e2) - std::log10(e1)) / (l2 - l1);
+  const double lstar = l2 + (std::log10(eps) - std::log10(e2)) / slope;
+  const double steps = std::ceil((lstar - l) / 8.0);
+  if (!(steps < 1e6)) return inc;
+  return std::max(8, 8 * static_cast<int>(steps));
+}
+
 }  // namespace
 
 extern "C" {
 
 rs_status_t rs_lowrank_sample_adaptive(rs_lowrank_t h, const double* A, int64_t lda, double eps, int32_t ell_inc,
-                                       int32_t q, int32_t* ell_out, double* est_out, double* history,
-                                       int32_t history_len) {
+                                       int32_t q, int32_t inc_policy, int32_t* ell_out, double* est_out,
+                                       double* history, int32_t history_len) {
   if (!h) return RS_ERR_INVALID_ARG;
   const Layout& L = h->L;
   if (h->p != 0) return fail(h, RS_ERR_INVALID_ARG, "adaptive sampling needs a handle created with p = 0 (k = l_max)");
   if (ell_inc < 8 || ell_inc % 8 != 0 || ell_inc > L.ell || q < 0 || !(eps >= 0.0))
     return fail(h, RS_ERR_INVALID_ARG, "need l_inc a positive multiple of 8, l_inc <= l_max, q >= 0, eps >= 0");
+  if (inc_policy != RS_INC_STATIC && inc_policy != RS_INC_INTERP)
+    return fail(h, RS_ERR_INVALID_ARG, "unknown l_inc policy %d", inc_policy);
   if (h->m_local > 0) {
     rs_status_t s = check_matrix(h, A, lda, h->m_local, "A");
     if (s != RS_OK) return s;
   }
   RS_CUDA(h, cudaMemsetAsync(h->info, 0, 16, h->st));
   RS_CUDA(h, cudaMemsetAsync(h->B, 0, static_cast<size_t>(L.lp) * h->n * 8, h->st));
-  const int rr = ell_inc;
+  int rr = ell_inc;
   const long long n = h->n;
+  std::vector<std::pair<int, double>> hv;  // (l, eps~) for f(l, l_inc)
   double* Bn = h->Bt;           // new block, rr x n, ld rr
   double* E = h->Rho;           // error block rr x n (Rho is free until pivot)
   double* dscal = h->gaps;      // device scalar for eps~
@@ -834,12 +857,33 @@ rs_status_t rs_lowrank_sample_adaptive(rs_lowrank_t h, const double* A, int64_t 
   int l = 0, hist = 0;
   double est = -1.0;
   bool converged = false;
+  h->robust_iters = 0;
   for (;;) {
-    if ((s = power_block(h, A, lda, l, rr, q, Bn)) != RS_OK) return s;      // line 7
-    if ((s = borth_qr_small(h, l, Bn, rr)) != RS_OK) return s;                // line 8 (R17)
+    // lines 7-8 (R17) with one shifted CholQR pass; if a block CholQR still breaks down (a block
+    // reaching far past the numerical rank, kappa ~ 1/u), redo the round from the saved sample
+    // with three shifted passes (R20)
+    RS_CUDA(h, copy_2d(h->st, Bn, rr, h->Rhat, rr, rr, n));
+    for (int attempt = 0;; ++attempt) {
+      const int nshift = attempt == 0 ? 1 : 3;
+      if ((s = power_block(h, A, lda, l, rr, q, Bn, nshift)) != RS_OK) return s;   // line 7
+      if ((s = borth_qr_small(h, l, Bn, rr, nshift)) != RS_OK) return s;          // line 8
+      int info[2] = {0, 0};
+      RS_CUDA(h, cudaMemcpyAsync(info, h->info, sizeof(info), cudaMemcpyDeviceToHost, h->st));
+      RS_CUDA(h, cudaStreamSynchronize(h->st));
+      if (info[0] != RS_ERR_NOT_SPD || attempt == 1) break;
+      RS_CUDA(h, cudaMemsetAsync(h->info, 0, 16, h->st));
+      RS_CUDA(h, copy_2d(h->st, h->Rhat, rr, Bn, rr, rr, n));
+      h->robust_iters++;
+    }
     RS_CUDA(h, copy_2d(h->st, Bn, rr, h->B + l, L.lp, rr, n));
     l += rr;                                                                  // line 9
-    if (l + rr > L.ell) break;
+    int inc = next_inc(inc_policy, hv, l, rr, eps);                          // line 11
+    if (l + inc > L.ell) {
+      if (inc_policy == RS_INC_STATIC) break;
+      inc = (L.ell - l) / 8 * 8;
+      if (inc < 8) break;
+    }
+    rr = inc;
     if ((s = sample_block(h, A, lda, l, rr, Bn)) != RS_OK) return s;          // lines 12-13
     // line 15: eps~ = max_i || b_i - b_i B_{1:l}^T B_{1:l} ||  (R18)
     RS_CUDA(h, copy_2d(h->st, Bn, rr, E, rr, rr, n));
@@ -863,6 +907,7 @@ rs_status_t rs_lowrank_sample_adaptive(rs_lowrank_t h, const double* A, int64_t 
       history[2 * hist + 1] = est;
     }
     ++hist;
+    hv.emplace_back(l, est);
     if (est <= eps) {                                                         // line 16
       converged = true;
       break;

@@ -64,7 +64,7 @@ def load_library(path: str = LIB_PATH):
         "rs_lowrank_pivot": (ctypes.c_int, [P, P]),
         "rs_lowrank_factor": (ctypes.c_int, [P, P, I64, P, I64, P, I64]),
         "rs_lowrank_run_host": (ctypes.c_int, [P, P, I64, P, I64, I32, P, P, I64, P, I64, P, I64, P, I64]),
-        "rs_lowrank_sample_adaptive": (ctypes.c_int, [P, P, I64, ctypes.c_double, I32, I32, ctypes.POINTER(I32),
+        "rs_lowrank_sample_adaptive": (ctypes.c_int, [P, P, I64, ctypes.c_double, I32, I32, I32, ctypes.POINTER(I32),
                                                       D, D, I32]),
         "rs_lowrank_destroy": (ctypes.c_int, [P]),
         "rs_lowrank_get_sample": (ctypes.c_int, [P, P, I64]),
@@ -205,14 +205,19 @@ def run_host(h: Handle, A_host: torch.Tensor, A_dev: torch.Tensor, q: int, perm_
         colmajor_ld(R_dev, "R_dev")), h.ptr)
 
 
-def sample_adaptive(h: Handle, A: torch.Tensor, eps: float, ell_inc: int, q: int = 0, *, raise_on_max=True):
+INC_POLICIES = {"static": 0, "interp": 1}
+
+
+def sample_adaptive(h: Handle, A: torch.Tensor, eps: float, ell_inc: int, q: int = 0, *, inc_policy="static",
+                    raise_on_max=True):
     """Fig. 3 adaptive sampling; returns (l, eps~, [(l, eps~) per round]).  The handle must have
-    been created with k = l_max and p = 0."""
+    been created with k = l_max and p = 0.  inc_policy: "static" or "interp"."""
     ell = ctypes.c_int32()
     est = ctypes.c_double()
     hist = (ctypes.c_double * 2048)()
     code = load_library().rs_lowrank_sample_adaptive(h.ptr, A.data_ptr(), colmajor_ld(A, "A"), eps, ell_inc, q,
-                                                     ctypes.byref(ell), ctypes.byref(est), hist, 1024)
+                                                     INC_POLICIES[inc_policy], ctypes.byref(ell),
+                                                     ctypes.byref(est), hist, 1024)
     rounds = []
     for r in range(1024):
         if hist[2 * r] == 0:

@@ -28,18 +28,20 @@ def main():
     ap.add_argument("--q", type=int, default=0)
     ap.add_argument("--lmax", type=int, default=400)
     ap.add_argument("--incs", default="8,16,32,64")
+    ap.add_argument("--policies", default="static,interp")
     args = ap.parse_args()
     A, sigma = make_matrix_torch(args.m, args.n, "exp-paper", 50, seed=2015, device="cuda")
-    for inc in [int(x) for x in args.incs.split(",")]:
+    runs = [(pol, int(x)) for pol in args.policies.split(",") for x in args.incs.split(",")]
+    for pol, inc in runs:
         h = rs.create(args.m, args.m, 0, args.n, args.lmax, 0, 0x5C15)
-        rs.sample_adaptive(h, A, args.eps, inc, args.q, raise_on_max=False)  # warm-up
+        rs.sample_adaptive(h, A, args.eps, inc, args.q, inc_policy=pol, raise_on_max=False)  # warm-up
         torch.cuda.synchronize()
         rs.reset_profile(h)
         rs.set_profiling(h, True)
         s = torch.cuda.current_stream()
         e0, e1, e2 = (torch.cuda.Event(enable_timing=True) for _ in range(3))
         e0.record(s)
-        ell, est, hist = rs.sample_adaptive(h, A, args.eps, inc, args.q, raise_on_max=False)
+        ell, est, hist = rs.sample_adaptive(h, A, args.eps, inc, args.q, inc_policy=pol, raise_on_max=False)
         e1.record(s)
         perm = torch.empty(args.n, dtype=torch.int64, device="cuda")
         Q = rs.empty_colmajor(args.m, args.lmax)
@@ -60,7 +62,7 @@ def main():
         gm = prof["gemm_sample"]
         line = {
             "experiment": "adaptive fixed-accuracy (Fig. 3 / Figs. 16-18)",
-            "m": args.m, "n": args.n, "eps": args.eps, "q": args.q, "l_inc": inc, "l": ell, "eps_est": est,
+            "m": args.m, "n": args.n, "eps": args.eps, "q": args.q, "inc_policy": pol, "l_inc": inc, "l": ell, "eps_est": est,
             "history": hist,
             "sample_ms": e0.elapsed_time(e1), "total_ms": e0.elapsed_time(e2), "factor_status": factor_status,
             "factor_rel_err_F": fac_err, "q_orth": q_orth,

@@ -102,3 +102,30 @@ def test_fig16_exponent_matrix_reaches_1e12_near_l_120_160():
     assert 112 <= res.ell <= 176
     ests = [e for _, e in res.history]
     assert ests[-1] <= 1e-12 and ests[0] > 1e-2
+
+
+def test_interp_increment_rule():
+    """R19b on a closed form: log10 eps~ linear in l (slope -0.1 per vector, as sigma_i = 10^(-i/10))
+    predicts l* exactly; the increment is rounded up to a multiple of 8."""
+    hist = [(8, 1e-1), (16, 10 ** -1.8)]          # slope -0.1 / vector
+    # eps = 1e-6 -> l* = 16 + (-6 + 1.8) / -0.1 = 58; at l = 24: need 34 -> 40
+    assert AD.next_inc("interp", hist, 24, 8, 1e-6) == 40
+    assert AD.next_inc("interp", hist, 24, 8, 10 ** -2.0) == 8      # l* = 18 < l: minimum 8
+    assert AD.next_inc("interp", hist[:1], 24, 16, 1e-6) == 16      # one estimate: unchanged
+    assert AD.next_inc("interp", [(8, 1e-3), (16, 1e-2)], 24, 16, 1e-6) == 16  # no decrease
+    assert AD.next_inc("interp", hist, 24, 8, 0.0) == 8             # eps = 0: unchanged
+    assert AD.next_inc("static", hist, 24, 8, 1e-6) == 8
+
+
+def test_interp_policy_reaches_tolerance_in_fewer_rounds():
+    """Fig. 17 "adapt. linc": on the exponent matrix the interpolated increment needs fewer rounds
+    than the static l_inc = 8 and still meets eps (bound (4) holds for the final basis)."""
+    A, s = make_matrix(1000, 400, "exp-paper", 50, seed=12)
+    r_s = AD.adaptive_sample(A, 1e-10, 8, 0, 5, 400)
+    r_i = AD.adaptive_sample(A, 1e-10, 8, 0, 5, 400, inc_policy="interp")
+    assert r_s.converged and r_i.converged
+    assert len(r_i.history) < len(r_s.history)
+    assert r_i.history[-1][1] <= 1e-10
+    err = np.linalg.norm(A - (A @ r_i.B.T) @ r_i.B, 2)
+    assert err <= 10 * math.sqrt(2 / math.pi) * r_i.history[-1][1]
+    np.testing.assert_allclose(r_i.B @ r_i.B.T, np.eye(r_i.ell), atol=1e-13)
