@@ -127,6 +127,13 @@ RS_API rs_status_t rs_lowrank_sample_adaptive(rs_lowrank_t h, const double* A, i
                                               int32_t ell_inc, int32_t q, int32_t inc_policy, int32_t* ell_out,
                                               double* est_out, double* history, int32_t history_len);
 
+/* Column sampling (Fig. 8(b)): B_c := Omega_c A^T, l x m_local, where Omega_c is the
+ * l x n Gaussian of DESIGN.md §3 keyed by the COLUMN index of A with Philox tag 1 (independent of
+ * the row-sampling Omega).  B_c (device, column-major, ldb >= l even) receives the columns of B_c
+ * that belong to this rank's rows of A -- no communication.  Enqueues only; independent of the
+ * sample/pivot/factor state (uses handle scratch only).                                        */
+RS_API rs_status_t rs_lowrank_sample_columns(rs_lowrank_t h, const double* A, int64_t lda, double* Bc, int64_t ldb);
+
 RS_API rs_status_t rs_lowrank_destroy(rs_lowrank_t h);
 
 /* ---- accessors (tests / bench) ---- */

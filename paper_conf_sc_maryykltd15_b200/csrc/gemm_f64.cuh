@@ -70,7 +70,10 @@ struct KCSmem {
   static constexpr int L_BYTES_TMA = MT * KT * 8;
   static constexpr int L_BYTES_RAW = PHILOX ? MT * PHX_LD * 8 : L_BYTES_TMA;
   static constexpr int L_BYTES = (L_BYTES_RAW + 1023) / 1024 * 1024;
-  static constexpr int TOTAL = 1024 + NSTAGE * (R_BYTES + L_BYTES) + 2 * NSTAGE * 8;
+  // small M (l <= 32): little MMA work per stage, so a deeper ring keeps more of A in flight and
+  // lets several generator groups work on different stages at once
+  static constexpr int NS = MFW <= 2 ? 8 : NSTAGE;
+  static constexpr int TOTAL = 1024 + NS * (R_BYTES + L_BYTES) + 2 * NS * 8;
 };
 
 template <int MFW>
@@ -149,9 +152,9 @@ __global__ void __launch_bounds__(GEMM_THREADS, 1)
   extern __shared__ unsigned char smem_raw[];
   unsigned char* smem = align1024(smem_raw);
   unsigned char* sR = smem;
-  unsigned char* sL = sR + NSTAGE * SM::R_BYTES;
-  uint64_t* full = reinterpret_cast<uint64_t*>(sL + NSTAGE * SM::L_BYTES);
-  uint64_t* empty = full + NSTAGE;
+  unsigned char* sL = sR + SM::NS * SM::R_BYTES;
+  uint64_t* full = reinterpret_cast<uint64_t*>(sL + SM::NS * SM::L_BYTES);
+  uint64_t* empty = full + SM::NS;
 
   const int warp = threadIdx.x >> 5, lane = threadIdx.x & 31;
   const int n0 = blockIdx.x * NT, m0 = blockIdx.y * MT;
@@ -161,7 +164,7 @@ __global__ void __launch_bounds__(GEMM_THREADS, 1)
 
   if (threadIdx.x == 0) {
 #pragma unroll
-    for (int s = 0; s < NSTAGE; ++s) {
+    for (int s = 0; s < SM::NS; ++s) {
       mbar_init(&full[s], 1);
       mbar_init(&empty[s], NCONS);
     }
@@ -170,8 +173,8 @@ __global__ void __launch_bounds__(GEMM_THREADS, 1)
   __syncthreads();
 
   auto issue = [&](int it) {  // one thread: fill stage `it`
-    const int s = it % NSTAGE;
-    if (it >= NSTAGE) mbar_wait(&empty[s], ((it / NSTAGE) - 1) & 1);
+    const int s = it % SM::NS;
+    if (it >= SM::NS) mbar_wait(&empty[s], ((it / SM::NS) - 1) & 1);
     mbar_arrive_expect_tx(&full[s], SM::R_BYTES + SM::L_BYTES_TMA);
     const int kc = static_cast<int>(kb + static_cast<long long>(it) * KT);
     tma_load_2d(sR + s * SM::R_BYTES, &tmR, &full[s], kc, n0);
@@ -180,7 +183,7 @@ __global__ void __launch_bounds__(GEMM_THREADS, 1)
   if (threadIdx.x == 0) {
     tma_prefetch_desc(&tmR);
     tma_prefetch_desc(&tmL);
-    for (int it = 0; it < NSTAGE - 1 && it < nk; ++it) issue(it);
+    for (int it = 0; it < SM::NS - 1 && it < nk; ++it) issue(it);
   }
 
   const int wm = warp >> 2, wn = warp & 3;
@@ -200,9 +203,9 @@ __global__ void __launch_bounds__(GEMM_THREADS, 1)
   };
 
   for (int it = 0; it < nk; ++it) {
-    const int s = it % NSTAGE;
-    if (threadIdx.x == 0 && it + NSTAGE - 1 < nk) issue(it + NSTAGE - 1);
-    mbar_wait(&full[s], (it / NSTAGE) & 1);
+    const int s = it % SM::NS;
+    if (threadIdx.x == 0 && it + SM::NS - 1 < nk) issue(it + SM::NS - 1);
+    mbar_wait(&full[s], (it / SM::NS) & 1);
     const unsigned char* Ls = sL + s * SM::L_BYTES;
     const unsigned char* Rs = sR + s * SM::R_BYTES;
     kc_stage_mma<MFW>(
@@ -236,12 +239,19 @@ __global__ void __launch_bounds__(PHX_THREADS, 1)
   using SM = KCSmem<MFW, true>;
   constexpr int MT = SM::MT;
   constexpr int ROWS = MT / CS;
+  // Generator groups: a stage needs ROWS*4 Philox blocks, i.e. ceil(ROWS*4/32) warps; the spare
+  // warps form further groups that generate other stages concurrently (group g takes stages
+  // it = g mod NGRP), since one stage's generation is a latency-bound dependent chain.
+  constexpr int GEN_WARPS_NEEDED = (ROWS * 4 + 31) / 32;
+  constexpr int NGRP_RAW = PHX_GEN_WARPS / GEN_WARPS_NEEDED;
+  constexpr int NGRP = NGRP_RAW < 1 ? 1 : (NGRP_RAW > SM::NS ? SM::NS : NGRP_RAW);
+  constexpr int GRP_WARPS = PHX_GEN_WARPS / NGRP;
   extern __shared__ unsigned char smem_raw[];
   unsigned char* smem = align1024(smem_raw);
   unsigned char* sR = smem;
-  unsigned char* sL = sR + NSTAGE * SM::R_BYTES;
-  uint64_t* full = reinterpret_cast<uint64_t*>(sL + NSTAGE * SM::L_BYTES);
-  uint64_t* empty = full + NSTAGE;
+  unsigned char* sL = sR + SM::NS * SM::R_BYTES;
+  uint64_t* full = reinterpret_cast<uint64_t*>(sL + SM::NS * SM::L_BYTES);
+  uint64_t* empty = full + SM::NS;
 
   const int warp = threadIdx.x >> 5, lane = threadIdx.x & 31;
   const int n0 = blockIdx.x * NT, m0 = blockIdx.y * MT;
@@ -252,8 +262,8 @@ __global__ void __launch_bounds__(PHX_THREADS, 1)
 
   if (threadIdx.x == 0) {
 #pragma unroll
-    for (int s = 0; s < NSTAGE; ++s) {
-      mbar_init(&full[s], 1 + PHX_GEN_WARPS);  // TMA producer + local generator warps (+ peers' tx bytes)
+    for (int s = 0; s < SM::NS; ++s) {
+      mbar_init(&full[s], 1 + GRP_WARPS);  // TMA producer + the stage's generator warps (+ peers' tx bytes)
       mbar_init(&empty[s], NCONS * CS);
     }
     fence_mbar_init();
@@ -268,14 +278,15 @@ __global__ void __launch_bounds__(PHX_THREADS, 1)
     asm volatile("setmaxnreg.dec.sync.aligned.u32 %0;\n" ::"n"(PHX_GEN_REGS));
     // work item w = (row, q): Omega[row, 4q .. 4q+3] of the stage (one Philox block when the
     // row offset is a multiple of 4); items are spread over all 128 generator threads.
-    const int g = threadIdx.x;
+    const int grp = warp / GRP_WARPS;
+    const int g = threadIdx.x - grp * GRP_WARPS * 32;  // thread index inside the group
     const int o = static_cast<int>(a.row_offset & 3);  // uniform
     constexpr int ITEMS = ROWS * 4;
-    if (g == 0) tma_prefetch_desc(&tmR);
-    for (int it = 0; it < nk; ++it) {
-      const int s = it % NSTAGE;
-      if (it >= NSTAGE) {
-        if (lane == 0) mbar_wait(&empty[s], ((it / NSTAGE) - 1) & 1);
+    if (threadIdx.x == 0) tma_prefetch_desc(&tmR);
+    for (int it = grp; it < nk; it += NGRP) {
+      const int s = it % SM::NS;
+      if (it >= SM::NS) {
+        if (lane == 0) mbar_wait(&empty[s], ((it / SM::NS) - 1) & 1);
         __syncwarp();
       }
       if (g == 0) {
@@ -285,7 +296,7 @@ __global__ void __launch_bounds__(PHX_THREADS, 1)
       const long long j0 = a.row_offset + kb + static_cast<long long>(it) * KT;  // global row of A
       const uint64_t t0 = static_cast<uint64_t>(j0 >> 2);
 #pragma unroll 1
-      for (int w = g; w < ITEMS; w += PHX_GEN_WARPS * 32) {
+      for (int w = g; w < ITEMS; w += GRP_WARPS * 32) {
         const int lrow = static_cast<int>(crank) * ROWS + (w >> 2);
         const int q = w & 3;
         const int gi = m0 + lrow;
@@ -348,10 +359,10 @@ __global__ void __launch_bounds__(PHX_THREADS, 1)
       return kc_row(ng >> 1, ng & 1, r);
     };
     for (int it = 0; it < nk; ++it) {
-      const int s = it % NSTAGE;
+      const int s = it % SM::NS;
       // CTA-scope wait: the slot's data is in this CTA's shared memory (no L1 to invalidate);
       // the remote generators' stores are ordered before their release.cluster arrive
-      mbar_wait(&full[s], (it / NSTAGE) & 1);
+      mbar_wait(&full[s], (it / SM::NS) & 1);
       const double* Ls = reinterpret_cast<const double*>(sL + s * SM::L_BYTES);
       const unsigned char* Rs = sR + s * SM::R_BYTES;
       kc_stage_mma<MFW>(

@@ -995,6 +995,34 @@ rs_status_t rs_lowrank_omega(rs_lowrank_t h, int64_t j0, int64_t ncols, double* 
   return RS_OK;
 }
 
+// Column sampling B_c = Omega_c A^T (Fig. 8(b)).  Omega_c (l x n, keyed by the column
+// index of A, Philox tag 1) is small -- n << m -- so it is materialised once into B1 and the
+// product runs on the MC GEMM family (L = Omega_c M-contiguous, R = A with N = rows contiguous);
+// every rank produces the columns of B_c that belong to its own rows of A (no communication).
+rs_status_t rs_lowrank_sample_columns(rs_lowrank_t h, const double* A, int64_t lda, double* Bc, int64_t ldb) {
+  if (!h) return RS_ERR_INVALID_ARG;
+  const Layout& L = h->L;
+  const long long ml = h->m_local, n = h->n;
+  if (ml > 0) {
+    rs_status_t s = check_matrix(h, A, lda, ml, "A");
+    if (s != RS_OK) return s;
+    if ((s = check_matrix(h, Bc, ldb, h->ell, "B_c")) != RS_OK) return s;
+  }
+  RS_CUDA(h, cudaMemsetAsync(h->B1, 0, static_cast<size_t>(L.lp) * n * 8, h->st));
+  {
+    Scope sc(h, "other", 0.0);
+    RS_CUDA(h, omega_materialize(h->st, h->seed, 1u, h->ell, 0, n, h->B1, L.lp));
+  }
+  if (ml > 0) {
+    Scope sc(h, "gemm_sample", 2.0 * h->ell * static_cast<double>(ml) * n);
+    View2D Ov{h->B1, L.lp, n, L.lp};
+    View2D Av{A, ml, n, lda};
+    GemmOutDesc out{Bc, 1, ldb, 0, h->ell, static_cast<int>(ml)};
+    RS_CUDA(h, gemm_mc(h->st, L.lp, static_cast<int>(ml), n, Ov, Av, out, 1));
+  }
+  return RS_OK;
+}
+
 rs_status_t rs_lowrank_get_info(rs_lowrank_t h, int64_t* info) {
   if (!h || !info) return RS_ERR_INVALID_ARG;
   RS_CUDA(h, cudaStreamSynchronize(h->st));

@@ -30,7 +30,7 @@ ABI_FUNCTIONS = (
     "rs_lowrank_destroy",
     "rs_lowrank_get_sample", "rs_lowrank_set_sample", "rs_lowrank_get_pivot_data", "rs_lowrank_omega",
     "rs_lowrank_get_info", "rs_lowrank_get_fallbacks", "rs_lowrank_set_profiling", "rs_lowrank_get_profile", "rs_lowrank_reset_profile",
-    "rs_lowrank_kernel_launches", "rs_qp3_workspace_bytes", "rs_qp3_truncated",
+    "rs_lowrank_kernel_launches", "rs_qp3_workspace_bytes", "rs_qp3_truncated", "rs_lowrank_sample_columns",
     "rs_lowrank_last_error", "rs_comm_get_unique_id", "rs_comm_init", "rs_comm_destroy",
 )
 
@@ -78,6 +78,7 @@ def load_library(path: str = LIB_PATH):
         "rs_lowrank_reset_profile": (ctypes.c_int, [P]),
         "rs_lowrank_kernel_launches": (I64, []),
         "rs_qp3_workspace_bytes": (SZ, [I64, I64, I32]),
+        "rs_lowrank_sample_columns": (ctypes.c_int, [P, P, I64, P, I64]),
         "rs_qp3_truncated": (ctypes.c_int, [I64, I64, I32, P, I64, P, P, D, P, SZ, P]),
         "rs_lowrank_last_error": (ctypes.c_char_p, [P]),
         "rs_comm_get_unique_id": (ctypes.c_int, [ctypes.c_char_p]),
@@ -229,6 +230,15 @@ def sample_adaptive(h: Handle, A: torch.Tensor, eps: float, ell_inc: int, q: int
         return int(ell.value), est.value, rounds
     _check(code, h.ptr)
     return int(ell.value), est.value, rounds
+
+
+def sample_columns(h: Handle, A: torch.Tensor, Bc: torch.Tensor | None = None) -> torch.Tensor:
+    """Column sampling B_c = Omega_c A^T (l x m_local, Fig. 8(b)); returns B_c."""
+    if Bc is None:
+        Bc = empty_colmajor(h.k + h.p, h.m_local, device=h.workspace.device)
+    _check(load_library().rs_lowrank_sample_columns(h.ptr, A.data_ptr(), colmajor_ld(A, "A"), Bc.data_ptr(),
+                                                    colmajor_ld(Bc, "B_c")), h.ptr)
+    return Bc
 
 
 def destroy(h: Handle):

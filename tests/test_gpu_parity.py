@@ -83,6 +83,34 @@ def test_sample_row_offset_partition_sums_to_whole():
     assert rel(Bs[0], OPL.sample(np.asfortranarray(A[:1499]), k + p, SEED)) <= 1e-13
 
 
+@pytest.mark.parametrize("m,n,k,p", [(3001, 257, 16, 8), (20000, 1000, 100, 10), (500, 64, 5, 3)])
+def test_sample_columns_parity(m, n, k, p):
+    """Column sampling B_c = Omega_c A^T (Fig. 8(b)); Omega_c keyed by column index, tag 1."""
+    A, _ = make_matrix(m, n, "exp-k", k, seed=m + 7)
+    h = rs.create(m, m, 0, n, k, p, SEED)
+    try:
+        Bc = to_np(rs.sample_columns(h, to_dev(A)))
+    finally:
+        rs.destroy(h)
+    want = OP.omega(k + p, 0, n, SEED, 1) @ A.T
+    assert Bc.shape == (k + p, m)
+    assert rel(Bc, want) <= 1e-13
+
+
+def test_sample_columns_row_partition_is_local():
+    """Each rank's rows of A give exactly its own columns of B_c (no reduction)."""
+    m, n, k, p = 2001, 300, 12, 4
+    A, _ = make_matrix(m, n, "exp-k", k, seed=9)
+    want = OP.omega(k + p, 0, n, SEED, 1) @ A.T
+    for r0, r1 in [(0, 1000), (1000, m)]:
+        h = rs.create(m, r1 - r0, r0, n, k, p, SEED)
+        try:
+            Bc = to_np(rs.sample_columns(h, to_dev(np.asfortranarray(A[r0:r1]))))
+        finally:
+            rs.destroy(h)
+        assert rel(Bc, want[:, r0:r1]) <= 1e-13
+
+
 def test_sample_with_padded_leading_dimension():
     m, n, k, p = 777, 150, 10, 5
     A, _ = make_matrix(m, n, "exp-k", k, seed=3)
