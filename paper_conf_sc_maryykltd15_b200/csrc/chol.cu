@@ -10,10 +10,12 @@
 // rows of X: a parallel update from the finished block rows, then a 16-step in-block solve per
 // column.  R (upper part of M) and X (strict lower part of M, its diagonal 1/R_ii kept apart)
 // share one padded n x n array.
-// n > 128: the same blocked schedule on an L2-resident copy in the workspace.
+// n > 128: chol_cluster_kernel below (8-CTA cluster, L2-resident matrix, smem-staged rank-16
+// updates on 4 x 4 register tiles).
 // A pivot d_k <= 0 or NaN is a CholQR breakdown: reported through *info (LAPACK potrf-style
 // 1-based column) and replaced by 1 so no NaN propagates.
 #include <cstdio>
+#include <cstdlib>
 
 #include "common.cuh"
 #include "internal.h"
@@ -187,11 +189,281 @@ __global__ void __launch_bounds__(CH_BLK_THREADS, 1)
   }
 }
 
+// ------------------------------------------------------------------------------------------
+// large kernel (128 < n <= 512): one 8-CTA thread-block cluster.  The matrix lives in an
+// L2-resident work array (every CTA reads it with ld.global.cg: other CTAs write it); each step's
+// rank-16 operands are staged in every CTA's shared memory and the work of each phase is split
+// over the 2048 threads of the cluster, phases separated by cluster barriers.
+//   factor  block b: (1) CTA 0 warp 0 factors the diagonal block in registers; (2) panel
+//           P = R11^{-T} A12, one thread per trailing column; (3) A22 -= P^T P on 4 x 4
+//           register tiles of the upper triangle, P from shared memory (LDS.128).
+//   inverse X = R^{-T} (strict lower part of M, diagonal 1/R_ii apart), right-looking by block
+//           row: (a) in-block forward solve of block row b, one thread per column c < b0+16;
+//           (b) X(i, c) -= sum_kk R(b0+kk, i) X(b0+kk, c) for the later rows, 4 x 4 tiles.
+// ------------------------------------------------------------------------------------------
+constexpr int CHL_THREADS = 256;
+constexpr int CHL_MAXN = 512;
+constexpr int CHL_CLUSTER = 8;
+
+__global__ void __launch_bounds__(CHL_THREADS, 1)
+    chol_cluster_kernel(const double* __restrict__ G, int ldg, int n, double* __restrict__ R, int ldr,
+                        double* __restrict__ Linv, int ldl, double* M, double* rdg, int* info, int code,
+                        int npad) {
+  extern __shared__ double P_dyn[];  // 2 x CB x CHL_MAXN: panel / X block row, and Rs
+  double (*P)[CHL_MAXN] = reinterpret_cast<double (*)[CHL_MAXN]>(P_dyn);
+  double (*Rs)[CHL_MAXN] = reinterpret_cast<double (*)[CHL_MAXN]>(P_dyn + CB * CHL_MAXN);
+  __shared__ double D[CB][CB + 1];  // diagonal block: D[kk][j] = R[b0+kk][b0+j]
+  // volatile view for the per-column solves: keeps the block values from being hoisted into
+  // registers across the column loop (they spill otherwise)
+  volatile double (*Dv)[CB + 1] = D;
+  __shared__ double rdl[CHL_MAXN];  // 1 / R_ii
+  const int np = (n + CB - 1) / CB * CB;
+  const int LM = np + 1;
+  const int nb = np / CB;
+  const int tid = threadIdx.x, warp = tid >> 5, lane = tid & 31;
+  const int crank = static_cast<int>(cluster_ctarank());
+  constexpr int GT = CHL_THREADS * CHL_CLUSTER;
+  const int gt = crank * CHL_THREADS + tid;
+
+  // upper triangle of G, identity on the padding, zero strict lower part (X's right-hand side);
+  // eight elements per thread per round so the loads overlap
+  for (int base = 0; base < np * np; base += 8 * GT) {
+    double v[8];
+#pragma unroll
+    for (int u = 0; u < 8; ++u) {
+      const int idx = base + u * GT + gt;
+      const int i = idx % np, j = idx / np;
+      v[u] = 0.0;
+      if (idx < np * np && i <= j) v[u] = (j < n) ? G[i + static_cast<long long>(j) * ldg] : (i == j ? 1.0 : 0.0);
+    }
+#pragma unroll
+    for (int u = 0; u < 8; ++u) {
+      const int idx = base + u * GT + gt;
+      if (idx < np * np) M[idx % np + (idx / np) * LM] = v[u];
+    }
+  }
+  cluster_sync_all();
+
+  for (int b = 0; b < nb; ++b) {
+    const int b0 = b * CB;
+    const int t2 = np - b0 - CB;
+    // (1) diagonal block (CTA 0, warp 0; lane j owns column b0+j)
+    if (crank == 0 && warp == 0) {
+      double col[CB];
+#pragma unroll
+      for (int i = 0; i < CB; ++i) col[i] = (lane < CB && i <= lane) ? __ldcg(&M[(b0 + i) + (b0 + lane) * LM]) : 0.0;
+#pragma unroll
+      for (int kk = 0; kk < CB; ++kk) {
+        double d = __shfl_sync(0xffffffffu, col[kk], kk);
+        if (!(d > 0.0)) {
+          if (lane == 0 && info && b0 + kk < n) atomicCAS(info, 0, code), atomicCAS(info + 1, 0, b0 + kk + 1);
+          d = 1.0;
+        }
+        const double ri = rsqrt(d);
+        if (lane == kk) {
+          col[kk] = d * ri;
+          rdg[b0 + kk] = ri;
+        } else if (lane > kk) {
+          col[kk] *= ri;
+        }
+        const double rkj = col[kk];
+#pragma unroll
+        for (int i = kk + 1; i < CB; ++i) {
+          const double rki = __shfl_sync(0xffffffffu, col[kk], i);
+          if (lane >= i && lane < CB) col[i] = fma(-rki, rkj, col[i]);
+        }
+      }
+      if (lane < CB) {
+#pragma unroll
+        for (int i = 0; i <= lane && i < CB; ++i) M[(b0 + i) + (b0 + lane) * LM] = col[i];
+      }
+    }
+    cluster_sync_all();
+    for (int e = tid; e < CB * CB; e += CHL_THREADS) {
+      const int kk = e / CB, j = e % CB;
+      D[kk][j] = kk <= j ? __ldcg(&M[(b0 + kk) + (b0 + j) * LM]) : 0.0;
+    }
+    if (tid < CB) rdl[b0 + tid] = __ldcg(&rdg[b0 + tid]);
+    __syncthreads();
+    // (2) panel: one thread per trailing column c, x = R11^{-T} A12(:, c)
+    for (int cc = gt; cc < t2; cc += GT) {
+      const int c = b0 + CB + cc;
+      double x[CB];
+#pragma unroll
+      for (int i = 0; i < CB; ++i) x[i] = __ldcg(&M[(b0 + i) + c * LM]);
+#pragma unroll
+      for (int kk = 0; kk < CB; ++kk) {
+        x[kk] *= rdl[b0 + kk];
+#pragma unroll
+        for (int i = kk + 1; i < CB; ++i) x[i] = fma(-Dv[kk][i], x[kk], x[i]);
+      }
+#pragma unroll
+      for (int i = 0; i < CB; ++i) M[(b0 + i) + c * LM] = x[i];
+    }
+    cluster_sync_all();
+    if (t2 == 0) continue;
+    for (int e = tid; e < CB * t2; e += CHL_THREADS) {
+      const int cc = e / CB, kk = e % CB;
+      P[kk][cc] = __ldcg(&M[(b0 + kk) + (b0 + CB + cc) * LM]);
+    }
+    __syncthreads();
+    // (3) trailing update, 4 x 4 tiles (I, J), I <= J, over the upper triangle
+    {
+      const int nt = t2 / 4;
+      const int ntiles = nt * (nt + 1) / 2;
+      for (int t = gt; t < ntiles; t += GT) {
+        int J = static_cast<int>((sqrt(8.0 * t + 1.0) - 1.0) * 0.5);
+        while (J * (J + 1) / 2 > t) --J;
+        while ((J + 1) * (J + 2) / 2 <= t) ++J;
+        const int I = t - J * (J + 1) / 2;
+        const int r0 = b0 + CB + 4 * I, c0 = b0 + CB + 4 * J;
+        double a[4][4];
+#pragma unroll
+        for (int q = 0; q < 4; ++q)
+#pragma unroll
+          for (int r = 0; r < 4; ++r) a[q][r] = __ldcg(&M[(r0 + r) + (c0 + q) * LM]);
+#pragma unroll
+        for (int kk = 0; kk < CB; ++kk) {
+          const double2 p01 = *reinterpret_cast<const double2*>(&P[kk][4 * I]);
+          const double2 p23 = *reinterpret_cast<const double2*>(&P[kk][4 * I + 2]);
+          const double2 q01 = *reinterpret_cast<const double2*>(&P[kk][4 * J]);
+          const double2 q23 = *reinterpret_cast<const double2*>(&P[kk][4 * J + 2]);
+          const double pr[4] = {p01.x, p01.y, p23.x, p23.y};
+          const double pc[4] = {q01.x, q01.y, q23.x, q23.y};
+#pragma unroll
+          for (int q = 0; q < 4; ++q)
+#pragma unroll
+            for (int r = 0; r < 4; ++r) a[q][r] = fma(-pr[r], pc[q], a[q][r]);
+        }
+#pragma unroll
+        for (int q = 0; q < 4; ++q)
+#pragma unroll
+          for (int r = 0; r < 4; ++r)
+            if (I < J || r <= q) M[(r0 + r) + (c0 + q) * LM] = a[q][r];
+      }
+    }
+    cluster_sync_all();
+  }
+
+  // ---- inverse: X = R^{-T}, X(i, c) (i > c) at M[i + c*LM] (zero-initialised above) ----
+  for (int b = 0; b < nb; ++b) {
+    const int b0 = b * CB;
+    const int ncol = b0 + CB;
+    for (int e = tid; e < CB * CB; e += CHL_THREADS) {
+      const int kk = e / CB, j = e % CB;
+      D[kk][j] = kk <= j ? __ldcg(&M[(b0 + kk) + (b0 + j) * LM]) : 0.0;
+    }
+    __syncthreads();
+    // (a) in-block forward solve R_bb^T X(b, c) = rhs, one thread per column c < ncol
+    for (int c = gt; c < ncol; c += GT) {
+      double x[CB];
+#pragma unroll
+      for (int ii = 0; ii < CB; ++ii) {
+        const int i = b0 + ii;
+        x[ii] = i > c ? __ldcg(&M[i + c * LM]) : 0.0;
+      }
+#pragma unroll
+      for (int ii = 0; ii < CB; ++ii) {
+        const int i = b0 + ii;
+        double v;
+        if (i < c) {
+          v = 0.0;
+        } else if (i == c) {
+          v = rdl[i];
+        } else {
+          double s = x[ii];
+#pragma unroll
+          for (int jj = 0; jj < ii; ++jj) s = fma(-Dv[jj][ii], x[jj], s);
+          v = s * rdl[i];
+        }
+        x[ii] = v;
+      }
+#pragma unroll
+      for (int ii = 0; ii < CB; ++ii) {
+        const int i = b0 + ii;
+        if (i > c) M[i + c * LM] = x[ii];
+      }
+    }
+    cluster_sync_all();
+    const int nrow = np - ncol;
+    if (nrow == 0) continue;
+    // stage X(b rows, c < ncol) (with its diagonal and zeros above) and R(b rows, later rows)
+    for (int e = tid; e < CB * ncol; e += CHL_THREADS) {
+      const int c = e / CB, ii = e % CB;
+      const int i = b0 + ii;
+      P[ii][c] = i > c ? __ldcg(&M[i + c * LM]) : (i == c ? rdl[i] : 0.0);
+    }
+    for (int e = tid; e < CB * nrow; e += CHL_THREADS) {
+      const int ii = e / CB, kk = e % CB;
+      Rs[kk][ii] = __ldcg(&M[(b0 + kk) + (ncol + ii) * LM]);
+    }
+    __syncthreads();
+    // (b) later rows: (nrow x 16) x (16 x ncol), 4 x 4 tiles
+    const int ntr = nrow / 4, ntc = ncol / 4;
+    for (int t = gt; t < ntr * ntc; t += GT) {
+      const int I = t % ntr, J = t / ntr;
+      const int r0 = ncol + 4 * I, c0 = 4 * J;
+      double a[4][4];
+#pragma unroll
+      for (int q = 0; q < 4; ++q)
+#pragma unroll
+        for (int r = 0; r < 4; ++r) a[q][r] = __ldcg(&M[(r0 + r) + (c0 + q) * LM]);
+#pragma unroll
+      for (int kk = 0; kk < CB; ++kk) {
+        const double2 p01 = *reinterpret_cast<const double2*>(&Rs[kk][4 * I]);
+        const double2 p23 = *reinterpret_cast<const double2*>(&Rs[kk][4 * I + 2]);
+        const double2 q01 = *reinterpret_cast<const double2*>(&P[kk][c0]);
+        const double2 q23 = *reinterpret_cast<const double2*>(&P[kk][c0 + 2]);
+        const double pr[4] = {p01.x, p01.y, p23.x, p23.y};
+        const double pc[4] = {q01.x, q01.y, q23.x, q23.y};
+#pragma unroll
+        for (int q = 0; q < 4; ++q)
+#pragma unroll
+          for (int r = 0; r < 4; ++r) a[q][r] = fma(-pr[r], pc[q], a[q][r]);
+      }
+#pragma unroll
+      for (int q = 0; q < 4; ++q)
+#pragma unroll
+        for (int r = 0; r < 4; ++r) M[(r0 + r) + (c0 + q) * LM] = a[q][r];
+    }
+    cluster_sync_all();
+  }
+
+  // outputs, zero-padded to npad x npad
+  for (int base = 0; base < npad * npad; base += 8 * GT) {
+    double mv[8];
+#pragma unroll
+    for (int u = 0; u < 8; ++u) {
+      const int idx = base + u * GT + gt;
+      const int i = idx % npad, j = idx / npad;
+      mv[u] = (idx < npad * npad && i < n && j < n) ? __ldcg(&M[i + j * LM]) : 0.0;
+    }
+#pragma unroll
+    for (int u = 0; u < 8; ++u) {
+      const int idx = base + u * GT + gt;
+      if (idx >= npad * npad) continue;
+      const int i = idx % npad, j = idx / npad;
+      double rv = 0.0, lv = 0.0;
+      if (i < n && j < n) {
+        if (i <= j) rv = mv[u];
+        if (i > j) lv = mv[u];
+        else if (i == j) lv = rdl[i];
+      }
+      R[i + static_cast<long long>(j) * ldr] = rv;
+      Linv[i + static_cast<long long>(j) * ldl] = lv;
+    }
+  }
+}
+
 cudaError_t chol_inv(cudaStream_t st, const double* G, int ldg, int n, int npad, double* R, int ldr, double* Linv,
                      int ldl, double* gwork, int* info, int info_code) {
   if (n <= 0) return cudaSuccess;
   if (n > 512) return cudaErrorInvalidValue;
-  if (n <= CH_SMEM_MAX_N) {
+  static const int smem_max_n = [] {  // RS_CHOL_SMEM_MAX_N: crossover experiments only
+    const char* v = getenv("RS_CHOL_SMEM_MAX_N");
+    return v ? atoi(v) : CH_SMEM_MAX_N;
+  }();
+  if (n <= smem_max_n && n <= CH_SMEM_MAX_N) {
     const int np = (n + CB - 1) / CB * CB;
     const size_t smem = static_cast<size_t>(np) * (np + 1) * 8;
     static bool attr = false;
@@ -203,9 +475,36 @@ cudaError_t chol_inv(cudaStream_t st, const double* G, int ldg, int n, int npad,
     }
     chol_blocked_kernel<true><<<1, CH_BLK_THREADS, smem, st>>>(G, ldg, n, R, ldr, Linv, ldl, gwork, info, info_code,
                                                                 npad);
-  } else {  // same schedule on an L2-resident copy in the workspace (np x (np+1) doubles)
-    chol_blocked_kernel<false><<<1, CH_BLK_THREADS, 0, st>>>(G, ldg, n, R, ldr, Linv, ldl, gwork, info, info_code,
-                                                             npad);
+  } else {  // one 8-CTA cluster on an L2-resident copy in the workspace (np x (np+1) + np doubles)
+    const size_t smem = 2 * static_cast<size_t>(CB) * CHL_MAXN * 8;
+    static bool attr_l = false;
+    if (!attr_l) {
+      cudaError_t e = cudaFuncSetAttribute(chol_cluster_kernel, cudaFuncAttributeMaxDynamicSharedMemorySize,
+                                           static_cast<int>(smem));
+      if (e != cudaSuccess) return e;
+      if (CHL_CLUSTER > 8) {
+        e = cudaFuncSetAttribute(chol_cluster_kernel, cudaFuncAttributeNonPortableClusterSizeAllowed, 1);
+        if (e != cudaSuccess) return e;
+      }
+      attr_l = true;
+    }
+    const int np = (n + CB - 1) / CB * CB;
+    cudaLaunchConfig_t cfg{};
+    cfg.gridDim = dim3(CHL_CLUSTER, 1, 1);
+    cfg.blockDim = dim3(CHL_THREADS, 1, 1);
+    cfg.dynamicSmemBytes = smem;
+    cfg.stream = st;
+    cudaLaunchAttribute attr[1];
+    attr[0].id = cudaLaunchAttributeClusterDimension;
+    attr[0].val.clusterDim.x = CHL_CLUSTER;
+    attr[0].val.clusterDim.y = 1;
+    attr[0].val.clusterDim.z = 1;
+    cfg.attrs = attr;
+    cfg.numAttrs = 1;
+    double* rdg = gwork + static_cast<size_t>(np) * (np + 1);
+    cudaError_t e = cudaLaunchKernelEx(&cfg, chol_cluster_kernel, G, ldg, n, R, ldr, Linv, ldl, gwork, rdg, info,
+                                       info_code, npad);
+    if (e != cudaSuccess) return e;
   }
   count_launch();
   return cudaGetLastError();

@@ -76,7 +76,7 @@ Layout plan(long long m_local, long long n, int k, int p) {
   L.off_Rf = take(sq);
   L.off_Linv = take(sq);
   const size_t np16 = static_cast<size_t>(round_up(L.lmax, 16));
-  L.off_cholw = take(np16 * (np16 + 1) * 8);  // chol_inv work array (n > 128)
+  L.off_cholw = take(np16 * (np16 + 1) * 8 + np16 * 8);  // chol_inv work array + 1/R_ii (n > 128)
   L.off_Rho = take(static_cast<size_t>(L.kp) * n * 8);
   L.off_Rhat = take(static_cast<size_t>(L.kp) * n * 8);
   L.off_T = take(static_cast<size_t>(L.kp) * std::max<long long>(n - 1, 1) * 8);  // adaptive runs use k < k0
