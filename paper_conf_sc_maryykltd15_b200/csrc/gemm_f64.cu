@@ -104,16 +104,51 @@ cudaError_t launch_phx_t(cudaStream_t st, dim3 grid, const CUtensorMap& tR, cons
   }
 }
 
-template <int MFW>
-cudaError_t launch_mc_t(cudaStream_t st, dim3 grid, const CUtensorMap& tL, const CUtensorMap& tR, const GemmArgs& a) {
-  constexpr int smem = MCSmem<MFW>::TOTAL;
+template <int MFW, int WM>
+cudaError_t launch_mc_wm(cudaStream_t st, dim3 grid, const CUtensorMap& tL, const CUtensorMap& tR, const GemmArgs& a) {
+  constexpr int smem = MCSmem<MFW, WM>::TOTAL;
   static bool attr_set = false;
   if (!attr_set) {
-    cudaError_t e = cudaFuncSetAttribute(mc_gemm_kernel<MFW>, cudaFuncAttributeMaxDynamicSharedMemorySize, smem);
+    for (auto fn : {mc_gemm_kernel<MFW, WM, 0>, mc_gemm_kernel<MFW, WM, 1>, mc_gemm_kernel<MFW, WM, 2>}) {
+      cudaError_t e = cudaFuncSetAttribute(fn, cudaFuncAttributeMaxDynamicSharedMemorySize, smem);
+      if (e != cudaSuccess) return e;
+    }
+    attr_set = true;
+  }
+  if (a.tri == 1)
+    mc_gemm_kernel<MFW, WM, 1><<<grid, GEMM_THREADS, smem, st>>>(tL, tR, a);
+  else if (a.tri == 2)
+    mc_gemm_kernel<MFW, WM, 2><<<grid, GEMM_THREADS, smem, st>>>(tL, tR, a);
+  else
+    mc_gemm_kernel<MFW, WM, 0><<<grid, GEMM_THREADS, smem, st>>>(tL, tR, a);
+  count_launch();
+  return cudaGetLastError();
+}
+
+// Warp grid: 2 x 4 when the two M halves are equal, or for the triangular (K = M) products; 1 x 8
+// for the dense products with odd MFW, where the lighter warps of an uneven split run ahead and
+// spin on the ring barrier beside the heavier ones (measured at cfg4, MFW = 7: C = B A^T 33.5 ms
+// with 1 x 8 vs 35.8 ms with 2 x 4; the L^-1 C apply 0.93 ms with 2 x 4 vs 1.18 ms with 1 x 8).
+template <int MFW>
+cudaError_t launch_mc_t(cudaStream_t st, dim3 grid, const CUtensorMap& tL, const CUtensorMap& tR, const GemmArgs& a) {
+  if constexpr (MFW < 3) {
+    return launch_mc_wm<MFW, 1>(st, grid, tL, tR, a);
+  } else {
+    if (MFW % 2 == 0 || a.tri != 0) return launch_mc_wm<MFW, 2>(st, grid, tL, tR, a);
+    return launch_mc_wm<MFW, 1>(st, grid, tL, tR, a);
+  }
+}
+
+template <int R>
+cudaError_t launch_syrk_t(cudaStream_t st, dim3 grid, const CUtensorMap& tX, const GemmArgs& a) {
+  constexpr int smem = SyrkSmem<R>::TOTAL;
+  static bool attr_set = false;
+  if (!attr_set) {
+    cudaError_t e = cudaFuncSetAttribute(syrk_kernel<R>, cudaFuncAttributeMaxDynamicSharedMemorySize, smem);
     if (e != cudaSuccess) return e;
     attr_set = true;
   }
-  mc_gemm_kernel<MFW><<<grid, GEMM_THREADS, smem, st>>>(tL, tR, a);
+  syrk_kernel<R><<<grid, GEMM_THREADS, smem, st>>>(tX, a);
   count_launch();
   return cudaGetLastError();
 }
@@ -214,10 +249,11 @@ cudaError_t gemm_kc(cudaStream_t st, int M, int N, long long K, const View2D& Lv
 }
 
 cudaError_t gemm_mc(cudaStream_t st, int M, int N, long long K, const View2D& Lv, const View2D& Rv,
-                    const GemmOutDesc& out, int splits) {
+                    const GemmOutDesc& out, int splits, int tri) {
   const int MT = gemm_mtile(M);
   const int mfw = MT / 16;
   GemmArgs a = make_args(M, N, K, splits, out);
+  a.tri = tri;
   const long long nsplit = (K + a.k_chunk - 1) / a.k_chunk;
   CUtensorMap tL, tR;
   if (!make_tmap(&tL, Lv, 16, 16)) return cudaErrorInvalidValue;
@@ -232,6 +268,26 @@ cudaError_t gemm_mc(cudaStream_t st, int M, int N, long long K, const View2D& Lv
       return cudaErrorInvalidConfiguration;
   }
 #undef RS_MC
+}
+
+cudaError_t gemm_syrk(cudaStream_t st, int rows, long long K, const View2D& Xv, const GemmOutDesc& out, int splits) {
+  if (rows < 1 || rows > 128) return cudaErrorInvalidValue;
+  const int R = (rows + 15) / 16;
+  GemmArgs a = make_args(rows, rows, K, splits, out);
+  const long long nsplit = (K + a.k_chunk - 1) / a.k_chunk;
+  CUtensorMap tX;
+  if (!make_tmap(&tX, Xv, 16, static_cast<uint32_t>(16 * R))) return cudaErrorInvalidValue;
+  dim3 grid(1, 1, static_cast<unsigned>(nsplit < 1 ? 1 : nsplit));
+  switch (R) {
+    case 1: return launch_syrk_t<1>(st, grid, tX, a);
+    case 2: return launch_syrk_t<2>(st, grid, tX, a);
+    case 3: return launch_syrk_t<3>(st, grid, tX, a);
+    case 4: return launch_syrk_t<4>(st, grid, tX, a);
+    case 5: return launch_syrk_t<5>(st, grid, tX, a);
+    case 6: return launch_syrk_t<6>(st, grid, tX, a);
+    case 7: return launch_syrk_t<7>(st, grid, tX, a);
+    default: return launch_syrk_t<8>(st, grid, tX, a);
+  }
 }
 
 }  // namespace rs

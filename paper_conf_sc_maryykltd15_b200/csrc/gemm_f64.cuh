@@ -61,6 +61,7 @@ struct GemmArgs {
   long long omega_row0;  // first Omega row of this tile set (adaptive rounds draw rows [l, l + l_inc))
   int ell;               // number of Omega rows generated (rows >= ell of the tile are zero)
   int gen_mode;  // 0 = Philox + RS-BM32 (production); 1, 2 = generation-cost experiments only
+  int tri;       // MC: 0 dense, 1 L lower triangular, 2 R upper triangular (zero blocks skipped)
 };
 
 template <int MFW, bool PHILOX>
@@ -74,14 +75,6 @@ struct KCSmem {
   // lets several generator groups work on different stages at once
   static constexpr int NS = MFW <= 2 ? 8 : NSTAGE;
   static constexpr int TOTAL = 1024 + NS * (R_BYTES + L_BYTES) + 2 * NS * 8;
-};
-
-template <int MFW>
-struct MCSmem {
-  static constexpr int MT = 16 * MFW;
-  static constexpr int R_BYTES = NT * KT * 8;
-  static constexpr int L_BYTES = MT * KT * 8;
-  static constexpr int TOTAL = 1024 + NSTAGE * (R_BYTES + L_BYTES) + 2 * NSTAGE * 8;
 };
 
 // Align the dynamic shared-memory base to 1024 bytes (128B-swizzle atoms) by pointer arithmetic
@@ -384,20 +377,83 @@ __global__ void __launch_bounds__(PHX_THREADS, 1)
 
 // ------------------------------------------------------------------------------------------
 // MC family.  tmL: dims {M (contiguous), K}, box {16, 16};  tmR: dims {N (contiguous), K},
-// box {16, 16}.  One 2 KB box per 16 rows of M (or N) per stage.  Warp w owns the N box w
-// (16 columns, two fragments) and all MT rows (2*MFW fragments).
+// box {16, 16}.  One 2 KB box per 16 rows of M (or N) per stage.
+//  WM = 1: warp w owns N box w (16 columns, two fragments) and all MT rows (2*MFW fragments):
+//          per k4 step (MFW + 1) LDS.128 feed 4*MFW DMMAs (small M).
+//  WM = 2: warp (wm, wn) owns N boxes 2wn, 2wn+1 (32 columns) and M boxes [wm*BH, (wm+1)*BH),
+//          BH = ceil(MFW/2): (BH + 2) LDS.128 feed 8*BH DMMAs -- fewer non-DMMA issue slots per
+//          DMMA (profiles/r01_probe_dmma_interference.jsonl).  Warps w and w+4 share an SM
+//          sub-partition and hold the two M halves, so the sub-partitions stay balanced for odd MFW.
+// a.tri = 1: L is lower triangular (L[m][k] = 0 for k > m): an M box skips the K stages past its
+//            last row (the C1 = L^{-1} C apply of CholQR);
+// a.tri = 2: R is upper triangular (R[k][n] = 0 for k > n): an N box skips the K stages past its
+//            last column (Q1 = X R^{-1}, step 3 of Fig. 2(b)).  Skipped terms are exact zeros.
+// Epilogue: the accumulators go through shared memory (the drained ring) so every global store
+// is a 16-byte run along the output's contiguous dimension.
 // ------------------------------------------------------------------------------------------
-template <int MFW>
+template <int MFW, int WM>
+struct MCSmem {
+  static constexpr int MT = 16 * MFW;
+  static constexpr int R_BYTES = NT * KT * 8;
+  static constexpr int L_BYTES = MT * KT * 8;
+  static constexpr int RING = NSTAGE * (R_BYTES + L_BYTES);
+  static constexpr int STAGE_LD = (MT > NT ? MT : NT) + 1;  // staged tile row (doubles; odd: fewer conflicts)
+  static constexpr int STAGE = (MT > NT ? MT : NT) * STAGE_LD * 8;  // rows: MT (N-contiguous out) or NT
+  static constexpr int BODY = RING > STAGE ? RING : STAGE;
+  static constexpr int TOTAL = 1024 + BODY + 2 * NSTAGE * 8;
+};
+
+// One MC pipeline stage for a warp holding NBOX (<= BH) M boxes from mbox0 and NB N boxes from
+// nbox0.  TRI != 0: warp-uniform skips of structurally zero K blocks (see a.tri).
+template <int BH, int NBOX, int NB, int TRI>
+RS_DEVINL void mc_stage(double (&acc)[BH][2][NB][2][2], const unsigned char* Ls, const unsigned char* Rs, int mbox0,
+                        int nbox0, int r, int kk, long long kc, int m0, int n0) {
+  bool nlive[NB];
+#pragma unroll
+  for (int nb = 0; nb < NB; ++nb) nlive[nb] = TRI != 2 || n0 + 16 * (nbox0 + nb) + 15 >= kc;
+  if (TRI == 2) {
+    bool any = false;
+#pragma unroll
+    for (int nb = 0; nb < NB; ++nb) any |= nlive[nb];
+    if (!any) return;
+  }
+#pragma unroll
+  for (int ks = 0; ks < KT / 4; ++ks) {
+    const uint32_t krow = 8 * (ks >> 1) + 2 * kk + (ks & 1);
+    const uint32_t off = krow * 128u + (((static_cast<uint32_t>(r) ^ krow) & 7u) << 4);
+    double2 b2[NB];
+#pragma unroll
+    for (int nb = 0; nb < NB; ++nb) b2[nb] = *reinterpret_cast<const double2*>(Rs + (nbox0 + nb) * 2048 + off);
+#pragma unroll
+    for (int bi = 0; bi < NBOX; ++bi) {
+      const int b = mbox0 + bi;
+      if (TRI == 1 && m0 + 16 * b + 15 < kc) continue;
+      const double2 a2 = *reinterpret_cast<const double2*>(Ls + b * 2048 + off);
+#pragma unroll
+      for (int nb = 0; nb < NB; ++nb) {
+        if (TRI == 2 && !nlive[nb]) continue;
+        dmma_8x8x4(acc[bi][0][nb][0][0], acc[bi][0][nb][0][1], a2.x, b2[nb].x);
+        dmma_8x8x4(acc[bi][0][nb][1][0], acc[bi][0][nb][1][1], a2.x, b2[nb].y);
+        dmma_8x8x4(acc[bi][1][nb][0][0], acc[bi][1][nb][0][1], a2.y, b2[nb].x);
+        dmma_8x8x4(acc[bi][1][nb][1][0], acc[bi][1][nb][1][1], a2.y, b2[nb].y);
+      }
+    }
+  }
+}
+
+template <int MFW, int WM, int TRI>
 __global__ void __launch_bounds__(GEMM_THREADS, 1)
     mc_gemm_kernel(const __grid_constant__ CUtensorMap tmL, const __grid_constant__ CUtensorMap tmR,
                    const GemmArgs a) {
-  using SM = MCSmem<MFW>;
+  using SM = MCSmem<MFW, WM>;
   constexpr int MT = SM::MT;
+  constexpr int BH = WM == 1 ? MFW : (MFW + 1) / 2;  // M boxes per warp
+  constexpr int NB = WM == 1 ? 1 : 2;                // N boxes per warp
   extern __shared__ unsigned char smem_raw[];
   unsigned char* smem = align1024(smem_raw);
   unsigned char* sR = smem;
   unsigned char* sL = sR + NSTAGE * SM::R_BYTES;
-  uint64_t* full = reinterpret_cast<uint64_t*>(sL + NSTAGE * SM::L_BYTES);
+  uint64_t* full = reinterpret_cast<uint64_t*>(smem + SM::BODY);
   uint64_t* empty = full + NSTAGE;
 
   const int warp = threadIdx.x >> 5, lane = threadIdx.x & 31;
@@ -433,55 +489,280 @@ __global__ void __launch_bounds__(GEMM_THREADS, 1)
   }
 
   const int r = lane >> 2, kk = lane & 3;
-  // acc[b][f][f'][e]: M fragment (box b, parity f), N fragment (box warp, parity f'), element e
-  double acc[MFW][2][2][2];
+  const int wm = WM == 1 ? 0 : warp >> 2;
+  const int nbox0 = WM == 1 ? warp : 2 * (warp & 3);  // first N box of this warp
+  const int mbox0 = wm * BH;                          // first M box of this warp
+  // acc[bi][f][nb][f2][e]: M fragment (box mbox0+bi, parity f), N fragment (box nbox0+nb,
+  // parity f2), element e
+  double acc[BH][2][NB][2][2];
 #pragma unroll
-  for (int b = 0; b < MFW; ++b)
+  for (int bi = 0; bi < BH; ++bi)
 #pragma unroll
     for (int f = 0; f < 2; ++f)
 #pragma unroll
-      for (int f2 = 0; f2 < 2; ++f2) acc[b][f][f2][0] = acc[b][f][f2][1] = 0.0;
+      for (int nb = 0; nb < NB; ++nb)
+#pragma unroll
+        for (int f2 = 0; f2 < 2; ++f2) acc[bi][f][nb][f2][0] = acc[bi][f][nb][f2][1] = 0.0;
 
   for (int it = 0; it < nk; ++it) {
     const int s = it % NSTAGE;
     if (threadIdx.x == 0 && it + NSTAGE - 1 < nk) issue(it + NSTAGE - 1);
     mbar_wait(&full[s], (it / NSTAGE) & 1);
+    const long long kc = kb + static_cast<long long>(it) * KT;  // first K of the stage
     const unsigned char* Ls = sL + s * SM::L_BYTES;
-    const unsigned char* Rs = sR + s * SM::R_BYTES + warp * 2048;
-#pragma unroll
-    for (int ks = 0; ks < KT / 4; ++ks) {
-      const uint32_t krow = 8 * (ks >> 1) + 2 * kk + (ks & 1);
-      const uint32_t off = krow * 128u + (((static_cast<uint32_t>(r) ^ krow) & 7u) << 4);
-      const double2 b2 = *reinterpret_cast<const double2*>(Rs + off);
-#pragma unroll
-      for (int b = 0; b < MFW; ++b) {
-        const double2 a2 = *reinterpret_cast<const double2*>(Ls + b * 2048 + off);
-        dmma_8x8x4(acc[b][0][0][0], acc[b][0][0][1], a2.x, b2.x);
-        dmma_8x8x4(acc[b][0][1][0], acc[b][0][1][1], a2.x, b2.y);
-        dmma_8x8x4(acc[b][1][0][0], acc[b][1][0][1], a2.y, b2.x);
-        dmma_8x8x4(acc[b][1][1][0], acc[b][1][1][1], a2.y, b2.y);
-      }
-    }
+    const unsigned char* Rs = sR + s * SM::R_BYTES;
+    // compile-time box counts: the dense path has no per-box branches
+    if (WM == 1 || wm == 0)
+      mc_stage<BH, BH, NB, TRI>(acc, Ls, Rs, mbox0, nbox0, r, kk, kc, m0, n0);
+    else
+      mc_stage<BH, MFW - BH, NB, TRI>(acc, Ls, Rs, mbox0, nbox0, r, kk, kc, m0, n0);
     __syncwarp();
     if (lane == 0) mbar_arrive(&empty[s]);
   }
 
+  // ---- epilogue: stage the MT x NT tile in shared memory, then coalesced 16-byte stores ----
   const GemmOut& o = a.out;
   double* base = o.ptr + static_cast<long long>(blockIdx.z) * o.split_stride;
+  const bool n_contig = o.ld_n == 1, m_contig = o.ld_m == 1;
+  if (!n_contig && !m_contig) {  // generic strides: direct stores
 #pragma unroll
-  for (int b = 0; b < MFW; ++b)
+    for (int bi = 0; bi < BH; ++bi)
+#pragma unroll
+      for (int f = 0; f < 2; ++f) {
+        const long long gm = m0 + 16 * (mbox0 + bi) + 2 * r + f;
+        if (mbox0 + bi >= MFW || gm >= o.m_store) continue;
+#pragma unroll
+        for (int nb = 0; nb < NB; ++nb)
+#pragma unroll
+          for (int f2 = 0; f2 < 2; ++f2)
+#pragma unroll
+            for (int e = 0; e < 2; ++e) {
+              const long long gn = n0 + 16 * (nbox0 + nb) + 2 * (2 * kk + e) + f2;
+              if (gn < o.n_store) gemm_put(base + gm * o.ld_m + gn * o.ld_n, acc[bi][f][nb][f2][e], o.mode);
+            }
+      }
+    return;
+  }
+  __syncthreads();  // every warp is done with the ring
+  double* st = reinterpret_cast<double*>(smem);
+  // n_contig: st[m * LDS + n] (rows along N); else st[n * LDS + m] (rows along M)
+  constexpr int LDS = SM::STAGE_LD;
+#pragma unroll
+  for (int bi = 0; bi < BH; ++bi) {
+    if (mbox0 + bi >= MFW) continue;
 #pragma unroll
     for (int f = 0; f < 2; ++f) {
-      const long long gm = m0 + 16 * b + 2 * r + f;
-      if (gm >= o.m_store) continue;
+      const int lm = 16 * (mbox0 + bi) + 2 * r + f;
 #pragma unroll
-      for (int f2 = 0; f2 < 2; ++f2)
+      for (int nb = 0; nb < NB; ++nb)
 #pragma unroll
-        for (int e = 0; e < 2; ++e) {
-          const long long gn = n0 + 16 * warp + 2 * (2 * kk + e) + f2;
-          if (gn < o.n_store) gemm_put(base + gm * o.ld_m + gn * o.ld_n, acc[b][f][f2][e], o.mode);
-        }
+        for (int f2 = 0; f2 < 2; ++f2)
+#pragma unroll
+          for (int e = 0; e < 2; ++e) {
+            const int ln = 16 * (nbox0 + nb) + 2 * (2 * kk + e) + f2;
+            st[n_contig ? lm * LDS + ln : ln * LDS + lm] = acc[bi][f][nb][f2][e];
+          }
     }
+  }
+  __syncthreads();
+  // rows of the staged tile: n_contig -> MT rows of NT; else NT rows of MT
+  const int nrows = n_contig ? MT : NT, rowlen = n_contig ? NT : MT;
+  const long long row0 = n_contig ? m0 : n0, col0 = n_contig ? n0 : m0;
+  const long long row_lim = n_contig ? o.m_store : o.n_store, col_lim = n_contig ? o.n_store : o.m_store;
+  const long long ld_row = n_contig ? o.ld_m : o.ld_n;
+  const int pairs = rowlen / 2;
+  for (int idx = threadIdx.x; idx < nrows * pairs; idx += GEMM_THREADS) {
+    const int lr = idx / pairs, lc = 2 * (idx - lr * pairs);
+    const long long gr = row0 + lr, gc = col0 + lc;
+    if (gr >= row_lim || gc >= col_lim) continue;
+    double* p = base + gr * ld_row + gc;
+    const double v0 = st[lr * LDS + lc], v1 = st[lr * LDS + lc + 1];
+    if (gc + 1 < col_lim && (reinterpret_cast<uintptr_t>(p) & 15) == 0) {
+      double2* p2 = reinterpret_cast<double2*>(p);
+      if (o.mode) {
+        double2 c = *p2;
+        c.x -= v0;
+        c.y -= v1;
+        *p2 = c;
+      } else {
+        *p2 = make_double2(v0, v1);
+      }
+    } else {
+      gemm_put(p, v0, o.mode);
+      if (gc + 1 < col_lim) gemm_put(p + 1, v1, o.mode);
+    }
+  }
+}
+
+// ------------------------------------------------------------------------------------------
+// SYRK: the Gram matrix G = X X^T of the <= 128 rows of a K-contiguous X (CholQR step (i),
+// G = C C^T of the distributed C, G = (A P1)^T (A P1) of step 3).  G is symmetric, so
+// only the lower-triangle 16 x 16 blocks (I, J), J <= I, are computed -- R(R+1)/2 of R^2 blocks,
+// and no N padding to 128 -- and each is stored to both triangles.  One operand tile per stage
+// (TMA box {16 (K), 16R}, 128B swizzle; the KC fragment layout of kc_row / kc_pair_off): a
+// thread's K pair of row kc_row(g, f, r) is both the A fragment (row r of the 8-row fragment)
+// and the B fragment (column r) of a DMMA, so one LDS.128 per 8 rows feeds every block that row
+// group takes part in.  Warp w takes a contiguous run of the row-major lower-triangle block list
+// (runs differ by at most one block; warps w and w + 4 share an SM sub-partition and together
+// hold about 2/8 of the blocks).  Each warp's block list and the row groups it must load are
+// compile-time constants (one specialised main loop per warp), so every group is loaded once
+// per K pair.  Split-K over blockIdx.z into partial Grams, reduced in a fixed order.
+// ------------------------------------------------------------------------------------------
+template <int R>
+struct SyrkPlan {
+  static constexpr int T = R * (R + 1) / 2;  // lower-triangle blocks
+  static constexpr int MAXB = (T + 7) / 8;
+  __host__ __device__ static constexpr int count(int w) { return T / 8 + (w < T % 8 ? 1 : 0); }
+  __host__ __device__ static constexpr int start(int w) {
+    int s = 0;
+    for (int i = 0; i < w; ++i) s += count(i);
+    return s;
+  }
+  __host__ __device__ static constexpr int blk_i(int idx) {
+    int I = 0;
+    while ((I + 1) * (I + 2) / 2 <= idx) ++I;
+    return I;
+  }
+  __host__ __device__ static constexpr int blk_j(int idx) { return idx - blk_i(idx) * (blk_i(idx) + 1) / 2; }
+  __host__ __device__ static constexpr bool need(int w, int g) {
+    for (int s = 0; s < count(w); ++s) {
+      const int idx = start(w) + s;
+      if (blk_i(idx) == g || blk_j(idx) == g) return true;
+    }
+    return false;
+  }
+};
+
+constexpr int SYRK_NS = 8;  // ring depth (stages are 16R x 16 doubles, <= 16 KB)
+
+template <int R>
+struct SyrkSmem {
+  static constexpr int X_BYTES = 16 * R * KT * 8;
+  static constexpr int TOTAL = 1024 + SYRK_NS * X_BYTES + 2 * SYRK_NS * 8;
+};
+
+template <int R, int W, typename Issue>
+RS_DEVINL void syrk_warp(const unsigned char* sX, uint64_t* full, uint64_t* empty, int nk, int lane, Issue&& issue,
+                         double* out, long long ld, int n_store) {
+  using P = SyrkPlan<R>;
+  constexpr int NB = P::count(W);
+  if constexpr (NB == 0) {
+    // no blocks: still release every slot so the producer can refill it
+    for (int it = 0; it < nk; ++it) {
+      const int s = it % SYRK_NS;
+      if (threadIdx.x == 0 && it + SYRK_NS - 1 < nk) issue(it + SYRK_NS - 1);
+      mbar_wait(&full[s], (it / SYRK_NS) & 1);
+      __syncwarp();
+      if (lane == 0) mbar_arrive(&empty[s]);
+    }
+    return;
+  } else {
+    const int r = lane >> 2, kk = lane & 3;
+    double acc[NB][2][2][2];
+#pragma unroll
+    for (int b = 0; b < NB; ++b)
+#pragma unroll
+      for (int f = 0; f < 2; ++f)
+#pragma unroll
+        for (int f2 = 0; f2 < 2; ++f2) acc[b][f][f2][0] = acc[b][f][f2][1] = 0.0;
+    for (int it = 0; it < nk; ++it) {
+      const int s = it % SYRK_NS;
+      if (threadIdx.x == 0 && it + SYRK_NS - 1 < nk) issue(it + SYRK_NS - 1);
+      mbar_wait(&full[s], (it / SYRK_NS) & 1);
+      const unsigned char* Xs = sX + s * SyrkSmem<R>::X_BYTES;
+#pragma unroll
+      for (int p = 0; p < 2; ++p) {
+        double2 fr[R][2];
+#pragma unroll
+        for (int g = 0; g < R; ++g) {
+          if (P::need(W, g)) {
+#pragma unroll
+            for (int f = 0; f < 2; ++f)
+              fr[g][f] = *reinterpret_cast<const double2*>(Xs + kc_pair_off(kc_row(g, f, r), p, kk));
+          }
+        }
+#pragma unroll
+        for (int b = 0; b < NB; ++b) {
+          const int I = P::blk_i(P::start(W) + b), J = P::blk_j(P::start(W) + b);
+#pragma unroll
+          for (int f = 0; f < 2; ++f)
+#pragma unroll
+            for (int f2 = 0; f2 < 2; ++f2) {
+              dmma_8x8x4(acc[b][f][f2][0], acc[b][f][f2][1], fr[I][f].x, fr[J][f2].x);
+              dmma_8x8x4(acc[b][f][f2][0], acc[b][f][f2][1], fr[I][f].y, fr[J][f2].y);
+            }
+        }
+      }
+      __syncwarp();
+      if (lane == 0) mbar_arrive(&empty[s]);
+    }
+    // G[kc_row(I, f, r)][kc_row(J, f2, 2kk + e)] and its mirror
+#pragma unroll
+    for (int b = 0; b < NB; ++b) {
+      const int I = P::blk_i(P::start(W) + b), J = P::blk_j(P::start(W) + b);
+#pragma unroll
+      for (int f = 0; f < 2; ++f)
+#pragma unroll
+        for (int f2 = 0; f2 < 2; ++f2)
+#pragma unroll
+          for (int e = 0; e < 2; ++e) {
+            const int i = kc_row(I, f, r), j = kc_row(J, f2, 2 * kk + e);
+            if (i < n_store && j < n_store) {
+              out[i + j * ld] = acc[b][f][f2][e];
+              out[j + i * ld] = acc[b][f][f2][e];
+            }
+          }
+    }
+  }
+}
+
+// tmX: dims {K (contiguous), rows}, box {16, 16R}.  out: partial Gram of split z at
+// out + z * split_stride, element (i, j) at i + j * ld_n (i, j < n_store).
+template <int R>
+__global__ void __launch_bounds__(GEMM_THREADS, 1)
+    syrk_kernel(const __grid_constant__ CUtensorMap tmX, const GemmArgs a) {
+  using SM = SyrkSmem<R>;
+  extern __shared__ unsigned char smem_raw[];
+  unsigned char* smem = align1024(smem_raw);
+  unsigned char* sX = smem;
+  uint64_t* full = reinterpret_cast<uint64_t*>(sX + SYRK_NS * SM::X_BYTES);
+  uint64_t* empty = full + SYRK_NS;
+  const int warp = threadIdx.x >> 5, lane = threadIdx.x & 31;
+  const long long kb = static_cast<long long>(blockIdx.z) * a.k_chunk;
+  const long long ke = min(a.K, kb + a.k_chunk);
+  const int nk = kb < ke ? static_cast<int>((ke - kb + KT - 1) / KT) : 0;
+  if (threadIdx.x == 0) {
+#pragma unroll
+    for (int s = 0; s < SYRK_NS; ++s) {
+      mbar_init(&full[s], 1);
+      mbar_init(&empty[s], NCONS);
+    }
+    fence_mbar_init();
+  }
+  __syncthreads();
+  auto issue = [&](int it) {
+    const int s = it % SYRK_NS;
+    if (it >= SYRK_NS) mbar_wait(&empty[s], ((it / SYRK_NS) - 1) & 1);
+    mbar_arrive_expect_tx(&full[s], SM::X_BYTES);
+    tma_load_2d(sX + s * SM::X_BYTES, &tmX, &full[s], static_cast<int>(kb + static_cast<long long>(it) * KT), 0);
+  };
+  if (threadIdx.x == 0) {
+    tma_prefetch_desc(&tmX);
+    for (int it = 0; it < SYRK_NS - 1 && it < nk; ++it) issue(it);
+  }
+  double* out = a.out.ptr + static_cast<long long>(blockIdx.z) * a.out.split_stride;
+  const long long ld = a.out.ld_n;
+  const int ns = a.out.n_store;
+  switch (warp) {
+    case 0: syrk_warp<R, 0>(sX, full, empty, nk, lane, issue, out, ld, ns); break;
+    case 1: syrk_warp<R, 1>(sX, full, empty, nk, lane, issue, out, ld, ns); break;
+    case 2: syrk_warp<R, 2>(sX, full, empty, nk, lane, issue, out, ld, ns); break;
+    case 3: syrk_warp<R, 3>(sX, full, empty, nk, lane, issue, out, ld, ns); break;
+    case 4: syrk_warp<R, 4>(sX, full, empty, nk, lane, issue, out, ld, ns); break;
+    case 5: syrk_warp<R, 5>(sX, full, empty, nk, lane, issue, out, ld, ns); break;
+    case 6: syrk_warp<R, 6>(sX, full, empty, nk, lane, issue, out, ld, ns); break;
+    default: syrk_warp<R, 7>(sX, full, empty, nk, lane, issue, out, ld, ns); break;
+  }
 }
 
 }  // namespace rs

@@ -36,8 +36,13 @@ struct PhiloxDesc {
 // `ns_kernel` (optional) receives the kernel's device time when events != nullptr.
 cudaError_t gemm_kc(cudaStream_t st, int M, int N, long long K, const View2D& Lv, const View2D& Rv,
                     const PhiloxDesc& phx, const GemmOutDesc& out, int splits);
+// tri (MC only): 0 dense; 1 L lower triangular; 2 R upper triangular -- structurally zero K
+// blocks are skipped (exact: they only add zeros).
 cudaError_t gemm_mc(cudaStream_t st, int M, int N, long long K, const View2D& Lv, const View2D& Rv,
-                    const GemmOutDesc& out, int splits);
+                    const GemmOutDesc& out, int splits, int tri = 0);
+// G (+split partials) = X X^T for the rows <= 128 rows of a K-contiguous X (Xv: dim0 = K, dim1 =
+// rows); lower-triangle blocks only, stored to both triangles (out.ld_m must be 1).
+cudaError_t gemm_syrk(cudaStream_t st, int rows, long long K, const View2D& Xv, const GemmOutDesc& out, int splits);
 int gemm_choose_splits(int M, int N, long long K, int max_splits, int num_sms);
 int gemm_nsplit(long long K, int splits);   // splits actually launched for a requested count
 int gemm_mtile(int M);   // rows per CTA tile used for M

@@ -215,8 +215,12 @@ rs_status_t gram_rows_kc(rs_lowrank_t h, const double* X, long long ldx, long lo
     if (K > 0) {
       View2D Xv{X, K, rows, ldx};
       GemmOutDesc out{h->part, 1, ld_g, static_cast<long long>(ld_g) * ld_g, ld_g, ld_g};
-      PhiloxDesc nophx{false, 0, 0, 0, 0};
-      RS_CUDA(h, gemm_kc(h->st, rows, rows, K, Xv, Xv, nophx, out, splits));
+      if (rows <= 128) {  // symmetric: lower-triangle blocks only
+        RS_CUDA(h, gemm_syrk(h->st, rows, K, Xv, out, splits));
+      } else {
+        PhiloxDesc nophx{false, 0, 0, 0, 0};
+        RS_CUDA(h, gemm_kc(h->st, rows, rows, K, Xv, Xv, nophx, out, splits));
+      }
     } else {
       RS_CUDA(h, cudaMemsetAsync(h->part, 0, static_cast<size_t>(ld_g) * ld_g * 8, h->st));
     }
@@ -300,7 +304,7 @@ rs_status_t cholqr_dist(rs_lowrank_t h, double* Cn, int rr, int rp, int npass, i
       View2D Lv{h->Linv, rp, rp, rp};
       View2D Cv{src, ml, rp, L.ldc};
       GemmOutDesc out{dst, L.ldc, 1, 0, rp, static_cast<int>(ml)};
-      RS_CUDA(h, gemm_mc(h->st, rp, static_cast<int>(ml), rp, Lv, Cv, out, 1));
+      RS_CUDA(h, gemm_mc(h->st, rp, static_cast<int>(ml), rp, Lv, Cv, out, 1, 1));  // Linv lower
     }
   }
   return RS_OK;
@@ -511,7 +515,7 @@ rs_status_t rs_lowrank_power_iterate(rs_lowrank_t h, const double* A, int64_t ld
       View2D Lv{h->Linv, L.lp, L.lp, L.lp};
       View2D Cv{h->C, ml, L.lp, L.ldc};
       GemmOutDesc out{h->C1, L.ldc, 1, 0, L.lp, static_cast<int>(ml)};
-      RS_CUDA(h, gemm_mc(h->st, L.lp, static_cast<int>(ml), L.lp, Lv, Cv, out, 1));
+      RS_CUDA(h, gemm_mc(h->st, L.lp, static_cast<int>(ml), L.lp, Lv, Cv, out, 1, 1));  // Linv lower
     }
     s = gram_rows_kc(h, h->C1, L.ldc, ml, L.lp, L.lp);
     if (s != RS_OK) return s;
@@ -622,7 +626,7 @@ rs_status_t rs_lowrank_factor(rs_lowrank_t h, const double* A, int64_t lda, doub
         View2D Xv{src, ml, k, ld_src};
         View2D Wv{h->Linv, k, k, L.kp};
         GemmOutDesc out{dst, 1, ld_dst, 0, static_cast<int>(ml), k};
-        RS_CUDA(h, gemm_mc(h->st, static_cast<int>(ml), k, k, Xv, Wv, out, 1));
+        RS_CUDA(h, gemm_mc(h->st, static_cast<int>(ml), k, k, Xv, Wv, out, 1, 2));  // R^-1 upper
       }
       {
         Scope sc(h, "other", 2.0 * k * static_cast<double>(k) * k);
