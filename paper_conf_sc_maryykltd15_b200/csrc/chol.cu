@@ -455,6 +455,155 @@ __global__ void __launch_bounds__(CHL_THREADS, 1)
   }
 }
 
+// ------------------------------------------------------------------------------------------
+// register-tile kernel (n <= 128): right-looking Cholesky and forward substitution for
+// X = R^{-T} advanced together, ONE barrier per pivot.  The upper triangle of G and the lower
+// triangle of the right-hand-side accumulators of X live in 4 x 4 register tiles (TPT per
+// thread).  At step k every thread reads the published row k of G and of X's accumulators and
+// forms 1/d_k = rsqrt(d_k)^2 itself (all threads see the same d_k, so all get the same value);
+// the rank-1 updates are G(i, j) -= G(k, i) G(k, j) / d_k (= R(k, i) R(k, j)) and
+// acc(i, c) -= G(k, i) acc(k, c) / d_k (= R(k, i) X(k, c)); the owners of row k + 1 publish it
+// into the other buffer.  The step loop is unrolled by 4 so the tile row being published is a
+// compile-time register index.  Rows <= k of a tile are dead after step k (already written out),
+// so the updates need no predicates.  Tiles are ordered by row block, descending, so whole warps
+// retire as k grows.
+// ------------------------------------------------------------------------------------------
+constexpr int CT_MAXN = 128;
+
+template <int TPT, int NTHR>
+struct CholTile {
+  double v[TPT][4][4];
+  int kind[TPT], TI[TPT], TJ[TPT];
+  bool has[TPT];
+};
+
+// one pivot step k with (k + 1) % 4 == A1 (the tile row that holds row k + 1)
+template <int A1, int TPT, int NTHR>
+RS_DEVINL void chol_tile_step(CholTile<TPT, NTHR>& T, int k, int n, int npad, double (*Gp)[CT_MAXN],
+                              double (*Xp)[CT_MAXN], double* __restrict__ R, int ldr, double* __restrict__ Linv,
+                              int ldl, int* info, int code) {
+  const int tid = threadIdx.x;
+  const int par = k & 1;
+  double d = Gp[par][k];
+  if (!(d > 0.0)) {
+    if (tid == 0 && info && k < n) atomicCAS(info, 0, code), atomicCAS(info + 1, 0, k + 1);
+    d = 1.0;
+  }
+  const double ri = rsqrt(d);
+  const double dinv = ri * ri;
+  const int ipub = (k + 1) >> 2;  // tile row block holding row k + 1
+#pragma unroll
+  for (int s2 = 0; s2 < TPT; ++s2) {
+    if (!T.has[s2] || 4 * T.TI[s2] + 3 <= k) continue;  // rows of the tile all finished
+    const double2* gpi = reinterpret_cast<const double2*>(&Gp[par][4 * T.TI[s2]]);
+    const double2 gi0 = gpi[0], gi1 = gpi[1];
+    const double ra[4] = {gi0.x * dinv, gi0.y * dinv, gi1.x * dinv, gi1.y * dinv};
+    const double2* src = T.kind[s2] == 0 ? reinterpret_cast<const double2*>(&Gp[par][4 * T.TJ[s2]])
+                                         : reinterpret_cast<const double2*>(&Xp[par][4 * T.TJ[s2]]);
+    const double2 c0 = src[0], c1 = src[1];
+    const double cb[4] = {c0.x, c0.y, c1.x, c1.y};
+#pragma unroll
+    for (int a = 0; a < 4; ++a)
+#pragma unroll
+      for (int bb = 0; bb < 4; ++bb) T.v[s2][a][bb] = fma(-ra[a], cb[bb], T.v[s2][a][bb]);
+    if (T.TI[s2] == ipub) {  // publish row k + 1 = tile row A1
+      const int c = 4 * T.TJ[s2];
+      if (T.kind[s2] == 0) {
+        reinterpret_cast<double2*>(&Gp[par ^ 1][c])[0] = make_double2(T.v[s2][A1][0], T.v[s2][A1][1]);
+        reinterpret_cast<double2*>(&Gp[par ^ 1][c])[1] = make_double2(T.v[s2][A1][2], T.v[s2][A1][3]);
+      } else {
+        const int lim = k + 1 - c;  // X(k + 1, c + bb) = 0 for c + bb > k + 1
+        reinterpret_cast<double2*>(&Xp[par ^ 1][c])[0] =
+            make_double2(lim >= 0 ? T.v[s2][A1][0] : 0.0, lim >= 1 ? T.v[s2][A1][1] : 0.0);
+        reinterpret_cast<double2*>(&Xp[par ^ 1][c])[1] =
+            make_double2(lim >= 2 ? T.v[s2][A1][2] : 0.0, lim >= 3 ? T.v[s2][A1][3] : 0.0);
+      }
+    }
+  }
+  // row k of R and of Linv = R^{-T}
+  if (k < n) {
+    for (int t = tid; t < npad; t += NTHR) {
+      double rv = 0.0, lv = 0.0;
+      if (t < n) {
+        if (t > k) rv = Gp[par][t] * ri;
+        else if (t == k) rv = d * ri;
+        if (t < k) lv = Xp[par][t] * ri;
+        else if (t == k) lv = ri;
+      }
+      R[k + static_cast<long long>(t) * ldr] = rv;
+      Linv[k + static_cast<long long>(t) * ldl] = lv;
+    }
+  }
+  __syncthreads();
+}
+
+template <int TPT, int NTHR>
+__global__ void __launch_bounds__(NTHR, 1)
+    chol_tile_kernel(const double* __restrict__ G, int ldg, int n, double* __restrict__ R, int ldr,
+                     double* __restrict__ Linv, int ldl, int* info, int code, int npad) {
+  __shared__ __align__(16) double Gp[2][CT_MAXN];
+  __shared__ __align__(16) double Xp[2][CT_MAXN];
+  const int tid = threadIdx.x;
+  const int np = (n + 3) / 4 * 4;
+  const int nt = np / 4;  // tile blocks per dimension
+  CholTile<TPT, NTHR> T;
+#pragma unroll
+  for (int s2 = 0; s2 < TPT; ++s2) {
+    const int t = tid + s2 * NTHR;
+    T.has[s2] = t < nt * (nt + 1);
+    T.kind[s2] = 0, T.TI[s2] = 0, T.TJ[s2] = 0;
+    if (T.has[s2]) {
+      // row block I (from nt-1 down) holds (nt - I) G tiles (J = I..nt-1), then I + 1 X tiles
+      const int q = t / (nt + 1), rr = t - q * (nt + 1);
+      const int I = nt - 1 - q;
+      T.TI[s2] = I;
+      if (rr < nt - I) {
+        T.TJ[s2] = I + rr;
+      } else {
+        T.kind[s2] = 1;
+        T.TJ[s2] = rr - (nt - I);
+      }
+    }
+#pragma unroll
+    for (int a = 0; a < 4; ++a)
+#pragma unroll
+      for (int bb = 0; bb < 4; ++bb) {
+        const int i = 4 * T.TI[s2] + a, j = 4 * T.TJ[s2] + bb;
+        double x = 0.0;
+        if (T.has[s2]) {
+          if (T.kind[s2] == 0) {
+            const int lo = i < j ? i : j, hi = i < j ? j : i;
+            x = (hi < n) ? G[lo + static_cast<long long>(hi) * ldg] : (i == j ? 1.0 : 0.0);
+          } else {
+            x = (i == j) ? 1.0 : 0.0;
+          }
+        }
+        T.v[s2][a][bb] = x;
+      }
+  }
+  // row 0; X's rows are published only up to the publishing tile's last column, so both X
+  // buffers start at zero (X(k, c) = 0 for c > k must read as zero)
+  for (int j = tid; j < CT_MAXN; j += NTHR) {
+    Gp[0][j] = j < np ? ((j < n) ? G[static_cast<long long>(j) * ldg] : (j == 0 ? 1.0 : 0.0)) : 0.0;
+    Gp[1][j] = 0.0;
+    Xp[0][j] = j == 0 ? 1.0 : 0.0;
+    Xp[1][j] = 0.0;
+  }
+  __syncthreads();
+  for (int k = 0; k < np; k += 4) {  // np is a multiple of 4
+    chol_tile_step<1>(T, k, n, npad, Gp, Xp, R, ldr, Linv, ldl, info, code);
+    chol_tile_step<2>(T, k + 1, n, npad, Gp, Xp, R, ldr, Linv, ldl, info, code);
+    chol_tile_step<3>(T, k + 2, n, npad, Gp, Xp, R, ldr, Linv, ldl, info, code);
+    chol_tile_step<0>(T, k + 3, n, npad, Gp, Xp, R, ldr, Linv, ldl, info, code);
+  }
+  // zero padding rows n..npad-1
+  for (int idx = tid; idx < (npad - n) * npad; idx += NTHR) {
+    const int kk = n + idx / npad, t = idx % npad;
+    R[kk + static_cast<long long>(t) * ldr] = 0.0;
+    Linv[kk + static_cast<long long>(t) * ldl] = 0.0;
+  }
+}
+
 cudaError_t chol_inv(cudaStream_t st, const double* G, int ldg, int n, int npad, double* R, int ldr, double* Linv,
                      int ldl, double* gwork, int* info, int info_code) {
   if (n <= 0) return cudaSuccess;
@@ -463,7 +612,14 @@ cudaError_t chol_inv(cudaStream_t st, const double* G, int ldg, int n, int npad,
     const char* v = getenv("RS_CHOL_SMEM_MAX_N");
     return v ? atoi(v) : CH_SMEM_MAX_N;
   }();
-  if (n <= smem_max_n && n <= CH_SMEM_MAX_N) {
+  static const bool use_tile = getenv("RS_CHOL_BLOCKED") == nullptr;  // development switch
+  if (use_tile && n <= CT_MAXN) {
+    const int nt = (n + 3) / 4;
+    if (nt * (nt + 1) <= 1024)  // one tile per thread (n <= 124)
+      chol_tile_kernel<1, 1024><<<1, 1024, 0, st>>>(G, ldg, n, R, ldr, Linv, ldl, info, info_code, npad);
+    else
+      chol_tile_kernel<2, 576><<<1, 576, 0, st>>>(G, ldg, n, R, ldr, Linv, ldl, info, info_code, npad);
+  } else if (n <= smem_max_n && n <= CH_SMEM_MAX_N) {
     const int np = (n + CB - 1) / CB * CB;
     const size_t smem = static_cast<size_t>(np) * (np + 1) * 8;
     static bool attr = false;

@@ -1,5 +1,7 @@
 // Host launchers for the FP64 DMMA GEMM families (tensor-map encoding, tile/split choice).
+#include <algorithm>
 #include <cstdio>
+#include <cstdlib>
 #include <mutex>
 
 #include "gemm_f64.cuh"
@@ -125,16 +127,58 @@ cudaError_t launch_mc_wm(cudaStream_t st, dim3 grid, const CUtensorMap& tL, cons
   return cudaGetLastError();
 }
 
-// Warp grid: 2 x 4 when the two M halves are equal, or for the triangular (K = M) products; 1 x 8
-// for the dense products with odd MFW, where the lighter warps of an uneven split run ahead and
-// spin on the ring barrier beside the heavier ones (measured at cfg4, MFW = 7: C = B A^T 33.5 ms
-// with 1 x 8 vs 35.8 ms with 2 x 4; the L^-1 C apply 0.93 ms with 2 x 4 vs 1.18 ms with 1 x 8).
+template <int MFW, int WM>
+cudaError_t launch_mcp_wm(cudaStream_t st, int grid, const CUtensorMap& tL, const CUtensorMap& tR, const GemmArgs& a,
+                          int ntn, int ntiles) {
+  constexpr int smem = MCPSmem<MFW, WM>::TOTAL;
+  static bool attr_set = false;
+  if (!attr_set) {
+    for (auto fn : {mc_persist_kernel<MFW, WM, 0>, mc_persist_kernel<MFW, WM, 1>, mc_persist_kernel<MFW, WM, 2>}) {
+      cudaError_t e = cudaFuncSetAttribute(fn, cudaFuncAttributeMaxDynamicSharedMemorySize, smem);
+      if (e != cudaSuccess) return e;
+    }
+    attr_set = true;
+  }
+  if (a.tri == 1)
+    mc_persist_kernel<MFW, WM, 1><<<grid, GEMM_THREADS, smem, st>>>(tL, tR, a, ntn, ntiles);
+  else if (a.tri == 2)
+    mc_persist_kernel<MFW, WM, 2><<<grid, GEMM_THREADS, smem, st>>>(tL, tR, a, ntn, ntiles);
+  else
+    mc_persist_kernel<MFW, WM, 0><<<grid, GEMM_THREADS, smem, st>>>(tL, tR, a, ntn, ntiles);
+  count_launch();
+  return cudaGetLastError();
+}
+
+template <int MFW>
+cudaError_t launch_mcp_t(cudaStream_t st, int grid, const CUtensorMap& tL, const CUtensorMap& tR, const GemmArgs& a,
+                         int ntn, int ntiles) {
+  if constexpr (MFW < 3) {
+    return launch_mcp_wm<MFW, 1>(st, grid, tL, tR, a, ntn, ntiles);
+  } else {
+    return launch_mcp_wm<MFW, 2>(st, grid, tL, tR, a, ntn, ntiles);
+  }
+}
+
+// Warp grid.  Dense (long-K) products: 1 x 8 -- each warp 16 columns and all M fragments.  The
+// 2 x 4 grid (each warp half of the M fragments, the middle box split by row parity at odd MFW,
+// and 32 columns; (MFW/2 + 2) instead of (MFW + 1) LDS.128 per 4 MFW DMMAs) measured slower at
+// cfg4 for C = B A^T (MFW = 7): 34.4 ms vs 33.5 ms with 1 x 8 (an earlier box-granular uneven
+// split: 35.8 ms).  Short-K triangular products (and the persistent kernel): 2 x 4, measured
+// faster for the L^-1 C apply (0.93 vs 1.18 ms at cfg4).  RS_MC_WM = 1 / 2 forces a grid.
+static inline int mc_wm_override() {
+  static const int v = [] {
+    const char* e = getenv("RS_MC_WM");  // development switch: 1 or 2
+    return e ? atoi(e) : 0;
+  }();
+  return v;
+}
 template <int MFW>
 cudaError_t launch_mc_t(cudaStream_t st, dim3 grid, const CUtensorMap& tL, const CUtensorMap& tR, const GemmArgs& a) {
   if constexpr (MFW < 3) {
     return launch_mc_wm<MFW, 1>(st, grid, tL, tR, a);
   } else {
-    if (MFW % 2 == 0 || a.tri != 0) return launch_mc_wm<MFW, 2>(st, grid, tL, tR, a);
+    const int wm = mc_wm_override() ? mc_wm_override() : (a.tri != 0 ? 2 : 1);
+    if (wm == 2) return launch_mc_wm<MFW, 2>(st, grid, tL, tR, a);
     return launch_mc_wm<MFW, 1>(st, grid, tL, tR, a);
   }
 }
@@ -154,6 +198,15 @@ cudaError_t launch_syrk_t(cudaStream_t st, dim3 grid, const CUtensorMap& tX, con
 }
 
 }  // namespace
+
+int num_sms_cached() {
+  static int sms = [] {
+    int dev = 0, n = 148;
+    if (cudaGetDevice(&dev) == cudaSuccess) cudaDeviceGetAttribute(&n, cudaDevAttrMultiProcessorCount, dev);
+    return n;
+  }();
+  return sms;
+}
 
 int gemm_mtile(int M) {
   if (M <= 128) return 16 * ((M + 15) / 16);
@@ -259,6 +312,21 @@ cudaError_t gemm_mc(cudaStream_t st, int M, int N, long long K, const View2D& Lv
   if (!make_tmap(&tL, Lv, 16, 16)) return cudaErrorInvalidValue;
   if (!make_tmap(&tR, Rv, 16, 16)) return cudaErrorInvalidValue;
   dim3 grid((N + NT - 1) / NT, (M + MT - 1) / MT, static_cast<unsigned>(nsplit < 1 ? 1 : nsplit));
+  // short K and many tiles: persistent CTAs (the ring runs on across tiles)
+  static const bool no_persist = getenv("RS_MC_NO_PERSIST") != nullptr;  // development switch
+  const long long ntiles = static_cast<long long>(grid.x) * grid.y;
+  if (!no_persist && nsplit <= 1 && K <= 8 * KT && ntiles >= 2LL * num_sms_cached()) {
+    const int pgrid = static_cast<int>(std::min<long long>(ntiles, num_sms_cached()));
+#define RS_MCP(W) \
+  case W:         \
+    return launch_mcp_t<W>(st, pgrid, tL, tR, a, static_cast<int>(grid.x), static_cast<int>(ntiles));
+    switch (mfw) {
+      RS_MCP(1) RS_MCP(2) RS_MCP(3) RS_MCP(4) RS_MCP(5) RS_MCP(6) RS_MCP(7) RS_MCP(8)
+      default:
+        return cudaErrorInvalidConfiguration;
+    }
+#undef RS_MCP
+  }
 #define RS_MC(W) \
   case W:        \
     return launch_mc_t<W>(st, grid, tL, tR, a);

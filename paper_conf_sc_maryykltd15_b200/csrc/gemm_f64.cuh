@@ -403,11 +403,16 @@ struct MCSmem {
   static constexpr int TOTAL = 1024 + BODY + 2 * NSTAGE * 8;
 };
 
-// One MC pipeline stage for a warp holding NBOX (<= BH) M boxes from mbox0 and NB N boxes from
-// nbox0.  TRI != 0: warp-uniform skips of structurally zero K blocks (see a.tri).
-template <int BH, int NBOX, int NB, int TRI>
-RS_DEVINL void mc_stage(double (&acc)[BH][2][NB][2][2], const unsigned char* Ls, const unsigned char* Rs, int mbox0,
-                        int nbox0, int r, int kk, long long kc, int m0, int n0) {
+// One MC pipeline stage for a warp holding the NFR 8-row M fragments PHI0 .. PHI0+NFR-1 (fragment
+// phi = rows 16*(phi/2) + 2r + phi%2 of the tile: box phi/2, parity phi%2) and NB N boxes from
+// nbox0.  A box whose two parities both belong to the warp feeds both from one LDS.128; at an odd
+// split the middle box serves one parity per warp half.  TRI != 0: warp-uniform skips of
+// structurally zero K blocks (see a.tri).  acc[fl][nb][f2][e]: local fragment fl, N box nb,
+// N parity f2, element e.
+template <int NFR, int PHI0, int NB, int TRI>
+RS_DEVINL void mc_stage(double (&acc)[NFR][NB][2][2], const unsigned char* Ls, const unsigned char* Rs, int nbox0,
+                        int r, int kk, long long kc, int m0, int n0) {
+  constexpr int B0 = PHI0 / 2, B1 = (PHI0 + NFR - 1) / 2;  // boxes touched
   bool nlive[NB];
 #pragma unroll
   for (int nb = 0; nb < NB; ++nb) nlive[nb] = TRI != 2 || n0 + 16 * (nbox0 + nb) + 15 >= kc;
@@ -425,17 +430,20 @@ RS_DEVINL void mc_stage(double (&acc)[BH][2][NB][2][2], const unsigned char* Ls,
 #pragma unroll
     for (int nb = 0; nb < NB; ++nb) b2[nb] = *reinterpret_cast<const double2*>(Rs + (nbox0 + nb) * 2048 + off);
 #pragma unroll
-    for (int bi = 0; bi < NBOX; ++bi) {
-      const int b = mbox0 + bi;
+    for (int b = B0; b <= B1; ++b) {
       if (TRI == 1 && m0 + 16 * b + 15 < kc) continue;
       const double2 a2 = *reinterpret_cast<const double2*>(Ls + b * 2048 + off);
 #pragma unroll
-      for (int nb = 0; nb < NB; ++nb) {
-        if (TRI == 2 && !nlive[nb]) continue;
-        dmma_8x8x4(acc[bi][0][nb][0][0], acc[bi][0][nb][0][1], a2.x, b2[nb].x);
-        dmma_8x8x4(acc[bi][0][nb][1][0], acc[bi][0][nb][1][1], a2.x, b2[nb].y);
-        dmma_8x8x4(acc[bi][1][nb][0][0], acc[bi][1][nb][0][1], a2.y, b2[nb].x);
-        dmma_8x8x4(acc[bi][1][nb][1][0], acc[bi][1][nb][1][1], a2.y, b2[nb].y);
+      for (int f = 0; f < 2; ++f) {
+        const int fl = 2 * b + f - PHI0;
+        if (fl < 0 || fl >= NFR) continue;
+        const double av = f == 0 ? a2.x : a2.y;
+#pragma unroll
+        for (int nb = 0; nb < NB; ++nb) {
+          if (TRI == 2 && !nlive[nb]) continue;
+          dmma_8x8x4(acc[fl][nb][0][0], acc[fl][nb][0][1], av, b2[nb].x);
+          dmma_8x8x4(acc[fl][nb][1][0], acc[fl][nb][1][1], av, b2[nb].y);
+        }
       }
     }
   }
@@ -447,8 +455,8 @@ __global__ void __launch_bounds__(GEMM_THREADS, 1)
                    const GemmArgs a) {
   using SM = MCSmem<MFW, WM>;
   constexpr int MT = SM::MT;
-  constexpr int BH = WM == 1 ? MFW : (MFW + 1) / 2;  // M boxes per warp
-  constexpr int NB = WM == 1 ? 1 : 2;                // N boxes per warp
+  constexpr int NFR = WM == 1 ? 2 * MFW : MFW;  // 8-row M fragments per warp
+  constexpr int NB = WM == 1 ? 1 : 2;            // N boxes per warp
   extern __shared__ unsigned char smem_raw[];
   unsigned char* smem = align1024(smem_raw);
   unsigned char* sR = smem;
@@ -491,18 +499,14 @@ __global__ void __launch_bounds__(GEMM_THREADS, 1)
   const int r = lane >> 2, kk = lane & 3;
   const int wm = WM == 1 ? 0 : warp >> 2;
   const int nbox0 = WM == 1 ? warp : 2 * (warp & 3);  // first N box of this warp
-  const int mbox0 = wm * BH;                          // first M box of this warp
-  // acc[bi][f][nb][f2][e]: M fragment (box mbox0+bi, parity f), N fragment (box nbox0+nb,
-  // parity f2), element e
-  double acc[BH][2][NB][2][2];
+  const int phi0 = wm * NFR;                          // first M fragment of this warp
+  double acc[NFR][NB][2][2];
 #pragma unroll
-  for (int bi = 0; bi < BH; ++bi)
+  for (int fl = 0; fl < NFR; ++fl)
 #pragma unroll
-    for (int f = 0; f < 2; ++f)
+    for (int nb = 0; nb < NB; ++nb)
 #pragma unroll
-      for (int nb = 0; nb < NB; ++nb)
-#pragma unroll
-        for (int f2 = 0; f2 < 2; ++f2) acc[bi][f][nb][f2][0] = acc[bi][f][nb][f2][1] = 0.0;
+      for (int f2 = 0; f2 < 2; ++f2) acc[fl][nb][f2][0] = acc[fl][nb][f2][1] = 0.0;
 
   for (int it = 0; it < nk; ++it) {
     const int s = it % NSTAGE;
@@ -511,11 +515,11 @@ __global__ void __launch_bounds__(GEMM_THREADS, 1)
     const long long kc = kb + static_cast<long long>(it) * KT;  // first K of the stage
     const unsigned char* Ls = sL + s * SM::L_BYTES;
     const unsigned char* Rs = sR + s * SM::R_BYTES;
-    // compile-time box counts: the dense path has no per-box branches
+    // compile-time fragment sets: the dense path has no per-box branches
     if (WM == 1 || wm == 0)
-      mc_stage<BH, BH, NB, TRI>(acc, Ls, Rs, mbox0, nbox0, r, kk, kc, m0, n0);
+      mc_stage<NFR, 0, NB, TRI>(acc, Ls, Rs, nbox0, r, kk, kc, m0, n0);
     else
-      mc_stage<BH, MFW - BH, NB, TRI>(acc, Ls, Rs, mbox0, nbox0, r, kk, kc, m0, n0);
+      mc_stage<NFR, NFR, NB, TRI>(acc, Ls, Rs, nbox0, r, kk, kc, m0, n0);
     __syncwarp();
     if (lane == 0) mbar_arrive(&empty[s]);
   }
@@ -526,21 +530,20 @@ __global__ void __launch_bounds__(GEMM_THREADS, 1)
   const bool n_contig = o.ld_n == 1, m_contig = o.ld_m == 1;
   if (!n_contig && !m_contig) {  // generic strides: direct stores
 #pragma unroll
-    for (int bi = 0; bi < BH; ++bi)
+    for (int fl = 0; fl < NFR; ++fl) {
+      const int phi = phi0 + fl;
+      const long long gm = m0 + 16 * (phi >> 1) + 2 * r + (phi & 1);
+      if (gm >= o.m_store) continue;
 #pragma unroll
-      for (int f = 0; f < 2; ++f) {
-        const long long gm = m0 + 16 * (mbox0 + bi) + 2 * r + f;
-        if (mbox0 + bi >= MFW || gm >= o.m_store) continue;
+      for (int nb = 0; nb < NB; ++nb)
 #pragma unroll
-        for (int nb = 0; nb < NB; ++nb)
+        for (int f2 = 0; f2 < 2; ++f2)
 #pragma unroll
-          for (int f2 = 0; f2 < 2; ++f2)
-#pragma unroll
-            for (int e = 0; e < 2; ++e) {
-              const long long gn = n0 + 16 * (nbox0 + nb) + 2 * (2 * kk + e) + f2;
-              if (gn < o.n_store) gemm_put(base + gm * o.ld_m + gn * o.ld_n, acc[bi][f][nb][f2][e], o.mode);
-            }
-      }
+          for (int e = 0; e < 2; ++e) {
+            const long long gn = n0 + 16 * (nbox0 + nb) + 2 * (2 * kk + e) + f2;
+            if (gn < o.n_store) gemm_put(base + gm * o.ld_m + gn * o.ld_n, acc[fl][nb][f2][e], o.mode);
+          }
+    }
     return;
   }
   __syncthreads();  // every warp is done with the ring
@@ -548,21 +551,18 @@ __global__ void __launch_bounds__(GEMM_THREADS, 1)
   // n_contig: st[m * LDS + n] (rows along N); else st[n * LDS + m] (rows along M)
   constexpr int LDS = SM::STAGE_LD;
 #pragma unroll
-  for (int bi = 0; bi < BH; ++bi) {
-    if (mbox0 + bi >= MFW) continue;
+  for (int fl = 0; fl < NFR; ++fl) {
+    const int phi = phi0 + fl;
+    const int lm = 16 * (phi >> 1) + 2 * r + (phi & 1);
 #pragma unroll
-    for (int f = 0; f < 2; ++f) {
-      const int lm = 16 * (mbox0 + bi) + 2 * r + f;
+    for (int nb = 0; nb < NB; ++nb)
 #pragma unroll
-      for (int nb = 0; nb < NB; ++nb)
+      for (int f2 = 0; f2 < 2; ++f2)
 #pragma unroll
-        for (int f2 = 0; f2 < 2; ++f2)
-#pragma unroll
-          for (int e = 0; e < 2; ++e) {
-            const int ln = 16 * (nbox0 + nb) + 2 * (2 * kk + e) + f2;
-            st[n_contig ? lm * LDS + ln : ln * LDS + lm] = acc[bi][f][nb][f2][e];
-          }
-    }
+        for (int e = 0; e < 2; ++e) {
+          const int ln = 16 * (nbox0 + nb) + 2 * (2 * kk + e) + f2;
+          st[n_contig ? lm * LDS + ln : ln * LDS + lm] = acc[fl][nb][f2][e];
+        }
   }
   __syncthreads();
   // rows of the staged tile: n_contig -> MT rows of NT; else NT rows of MT
@@ -590,6 +590,156 @@ __global__ void __launch_bounds__(GEMM_THREADS, 1)
     } else {
       gemm_put(p, v0, o.mode);
       if (gc + 1 < col_lim) gemm_put(p + 1, v1, o.mode);
+    }
+  }
+}
+
+// ------------------------------------------------------------------------------------------
+// Persistent MC for the short-K products (K <= 128: C1 = L^{-1} C, Q1 = X R^{-1}): a CTA has
+// only ceil(K/16) stages of work per tile, so one tile per CTA leaves the TMA round trip and the
+// epilogue exposed.  Here each CTA walks tiles blockIdx.x, + gridDim.x, ...; the TMA thread keeps
+// issuing the next tile's stages into the same ring while the warps finish and store the current
+// one.  Epilogue: direct 16-byte stores of the fragment pairs adjacent along the contiguous output
+// dimension (rows 2r, 2r+1 for M-contiguous, columns 2(2kk+e), +1 for N-contiguous).
+// ------------------------------------------------------------------------------------------
+template <int MFW, int WM>
+struct MCPSmem {
+  static constexpr int MT = 16 * MFW;
+  static constexpr int R_BYTES = NT * KT * 8;
+  static constexpr int L_BYTES = MT * KT * 8;
+  static constexpr int RING = NSTAGE * (R_BYTES + L_BYTES);
+  static constexpr int TOTAL = 1024 + RING + 2 * NSTAGE * 8;
+};
+
+RS_DEVINL void put2(double* p, double v0, double v1, bool ok1, int mode) {
+  if (ok1 && (reinterpret_cast<uintptr_t>(p) & 15) == 0) {
+    double2* p2 = reinterpret_cast<double2*>(p);
+    if (mode) {
+      double2 c = *p2;
+      c.x -= v0;
+      c.y -= v1;
+      *p2 = c;
+    } else {
+      *p2 = make_double2(v0, v1);
+    }
+  } else {
+    gemm_put(p, v0, mode);
+    if (ok1) gemm_put(p + 1, v1, mode);
+  }
+}
+
+template <int MFW, int WM, int TRI>
+__global__ void __launch_bounds__(GEMM_THREADS, 1)
+    mc_persist_kernel(const __grid_constant__ CUtensorMap tmL, const __grid_constant__ CUtensorMap tmR,
+                      const GemmArgs a, int ntn, int ntiles) {
+  using SM = MCPSmem<MFW, WM>;
+  constexpr int MT = SM::MT;
+  constexpr int NFR = WM == 1 ? 2 * MFW : MFW;
+  constexpr int NB = WM == 1 ? 1 : 2;
+  extern __shared__ unsigned char smem_raw[];
+  unsigned char* smem = align1024(smem_raw);
+  unsigned char* sR = smem;
+  unsigned char* sL = sR + NSTAGE * SM::R_BYTES;
+  uint64_t* full = reinterpret_cast<uint64_t*>(smem + SM::RING);
+  uint64_t* empty = full + NSTAGE;
+  const int warp = threadIdx.x >> 5, lane = threadIdx.x & 31;
+  const int nk = static_cast<int>((a.K + KT - 1) / KT);
+  const int mytiles = blockIdx.x < ntiles ? (ntiles - blockIdx.x + gridDim.x - 1) / gridDim.x : 0;
+  const int total = mytiles * nk;
+
+  if (threadIdx.x == 0) {
+#pragma unroll
+    for (int s = 0; s < NSTAGE; ++s) {
+      mbar_init(&full[s], 1);
+      mbar_init(&empty[s], NCONS);
+    }
+    fence_mbar_init();
+  }
+  __syncthreads();
+  auto tile_of = [&](int i, int& m0, int& n0) {
+    const int T = blockIdx.x + i * gridDim.x;
+    n0 = (T % ntn) * NT;
+    m0 = (T / ntn) * MT;
+  };
+  auto issue = [&](int g) {
+    const int s = g % NSTAGE;
+    if (g >= NSTAGE) mbar_wait(&empty[s], ((g / NSTAGE) - 1) & 1);
+    int m0, n0;
+    tile_of(g / nk, m0, n0);
+    const int kc = (g % nk) * KT;
+    mbar_arrive_expect_tx(&full[s], SM::R_BYTES + SM::L_BYTES);
+#pragma unroll 1
+    for (int b = 0; b < MT / 16; ++b) tma_load_2d(sL + s * SM::L_BYTES + b * 2048, &tmL, &full[s], m0 + 16 * b, kc);
+#pragma unroll 1
+    for (int b = 0; b < NT / 16; ++b) tma_load_2d(sR + s * SM::R_BYTES + b * 2048, &tmR, &full[s], n0 + 16 * b, kc);
+  };
+  if (threadIdx.x == 0) {
+    tma_prefetch_desc(&tmL);
+    tma_prefetch_desc(&tmR);
+    for (int g = 0; g < NSTAGE - 1 && g < total; ++g) issue(g);
+  }
+  const int r = lane >> 2, kk = lane & 3;
+  const int wm = WM == 1 ? 0 : warp >> 2;
+  const int nbox0 = WM == 1 ? warp : 2 * (warp & 3);
+  const int phi0 = wm * NFR;
+  const GemmOut& o = a.out;
+  for (int i = 0; i < mytiles; ++i) {
+    int m0, n0;
+    tile_of(i, m0, n0);
+    double acc[NFR][NB][2][2];
+#pragma unroll
+    for (int fl = 0; fl < NFR; ++fl)
+#pragma unroll
+      for (int nb = 0; nb < NB; ++nb)
+#pragma unroll
+        for (int f2 = 0; f2 < 2; ++f2) acc[fl][nb][f2][0] = acc[fl][nb][f2][1] = 0.0;
+    for (int it = 0; it < nk; ++it) {
+      const int g = i * nk + it;
+      const int s = g % NSTAGE;
+      if (threadIdx.x == 0 && g + NSTAGE - 1 < total) issue(g + NSTAGE - 1);
+      mbar_wait(&full[s], (g / NSTAGE) & 1);
+      const unsigned char* Ls = sL + s * SM::L_BYTES;
+      const unsigned char* Rs = sR + s * SM::R_BYTES;
+      const long long kc = static_cast<long long>(it) * KT;
+      if (WM == 1 || wm == 0)
+        mc_stage<NFR, 0, NB, TRI>(acc, Ls, Rs, nbox0, r, kk, kc, m0, n0);
+      else
+        mc_stage<NFR, NFR, NB, TRI>(acc, Ls, Rs, nbox0, r, kk, kc, m0, n0);
+      __syncwarp();
+      if (lane == 0) mbar_arrive(&empty[s]);
+    }
+    // epilogue straight from the fragments: the parity pair (rows 2r, 2r+1 of a box) is adjacent
+    // along M, the f2 pair along N
+#pragma unroll
+    for (int fl = 0; fl < NFR; ++fl) {
+      const int phi = phi0 + fl;
+      const long long gm = m0 + 16 * (phi >> 1) + 2 * r + (phi & 1);
+#pragma unroll
+      for (int nb = 0; nb < NB; ++nb)
+#pragma unroll
+        for (int e = 0; e < 2; ++e) {
+          const long long gn0 = n0 + 16 * (nbox0 + nb) + 2 * (2 * kk + e);  // cols gn0 (f2 = 0), gn0 + 1
+          if (o.ld_m == 1 && (phi & 1) == 0 && fl + 1 < NFR) {  // pair (fl, fl + 1) along M
+#pragma unroll
+            for (int f2 = 0; f2 < 2; ++f2) {
+              const long long gn = gn0 + f2;
+              if (gn >= o.n_store || gm >= o.m_store) continue;
+              put2(o.ptr + gm + gn * o.ld_n, acc[fl][nb][f2][e], acc[fl + 1][nb][f2][e], gm + 1 < o.m_store, o.mode);
+            }
+          } else if (o.ld_m == 1 && (((phi & 1) == 1 && fl > 0))) {
+            // stored with fl - 1
+          } else if (o.ld_n == 1) {  // pair along N
+            if (gm < o.m_store && gn0 < o.n_store)
+              put2(o.ptr + gm * o.ld_m + gn0, acc[fl][nb][0][e], acc[fl][nb][1][e], gn0 + 1 < o.n_store, o.mode);
+          } else {
+#pragma unroll
+            for (int f2 = 0; f2 < 2; ++f2) {
+              const long long gn = gn0 + f2;
+              if (gm < o.m_store && gn < o.n_store)
+                gemm_put(o.ptr + gm * o.ld_m + gn * o.ld_n, acc[fl][nb][f2][e], o.mode);
+            }
+          }
+        }
     }
   }
 }

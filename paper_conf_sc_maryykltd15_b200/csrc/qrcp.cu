@@ -313,7 +313,7 @@ constexpr int QRR_ROWS = 32;               // rows per lane: l <= 128
 __global__ void __launch_bounds__(QRR_THREADS, 1)
     qrcp_reg_kernel(const double* __restrict__ B, int ldb, int ell, long long n, int k, QrWork* work, int NB,
                     int64_t* __restrict__ piv, double* __restrict__ Rho, int ldr, double* __restrict__ gaps,
-                    int* info) {
+                    int* info, long long* tbuf) {
   const int blk = blockIdx.x;
   const int tid = threadIdx.x, warp = tid >> 5, lane = tid & 31;
   const int mc = tid >> 2, q = tid & 3;
@@ -337,8 +337,11 @@ __global__ void __launch_bounds__(QRR_THREADS, 1)
 #pragma unroll
   for (int t = 0; t < QRR_ROWS; ++t) s = fma(x[t], x[t], s);
 
+#define QT(ph) \
+  if (tbuf && blk == 0 && tid == 0) tbuf[j * 8 + (ph)] = clock64();
   for (int j = 0; j < k; ++j) {
     const int par = j & 1;
+    QT(0)
     // ---- (A) CTA best / runner-up of the residual norms (s holds rows >= j) ----
     double sc = s;
     sc += __shfl_xor_sync(0xffffffffu, sc, 1);
@@ -377,7 +380,9 @@ __global__ void __launch_bounds__(QRR_THREADS, 1)
         if (i >= j && i < ell) dst[i] = x[t];
       }
     }
+    QT(1)
     grid_sync_count(&work->count, static_cast<unsigned int>(j + 1) * NB);
+    QT(2)
 
     // ---- (B) every warp scans the NB candidates (no CTA broadcast needed) ----
     Arg g{-1.0, -1, -1};
@@ -395,6 +400,7 @@ __global__ void __launch_bounds__(QRR_THREADS, 1)
       }
     }
     warp_top2(g, g2);
+    QT(3)
     const long long gidx = g.i;
     const int gblk = g.b < 0 ? 0 : g.b;
     // this warp's copy of the pivot column (rows >= j) in shared memory; alpha and
@@ -428,6 +434,7 @@ __global__ void __launch_bounds__(QRR_THREADS, 1)
       vw[i] = (i < j) ? 0.0 : (i == j ? 1.0 : (tau != 0.0 ? pv[u] / den : 0.0));
     }
     __syncwarp();
+    QT(4)
     if (blk == 0 && tid == 0) {
       if (g.i < 0 || !(g.v > 0.0)) {
         if (info) atomicCAS(info, 0, 6 /* RS_ERR_RANK_DEFICIENT */), atomicCAS(info + 1, 0, j + 1);
@@ -470,8 +477,11 @@ __global__ void __launch_bounds__(QRR_THREADS, 1)
       }
       active = false;
     }
+    QT(5)
     __syncthreads();  // s_warg reuse and candidate buffers of parity `par`
+    QT(6)
   }
+#undef QT
   if (active) {
 #pragma unroll
     for (int t = 0; t < QRR_ROWS; ++t) {
@@ -529,11 +539,10 @@ cudaError_t qrcp_truncated(cudaStream_t st, const double* B, int ldb, int ell, l
                   (void*)&gaps, (void*)&info, (void*)&tb};
   count_launch();
   if (use_reg) {
-    void* rargs[] = {(void*)&B, (void*)&ldb, (void*)&ell, (void*)&n,  (void*)&k,    (void*)&w,
-                     (void*)&NB, (void*)&piv, (void*)&Rho, (void*)&ldr, (void*)&gaps, (void*)&info};
+    void* rargs[] = {(void*)&B,   (void*)&ldb, (void*)&ell, (void*)&n,    (void*)&k,    (void*)&w, (void*)&NB,
+                     (void*)&piv, (void*)&Rho, (void*)&ldr, (void*)&gaps, (void*)&info, (void*)&tb};
     e = cudaLaunchCooperativeKernel(reinterpret_cast<void*>(qrcp_reg_kernel), dim3(NB), dim3(QRR_THREADS), rargs, 0,
                                     st);
-    tb = nullptr;
   } else {
     e = cudaLaunchCooperativeKernel(reinterpret_cast<void*>(qrcp_kernel), dim3(NB), dim3(QR_THREADS), args, smem, st);
   }
@@ -551,7 +560,7 @@ cudaError_t qrcp_truncated(cudaStream_t st, const double* B, int ldb, int ell, l
       for (int p = 0; p < 6; ++p) acc[p] += static_cast<double>(h[j * 8 + p + 1] - h[j * 8 + p]);
     for (int j = 1; j < k; ++j) acc[6] += static_cast<double>(h[j * 8] - h[(j - 1) * 8 + 6]);
     fprintf(stderr,
-            "QRCP NB=%d cols=%d cycles/step: A=%.0f barrier=%.0f scan=%.0f vload=%.0f dlarfg=%.0f update=%.0f "
+            "QRCP NB=%d cols=%d cycles/step: p0-1=%.0f p1-2=%.0f p2-3=%.0f p3-4=%.0f p4-5=%.0f p5-6=%.0f "
             "tail=%.0f\n",
             NB, cols_per, acc[0] / (k - 1), acc[1] / (k - 1), acc[2] / (k - 1), acc[3] / (k - 1), acc[4] / (k - 1),
             acc[5] / (k - 1), acc[6] / (k - 1));
