@@ -98,6 +98,15 @@ RS_DEVINL void tma_load_2d(void* smem_dst, const CUtensorMap* m, uint64_t* bar, 
       : "memory");
 }
 
+// 3-D tiled load: coordinates (c0, c1, c2), OOB -> zeros.
+RS_DEVINL void tma_load_3d(void* smem_dst, const CUtensorMap* m, uint64_t* bar, int32_t c0, int32_t c1, int32_t c2) {
+  asm volatile(
+      "cp.async.bulk.tensor.3d.shared::cluster.global.mbarrier::complete_tx::bytes [%0], [%1, {%3, %4, %5}], [%2];" ::"r"(
+          smem_u32(smem_dst)),
+      "l"(reinterpret_cast<uint64_t>(m)), "r"(smem_u32(bar)), "r"(c0), "r"(c1), "r"(c2)
+      : "memory");
+}
+
 // ---- FP64 tensor core: mma.sync m8n8k4 (lowers to DMMA.8x8x4 on sm_100a) ---------------
 // A fragment: a = A[lane/4][lane%4]; B fragment: b = B[lane%4][lane/4];
 // C/D: d0 = C[lane/4][2*(lane%4)], d1 = C[lane/4][2*(lane%4)+1].

@@ -42,6 +42,22 @@ bool make_tmap(CUtensorMap* m, const View2D& v, uint32_t box0, uint32_t box1) {
   return r == CUDA_SUCCESS;
 }
 
+// 3-D "stacked boxes" map of an MC operand (dim0 contiguous, a multiple of 16): dims {16, dim1,
+// dim0/16}, strides {ld, 16} elements, box {16, 16, nbx}: one TMA = nbx {16, 16} boxes laid out
+// back to back (see mc_load).
+bool make_tmap3(CUtensorMap* m, const View2D& v, uint32_t nbx) {
+  EncodeTiledFn enc = get_encode();
+  if (!enc || v.dim0 % 16 != 0) return false;
+  cuuint64_t dims[3] = {16, static_cast<cuuint64_t>(v.dim1), static_cast<cuuint64_t>(v.dim0 / 16)};
+  cuuint64_t strides[2] = {static_cast<cuuint64_t>(v.ld) * 8, 128};
+  cuuint32_t box[3] = {16, 16, nbx};
+  cuuint32_t estr[3] = {1, 1, 1};
+  CUresult r = enc(m, CU_TENSOR_MAP_DATA_TYPE_FLOAT64, 3, const_cast<double*>(v.base), dims, strides, box, estr,
+                   CU_TENSOR_MAP_INTERLEAVE_NONE, CU_TENSOR_MAP_SWIZZLE_128B, CU_TENSOR_MAP_L2_PROMOTION_L2_256B,
+                   CU_TENSOR_MAP_FLOAT_OOB_FILL_NONE);
+  return r == CUDA_SUCCESS;
+}
+
 template <int MFW>
 cudaError_t launch_kc_t(cudaStream_t st, dim3 grid, const CUtensorMap& tR, const CUtensorMap& tL, const GemmArgs& a) {
   constexpr int smem = KCSmem<MFW, false>::TOTAL;
@@ -127,36 +143,70 @@ cudaError_t launch_mc_wm(cudaStream_t st, dim3 grid, const CUtensorMap& tL, cons
   return cudaGetLastError();
 }
 
-template <int MFW, int WM>
-cudaError_t launch_mcp_wm(cudaStream_t st, int grid, const CUtensorMap& tL, const CUtensorMap& tR, const GemmArgs& a,
-                          int ntn, int ntiles) {
-  constexpr int smem = MCPSmem<MFW, WM>::TOTAL;
+template <int MFW>
+cudaError_t launch_mcp_t(cudaStream_t st, int grid, const CUtensorMap& tL, const CUtensorMap& tR, const GemmArgs& a,
+                         int ntn, int ntiles, int res_l) {
+  constexpr int smem = MCPSmem<MFW>::TOTAL;
   static bool attr_set = false;
   if (!attr_set) {
-    for (auto fn : {mc_persist_kernel<MFW, WM, 0>, mc_persist_kernel<MFW, WM, 1>, mc_persist_kernel<MFW, WM, 2>}) {
+    for (auto fn : {mc_persist_kernel<MFW, 0>, mc_persist_kernel<MFW, 1>, mc_persist_kernel<MFW, 2>}) {
       cudaError_t e = cudaFuncSetAttribute(fn, cudaFuncAttributeMaxDynamicSharedMemorySize, smem);
       if (e != cudaSuccess) return e;
     }
     attr_set = true;
   }
   if (a.tri == 1)
-    mc_persist_kernel<MFW, WM, 1><<<grid, GEMM_THREADS, smem, st>>>(tL, tR, a, ntn, ntiles);
+    mc_persist_kernel<MFW, 1><<<grid, GEMM_THREADS, smem, st>>>(tL, tR, a, ntn, ntiles, res_l);
   else if (a.tri == 2)
-    mc_persist_kernel<MFW, WM, 2><<<grid, GEMM_THREADS, smem, st>>>(tL, tR, a, ntn, ntiles);
+    mc_persist_kernel<MFW, 2><<<grid, GEMM_THREADS, smem, st>>>(tL, tR, a, ntn, ntiles, res_l);
   else
-    mc_persist_kernel<MFW, WM, 0><<<grid, GEMM_THREADS, smem, st>>>(tL, tR, a, ntn, ntiles);
+    mc_persist_kernel<MFW, 0><<<grid, GEMM_THREADS, smem, st>>>(tL, tR, a, ntn, ntiles, res_l);
   count_launch();
   return cudaGetLastError();
 }
 
-template <int MFW>
-cudaError_t launch_mcp_t(cudaStream_t st, int grid, const CUtensorMap& tL, const CUtensorMap& tR, const GemmArgs& a,
-                         int ntn, int ntiles) {
-  if constexpr (MFW < 3) {
-    return launch_mcp_wm<MFW, 1>(st, grid, tL, tR, a, ntn, ntiles);
-  } else {
-    return launch_mcp_wm<MFW, 2>(st, grid, tL, tR, a, ntn, ntiles);
-  }
+// N boxes of the four warp columns of the persistent kernel: identity, or -- for an upper-
+// triangular R in a single N tile (box b is live in stages 0..b, boxes past N never) -- the
+// pairing of the 8 boxes that minimises the largest pair's live stages (exhaustive over the 105
+// pairings), so no warp column sets the ring's pace alone.
+void mcp_nmap(GemmArgs& a, int N, long long K, int ntn) {
+  auto pack = [&](const int* m) {
+    a.nmap = 0;
+    for (int b = 0; b < 8; ++b) a.nmap |= static_cast<unsigned long long>(m[b]) << (8 * b);
+  };
+  const int ident[8] = {0, 1, 2, 3, 4, 5, 6, 7};
+  pack(ident);
+  if (a.tri != 2 || ntn != 1) return;
+  const int nk = static_cast<int>((K + KT - 1) / KT);
+  int w[8];
+  for (int b = 0; b < 8; ++b) w[b] = 16 * b < N ? std::min(b + 1, nk) : 0;
+  int best = 1 << 30, bestp[8] = {0, 1, 2, 3, 4, 5, 6, 7};
+  int p[8];
+  bool used[8] = {false};
+  // recursive pairing enumeration (first unused box with each later unused box)
+  auto rec = [&](auto&& self, int depth, int cur) -> void {
+    if (depth == 4) {
+      if (cur < best) {
+        best = cur;
+        for (int i = 0; i < 8; ++i) bestp[i] = p[i];
+      }
+      return;
+    }
+    int f = 0;
+    while (used[f]) ++f;
+    used[f] = true;
+    for (int s2 = f + 1; s2 < 8; ++s2) {
+      if (used[s2]) continue;
+      used[s2] = true;
+      p[2 * depth] = f;
+      p[2 * depth + 1] = s2;
+      self(self, depth + 1, std::max(cur, w[f] + w[s2]));
+      used[s2] = false;
+    }
+    used[f] = false;
+  };
+  rec(rec, 0, 0);
+  pack(bestp);
 }
 
 // Warp grid.  Dense (long-K) products: 1 x 8 -- each warp 16 columns and all M fragments.  The
@@ -309,17 +359,25 @@ cudaError_t gemm_mc(cudaStream_t st, int M, int N, long long K, const View2D& Lv
   a.tri = tri;
   const long long nsplit = (K + a.k_chunk - 1) / a.k_chunk;
   CUtensorMap tL, tR;
-  if (!make_tmap(&tL, Lv, 16, 16)) return cudaErrorInvalidValue;
-  if (!make_tmap(&tR, Rv, 16, 16)) return cudaErrorInvalidValue;
+  static const bool no3d = getenv("RS_MC_NO_TMA3D") != nullptr;  // development switch
+  a.l3d = !no3d && make_tmap3(&tL, Lv, static_cast<uint32_t>(MT / 16));
+  a.r3d = !no3d && make_tmap3(&tR, Rv, static_cast<uint32_t>(NT / 16));
+  if (!a.l3d && !make_tmap(&tL, Lv, 16, 16)) return cudaErrorInvalidValue;
+  if (!a.r3d && !make_tmap(&tR, Rv, 16, 16)) return cudaErrorInvalidValue;
   dim3 grid((N + NT - 1) / NT, (M + MT - 1) / MT, static_cast<unsigned>(nsplit < 1 ? 1 : nsplit));
   // short K and many tiles: persistent CTAs (the ring runs on across tiles)
   static const bool no_persist = getenv("RS_MC_NO_PERSIST") != nullptr;  // development switch
   const long long ntiles = static_cast<long long>(grid.x) * grid.y;
-  if (!no_persist && nsplit <= 1 && K <= 8 * KT && ntiles >= 2LL * num_sms_cached()) {
+  // (one of the two operands must be shared by every tile: a single M tile or a single N tile)
+  // (measured: at 391 tiles (m = 50 000) the resident-operand start-up costs more than it saves;
+  // at 7 813 tiles (m = 1e6) the factor's X R^-1 pair drops from 2.45 to 2.25 ms)
+  if (!no_persist && nsplit <= 1 && K <= 8 * KT && ntiles >= 8LL * num_sms_cached() && (grid.y == 1 || grid.x == 1)) {
     const int pgrid = static_cast<int>(std::min<long long>(ntiles, num_sms_cached()));
+    const int res_l = grid.y == 1 ? 1 : 0;
+    mcp_nmap(a, N, K, static_cast<int>(grid.x));
 #define RS_MCP(W) \
   case W:         \
-    return launch_mcp_t<W>(st, pgrid, tL, tR, a, static_cast<int>(grid.x), static_cast<int>(ntiles));
+    return launch_mcp_t<W>(st, pgrid, tL, tR, a, static_cast<int>(grid.x), static_cast<int>(ntiles), res_l);
     switch (mfw) {
       RS_MCP(1) RS_MCP(2) RS_MCP(3) RS_MCP(4) RS_MCP(5) RS_MCP(6) RS_MCP(7) RS_MCP(8)
       default:

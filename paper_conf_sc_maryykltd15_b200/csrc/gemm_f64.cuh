@@ -62,6 +62,8 @@ struct GemmArgs {
   int ell;               // number of Omega rows generated (rows >= ell of the tile are zero)
   int gen_mode;  // 0 = Philox + RS-BM32 (production); 1, 2 = generation-cost experiments only
   int tri;       // MC: 0 dense, 1 L lower triangular, 2 R upper triangular (zero blocks skipped)
+  unsigned long long nmap;  // persistent MC: N box of warp column wn, slot nb = byte 2 wn + nb
+  int l3d, r3d;  // MC: operand tensor map is the 3-D stacked-box form (one TMA per stage), see mc_load
 };
 
 template <int MFW, bool PHILOX>
@@ -403,6 +405,22 @@ struct MCSmem {
   static constexpr int TOTAL = 1024 + BODY + 2 * NSTAGE * 8;
 };
 
+// One stage of an MC operand (rows0 = first M or N index of the tile, nbx 16-wide boxes, K offset
+// kc).  3-D form (when the contiguous dimension is a multiple of 16): the tensor map is
+// {16, K, dim/16} with strides {ld, 16 elements} and box {16, 16, nbx}, so ONE TMA fills the
+// nbx boxes in exactly the layout of nbx separate {16, 16} 2-D boxes (box b at b * 2048 bytes,
+// 128B swizzle keyed by the K row) -- the issuing thread sits in an MMA warp, and 15 TMA issues
+// per stage measurably delayed it.  2-D form otherwise.
+RS_DEVINL void mc_load(unsigned char* dst, const CUtensorMap* tm, uint64_t* bar, bool is3d, int rows0, int nbx,
+                       int kc) {
+  if (is3d) {
+    tma_load_3d(dst, tm, bar, 0, kc, rows0 >> 4);
+  } else {
+#pragma unroll 1
+    for (int b = 0; b < nbx; ++b) tma_load_2d(dst + b * 2048, tm, bar, rows0 + 16 * b, kc);
+  }
+}
+
 // One MC pipeline stage for a warp holding the NFR 8-row M fragments PHI0 .. PHI0+NFR-1 (fragment
 // phi = rows 16*(phi/2) + 2r + phi%2 of the tile: box phi/2, parity phi%2) and NB N boxes from
 // nbox0.  A box whose two parities both belong to the warp feeds both from one LDS.128; at an odd
@@ -485,10 +503,8 @@ __global__ void __launch_bounds__(GEMM_THREADS, 1)
     if (it >= NSTAGE) mbar_wait(&empty[s], ((it / NSTAGE) - 1) & 1);
     mbar_arrive_expect_tx(&full[s], SM::R_BYTES + SM::L_BYTES);
     const int kc = static_cast<int>(kb + static_cast<long long>(it) * KT);
-#pragma unroll 1
-    for (int b = 0; b < MT / 16; ++b) tma_load_2d(sL + s * SM::L_BYTES + b * 2048, &tmL, &full[s], m0 + 16 * b, kc);
-#pragma unroll 1
-    for (int b = 0; b < NT / 16; ++b) tma_load_2d(sR + s * SM::R_BYTES + b * 2048, &tmR, &full[s], n0 + 16 * b, kc);
+    mc_load(sL + s * SM::L_BYTES, &tmL, &full[s], a.l3d, m0, MT / 16, kc);
+    mc_load(sR + s * SM::R_BYTES, &tmR, &full[s], a.r3d, n0, NT / 16, kc);
   };
   if (threadIdx.x == 0) {
     tma_prefetch_desc(&tmL);
@@ -602,13 +618,20 @@ __global__ void __launch_bounds__(GEMM_THREADS, 1)
 // one.  Epilogue: direct 16-byte stores of the fragment pairs adjacent along the contiguous output
 // dimension (rows 2r, 2r+1 for M-contiguous, columns 2(2kk+e), +1 for N-contiguous).
 // ------------------------------------------------------------------------------------------
-template <int MFW, int WM>
+// Short-K persistent layout: the operand shared by every tile (L when there is one M tile, R when
+// there is one N tile) is loaded ONCE into a resident region (all K stages, <= 8 x 16 KB); only the
+// other operand streams through a MCP_NS-deep ring, so twice the bytes are in flight per SM for
+// the same shared memory and each stage needs 8 instead of 16 TMA boxes.
+constexpr int MCP_NS = 6;
+template <int MFW>
 struct MCPSmem {
   static constexpr int MT = 16 * MFW;
-  static constexpr int R_BYTES = NT * KT * 8;
-  static constexpr int L_BYTES = MT * KT * 8;
-  static constexpr int RING = NSTAGE * (R_BYTES + L_BYTES);
-  static constexpr int TOTAL = 1024 + RING + 2 * NSTAGE * 8;
+  static constexpr int R_BYTES = NT * KT * 8;   // one K stage of R
+  static constexpr int L_BYTES = MT * KT * 8;   // one K stage of L
+  static constexpr int RES = 8 * (R_BYTES > L_BYTES ? R_BYTES : L_BYTES);  // resident operand, K <= 128
+  static constexpr int SLOT = R_BYTES > L_BYTES ? R_BYTES : L_BYTES;
+  static constexpr int RING = MCP_NS * SLOT;
+  static constexpr int TOTAL = 1024 + RES + RING + (2 * MCP_NS + 1) * 8;
 };
 
 RS_DEVINL void put2(double* p, double v0, double v1, bool ok1, int mode) {
@@ -628,31 +651,153 @@ RS_DEVINL void put2(double* p, double v0, double v1, bool ok1, int mode) {
   }
 }
 
-template <int MFW, int WM, int TRI>
+// Fragment sets of the two warp halves (wm = 0, 1) of the persistent 2 x 4 grid, as bit masks
+// over the 8-row M fragments phi = 2 * box + parity.  Dense / N-triangular products: contiguous
+// halves (the middle box split by parity at odd MFW).  M-triangular products (TRI == 1, box b is
+// live in stages 0..b): whole boxes, greedily balanced so both halves carry the same number of
+// live box-stages (MFW = 7: boxes {6, 3, 2} and {5, 4, 1, 0}, 14 each) -- with contiguous halves
+// one half would carry 40 of 56 fragment-stages and the ring would advance at its pace.
+template <int MFW, int TRI>
+struct McpFrag {
+  __host__ __device__ static constexpr unsigned mask(int wm) {
+    if (TRI != 1) {
+      unsigned m = 0;
+      for (int phi = wm * MFW; phi < (wm + 1) * MFW; ++phi) m |= 1u << phi;
+      return m;
+    }
+    unsigned m0 = 0, m1 = 0;
+    int w0 = 0, w1 = 0;
+    for (int bx = MFW - 1; bx >= 0; --bx) {
+      if (w0 <= w1) {
+        m0 |= 3u << (2 * bx);
+        w0 += bx + 1;
+      } else {
+        m1 |= 3u << (2 * bx);
+        w1 += bx + 1;
+      }
+    }
+    return wm == 0 ? m0 : m1;
+  }
+  __host__ __device__ static constexpr int count(unsigned m) {
+    int c = 0;
+    for (int i = 0; i < 32; ++i) c += (m >> i) & 1u;
+    return c;
+  }
+  __host__ __device__ static constexpr int nfr() {
+    return count(mask(0)) > count(mask(1)) ? count(mask(0)) : count(mask(1));
+  }
+  // local accumulator slot of fragment phi in mask m
+  __host__ __device__ static constexpr int slot(unsigned m, int phi) { return count(m & ((1u << phi) - 1u)); }
+};
+
+// One stage of the persistent MC kernel for a warp with compile-time fragment mask FM and the
+// two N boxes nbx[0..1] (runtime; dead boxes -- past N or triangular-zero -- are skipped).
+template <int MFW, int TRI, unsigned FM, int NFR>
+RS_DEVINL void mcp_stage(double (&acc)[NFR][2][2][2], const unsigned char* Ls, const unsigned char* Rs,
+                         const int (&nbx)[2], const bool (&nl)[2], int r, int kk, long long kc, int m0) {
+  using F = McpFrag<MFW, TRI>;
+#pragma unroll
+  for (int ks = 0; ks < KT / 4; ++ks) {
+    const uint32_t krow = 8 * (ks >> 1) + 2 * kk + (ks & 1);
+    const uint32_t off = krow * 128u + (((static_cast<uint32_t>(r) ^ krow) & 7u) << 4);
+    double2 b2[2];
+#pragma unroll
+    for (int nb = 0; nb < 2; ++nb)
+      b2[nb] = nl[nb] ? *reinterpret_cast<const double2*>(Rs + nbx[nb] * 2048 + off) : make_double2(0.0, 0.0);
+#pragma unroll
+    for (int bx = 0; bx < MFW; ++bx) {
+      if (((FM >> (2 * bx)) & 3u) == 0) continue;
+      if (TRI == 1 && m0 + 16 * bx + 15 < kc) continue;
+      const double2 a2 = *reinterpret_cast<const double2*>(Ls + bx * 2048 + off);
+#pragma unroll
+      for (int f = 0; f < 2; ++f) {
+        if (((FM >> (2 * bx + f)) & 1u) == 0) continue;
+        const int fl = F::slot(FM, 2 * bx + f);
+        const double av = f == 0 ? a2.x : a2.y;
+#pragma unroll
+        for (int nb = 0; nb < 2; ++nb) {
+          if (!nl[nb]) continue;
+          dmma_8x8x4(acc[fl][nb][0][0], acc[fl][nb][0][1], av, b2[nb].x);
+          dmma_8x8x4(acc[fl][nb][1][0], acc[fl][nb][1][1], av, b2[nb].y);
+        }
+      }
+    }
+  }
+}
+
+template <int MFW, int TRI, unsigned FM, int NFR>
+RS_DEVINL void mcp_store(const double (&acc)[NFR][2][2][2], const GemmOut& o, const int (&nbx)[2], int r, int kk,
+                         int m0, int n0) {
+  using F = McpFrag<MFW, TRI>;
+#pragma unroll
+  for (int phi = 0; phi < 2 * MFW; ++phi) {
+    if (((FM >> phi) & 1u) == 0) continue;
+    const int fl = F::slot(FM, phi);
+    const bool pair_m = (phi & 1) == 0 && ((FM >> (phi + 1)) & 1u);  // rows 2r, 2r+1 both here
+    if ((phi & 1) == 1 && ((FM >> (phi - 1)) & 1u) && o.ld_m == 1) continue;  // stored with phi - 1
+    const long long gm = m0 + 16 * (phi >> 1) + 2 * r + (phi & 1);
+#pragma unroll
+    for (int nb = 0; nb < 2; ++nb)
+#pragma unroll
+      for (int e = 0; e < 2; ++e) {
+        const long long gn0 = n0 + 16 * nbx[nb] + 2 * (2 * kk + e);  // cols gn0 (f2 = 0), gn0 + 1
+        if (o.ld_m == 1 && pair_m) {
+#pragma unroll
+          for (int f2 = 0; f2 < 2; ++f2) {
+            const long long gn = gn0 + f2;
+            if (gn >= o.n_store || gm >= o.m_store) continue;
+            put2(o.ptr + gm + gn * o.ld_n, acc[fl][nb][f2][e], acc[fl + 1][nb][f2][e], gm + 1 < o.m_store, o.mode);
+          }
+        } else if (o.ld_n == 1) {
+          if (gm < o.m_store && gn0 < o.n_store)
+            put2(o.ptr + gm * o.ld_m + gn0, acc[fl][nb][0][e], acc[fl][nb][1][e], gn0 + 1 < o.n_store, o.mode);
+        } else {
+#pragma unroll
+          for (int f2 = 0; f2 < 2; ++f2) {
+            const long long gn = gn0 + f2;
+            if (gm < o.m_store && gn < o.n_store)
+              gemm_put(o.ptr + gm * o.ld_m + gn * o.ld_n, acc[fl][nb][f2][e], o.mode);
+          }
+        }
+      }
+  }
+}
+
+// byte 2 wn + nb of a.nmap: the N box of warp column wn (identity, or balanced pairs for TRI == 2).
+// byte 2 wn + nb of a.nmap: the N box of warp column wn (identity, or balanced pairs for TRI == 2).
+// res_l = 1: L (one M tile) is the resident operand and tiles walk N; res_l = 0: R (one N tile) is
+// resident and tiles walk M.
+template <int MFW, int TRI>
 __global__ void __launch_bounds__(GEMM_THREADS, 1)
     mc_persist_kernel(const __grid_constant__ CUtensorMap tmL, const __grid_constant__ CUtensorMap tmR,
-                      const GemmArgs a, int ntn, int ntiles) {
-  using SM = MCPSmem<MFW, WM>;
+                      const GemmArgs a, int ntn, int ntiles, int res_l) {
+  using SM = MCPSmem<MFW>;
+  using F = McpFrag<MFW, TRI>;
   constexpr int MT = SM::MT;
-  constexpr int NFR = WM == 1 ? 2 * MFW : MFW;
-  constexpr int NB = WM == 1 ? 1 : 2;
+  constexpr unsigned FM0 = F::mask(0), FM1 = F::mask(1);
+  constexpr int NFR = F::nfr();
   extern __shared__ unsigned char smem_raw[];
   unsigned char* smem = align1024(smem_raw);
-  unsigned char* sR = smem;
-  unsigned char* sL = sR + NSTAGE * SM::R_BYTES;
-  uint64_t* full = reinterpret_cast<uint64_t*>(smem + SM::RING);
-  uint64_t* empty = full + NSTAGE;
+  unsigned char* sRes = smem;                 // resident operand, stage it at it * (its stage bytes)
+  unsigned char* sRing = smem + SM::RES;      // streamed operand
+  uint64_t* full = reinterpret_cast<uint64_t*>(sRing + SM::RING);
+  uint64_t* empty = full + MCP_NS;
+  uint64_t* resb = empty + MCP_NS;
   const int warp = threadIdx.x >> 5, lane = threadIdx.x & 31;
   const int nk = static_cast<int>((a.K + KT - 1) / KT);
   const int mytiles = blockIdx.x < ntiles ? (ntiles - blockIdx.x + gridDim.x - 1) / gridDim.x : 0;
   const int total = mytiles * nk;
+  const int res_bytes = res_l ? SM::L_BYTES : SM::R_BYTES;   // per stage
+  const int str_bytes = res_l ? SM::R_BYTES : SM::L_BYTES;
+  const int str_boxes = res_l ? NT / 16 : MT / 16;
 
   if (threadIdx.x == 0) {
 #pragma unroll
-    for (int s = 0; s < NSTAGE; ++s) {
+    for (int s = 0; s < MCP_NS; ++s) {
       mbar_init(&full[s], 1);
       mbar_init(&empty[s], NCONS);
     }
+    mbar_init(resb, 1);
     fence_mbar_init();
   }
   __syncthreads();
@@ -662,85 +807,73 @@ __global__ void __launch_bounds__(GEMM_THREADS, 1)
     m0 = (T / ntn) * MT;
   };
   auto issue = [&](int g) {
-    const int s = g % NSTAGE;
-    if (g >= NSTAGE) mbar_wait(&empty[s], ((g / NSTAGE) - 1) & 1);
+    const int s = g % MCP_NS;
+    if (g >= MCP_NS) mbar_wait(&empty[s], ((g / MCP_NS) - 1) & 1);
     int m0, n0;
     tile_of(g / nk, m0, n0);
     const int kc = (g % nk) * KT;
-    mbar_arrive_expect_tx(&full[s], SM::R_BYTES + SM::L_BYTES);
-#pragma unroll 1
-    for (int b = 0; b < MT / 16; ++b) tma_load_2d(sL + s * SM::L_BYTES + b * 2048, &tmL, &full[s], m0 + 16 * b, kc);
-#pragma unroll 1
-    for (int b = 0; b < NT / 16; ++b) tma_load_2d(sR + s * SM::R_BYTES + b * 2048, &tmR, &full[s], n0 + 16 * b, kc);
+    mbar_arrive_expect_tx(&full[s], str_bytes);
+    unsigned char* dst = sRing + s * SM::SLOT;
+    if (res_l)
+      mc_load(dst, &tmR, &full[s], a.r3d, n0, str_boxes, kc);
+    else
+      mc_load(dst, &tmL, &full[s], a.l3d, m0, str_boxes, kc);
   };
   if (threadIdx.x == 0) {
     tma_prefetch_desc(&tmL);
     tma_prefetch_desc(&tmR);
-    for (int g = 0; g < NSTAGE - 1 && g < total; ++g) issue(g);
+    // the resident operand: all nk stages, one barrier
+    mbar_arrive_expect_tx(resb, static_cast<uint32_t>(res_bytes * nk));
+    const int rboxes = res_l ? MT / 16 : NT / 16;
+#pragma unroll 1
+    for (int it = 0; it < nk; ++it) {
+      if (res_l)
+        mc_load(sRes + it * res_bytes, &tmL, resb, a.l3d, 0, rboxes, it * KT);
+      else
+        mc_load(sRes + it * res_bytes, &tmR, resb, a.r3d, 0, rboxes, it * KT);
+    }
+    for (int g = 0; g < MCP_NS - 1 && g < total; ++g) issue(g);
   }
+  mbar_wait(resb, 0);
   const int r = lane >> 2, kk = lane & 3;
-  const int wm = WM == 1 ? 0 : warp >> 2;
-  const int nbox0 = WM == 1 ? warp : 2 * (warp & 3);
-  const int phi0 = wm * NFR;
+  const int wm = warp >> 2, wn = warp & 3;
+  const int nbx[2] = {static_cast<int>((a.nmap >> (16 * wn)) & 0xffu), static_cast<int>((a.nmap >> (16 * wn + 8)) & 0xffu)};
   const GemmOut& o = a.out;
   for (int i = 0; i < mytiles; ++i) {
     int m0, n0;
     tile_of(i, m0, n0);
-    double acc[NFR][NB][2][2];
+    double acc[NFR][2][2][2];
 #pragma unroll
     for (int fl = 0; fl < NFR; ++fl)
 #pragma unroll
-      for (int nb = 0; nb < NB; ++nb)
+      for (int nb = 0; nb < 2; ++nb)
 #pragma unroll
         for (int f2 = 0; f2 < 2; ++f2) acc[fl][nb][f2][0] = acc[fl][nb][f2][1] = 0.0;
     for (int it = 0; it < nk; ++it) {
       const int g = i * nk + it;
-      const int s = g % NSTAGE;
-      if (threadIdx.x == 0 && g + NSTAGE - 1 < total) issue(g + NSTAGE - 1);
-      mbar_wait(&full[s], (g / NSTAGE) & 1);
-      const unsigned char* Ls = sL + s * SM::L_BYTES;
-      const unsigned char* Rs = sR + s * SM::R_BYTES;
+      const int s = g % MCP_NS;
+      if (threadIdx.x == 0 && g + MCP_NS - 1 < total) issue(g + MCP_NS - 1);
+      mbar_wait(&full[s], (g / MCP_NS) & 1);
       const long long kc = static_cast<long long>(it) * KT;
-      if (WM == 1 || wm == 0)
-        mc_stage<NFR, 0, NB, TRI>(acc, Ls, Rs, nbox0, r, kk, kc, m0, n0);
-      else
-        mc_stage<NFR, NFR, NB, TRI>(acc, Ls, Rs, nbox0, r, kk, kc, m0, n0);
+      bool nl[2];
+#pragma unroll
+      for (int nb = 0; nb < 2; ++nb)
+        nl[nb] = n0 + 16 * nbx[nb] < a.N && (TRI != 2 || n0 + 16 * nbx[nb] + 15 >= kc);
+      if (nl[0] || nl[1]) {
+        const unsigned char* Ls = res_l ? sRes + it * SM::L_BYTES : sRing + s * SM::SLOT;
+        const unsigned char* Rs = res_l ? sRing + s * SM::SLOT : sRes + it * SM::R_BYTES;
+        if (wm == 0)
+          mcp_stage<MFW, TRI, FM0, NFR>(acc, Ls, Rs, nbx, nl, r, kk, kc, m0);
+        else
+          mcp_stage<MFW, TRI, FM1, NFR>(acc, Ls, Rs, nbx, nl, r, kk, kc, m0);
+      }
       __syncwarp();
       if (lane == 0) mbar_arrive(&empty[s]);
     }
-    // epilogue straight from the fragments: the parity pair (rows 2r, 2r+1 of a box) is adjacent
-    // along M, the f2 pair along N
-#pragma unroll
-    for (int fl = 0; fl < NFR; ++fl) {
-      const int phi = phi0 + fl;
-      const long long gm = m0 + 16 * (phi >> 1) + 2 * r + (phi & 1);
-#pragma unroll
-      for (int nb = 0; nb < NB; ++nb)
-#pragma unroll
-        for (int e = 0; e < 2; ++e) {
-          const long long gn0 = n0 + 16 * (nbox0 + nb) + 2 * (2 * kk + e);  // cols gn0 (f2 = 0), gn0 + 1
-          if (o.ld_m == 1 && (phi & 1) == 0 && fl + 1 < NFR) {  // pair (fl, fl + 1) along M
-#pragma unroll
-            for (int f2 = 0; f2 < 2; ++f2) {
-              const long long gn = gn0 + f2;
-              if (gn >= o.n_store || gm >= o.m_store) continue;
-              put2(o.ptr + gm + gn * o.ld_n, acc[fl][nb][f2][e], acc[fl + 1][nb][f2][e], gm + 1 < o.m_store, o.mode);
-            }
-          } else if (o.ld_m == 1 && (((phi & 1) == 1 && fl > 0))) {
-            // stored with fl - 1
-          } else if (o.ld_n == 1) {  // pair along N
-            if (gm < o.m_store && gn0 < o.n_store)
-              put2(o.ptr + gm * o.ld_m + gn0, acc[fl][nb][0][e], acc[fl][nb][1][e], gn0 + 1 < o.n_store, o.mode);
-          } else {
-#pragma unroll
-            for (int f2 = 0; f2 < 2; ++f2) {
-              const long long gn = gn0 + f2;
-              if (gm < o.m_store && gn < o.n_store)
-                gemm_put(o.ptr + gm * o.ld_m + gn * o.ld_n, acc[fl][nb][f2][e], o.mode);
-            }
-          }
-        }
-    }
+    if (wm == 0)
+      mcp_store<MFW, TRI, FM0, NFR>(acc, o, nbx, r, kk, m0, n0);
+    else
+      mcp_store<MFW, TRI, FM1, NFR>(acc, o, nbx, r, kk, m0, n0);
   }
 }
 

@@ -323,6 +323,11 @@ __global__ void __launch_bounds__(QRR_THREADS, 1)
   __shared__ Arg s_warg[QRR_THREADS / 32];
   __shared__ double s_wsec[QRR_THREADS / 32];
   __shared__ double s_v[QRR_THREADS / 32][4 * QRR_ROWS];
+  // every CTA's candidate and its column (rows j..ell-1), staged after the barrier in ONE round
+  // trip: the pivot column no longer waits for the argmax
+  extern __shared__ double s_dyn[];
+  QrCand* s_cand = reinterpret_cast<QrCand*>(s_dyn);
+  double* s_col = s_dyn + 4 * NB;  // s_col[b * ell + (i - j)]
   QrCand* cand = reinterpret_cast<QrCand*>(work + 1);
   double* candcol = reinterpret_cast<double*>(cand + 2 * NB);
 
@@ -384,13 +389,30 @@ __global__ void __launch_bounds__(QRR_THREADS, 1)
     grid_sync_count(&work->count, static_cast<unsigned int>(j + 1) * NB);
     QT(2)
 
-    // ---- (B) every warp scans the NB candidates (no CTA broadcast needed) ----
+    // ---- (B) stage all candidates + columns, then every warp scans them in shared memory ----
+    {
+      const int len = ell - j;
+      for (int b = tid; b < NB; b += QRR_THREADS) {
+        QrCand cd;
+        cd.best = __ldcg(&cand[par * NB + b].best);
+        cd.second = __ldcg(&cand[par * NB + b].second);
+        cd.idx = __ldcg(&cand[par * NB + b].idx);
+        cd.pad = 0;
+        s_cand[b] = cd;
+      }
+      const double* cc = candcol + static_cast<size_t>(par) * NB * ell + j;
+      for (int e = tid; e < NB * len; e += QRR_THREADS) {
+        const int b = e / len, i = e - b * len;
+        s_col[b * ell + i] = __ldcg(cc + static_cast<size_t>(b) * ell + i);
+      }
+    }
+    __syncthreads();
     Arg g{-1.0, -1, -1};
     double g2 = -1.0;
     for (int b = lane; b < NB; b += 32) {
-      const long long ci = __ldcg(&cand[par * NB + b].idx);
-      const double cb = __ldcg(&cand[par * NB + b].best);
-      const double cs = __ldcg(&cand[par * NB + b].second);
+      const long long ci = s_cand[b].idx;
+      const double cb = s_cand[b].best;
+      const double cs = s_cand[b].second;
       g2 = fmax(g2, cs);
       if (better(cb, ci, g.v, g.i)) {
         if (g.i >= 0) g2 = fmax(g2, g.v);
@@ -405,14 +427,14 @@ __global__ void __launch_bounds__(QRR_THREADS, 1)
     const int gblk = g.b < 0 ? 0 : g.b;
     // this warp's copy of the pivot column (rows >= j) in shared memory; alpha and
     // xs = ||x_p[j+1:]||^2 by a warp reduction, reflector formed redundantly per warp
-    const double* src = candcol + (static_cast<size_t>(par) * NB + gblk) * ell;
+    const double* src = s_col + gblk * ell - j;  // src[i] = row i of the pivot column, i >= j
     double* vw = s_v[warp];
     double pv[QRR_ROWS / 8];
     double xs = 0.0, alpha = 0.0;
 #pragma unroll
     for (int u = 0; u < QRR_ROWS / 8; ++u) {
       const int i = lane + 32 * u;
-      pv[u] = (i >= j && i < ell) ? __ldcg(src + i) : 0.0;
+      pv[u] = (i >= j && i < ell) ? src[i] : 0.0;
       if (i > j) xs = fma(pv[u], pv[u], xs);
       if (i == j) alpha = pv[u];
     }
@@ -447,27 +469,33 @@ __global__ void __launch_bounds__(QRR_THREADS, 1)
     const bool is_piv = active && gi == gidx;
     const bool upd = active && !is_piv && tau != 0.0;
     double w = 0.0;
-    if (upd) {
+    if (upd) {  // four partial sums: a 32-term FMA chain is latency-bound
+      double w4[4] = {0.0, 0.0, 0.0, 0.0};
 #pragma unroll
-      for (int t = 0; t < QRR_ROWS; ++t) w = fma(vw[q + 4 * t], x[t], w);  // v = 0 outside rows >= j
+      for (int t = 0; t < QRR_ROWS; ++t) w4[t & 3] = fma(vw[q + 4 * t], x[t], w4[t & 3]);  // v = 0 outside rows >= j
+      w = (w4[0] + w4[1]) + (w4[2] + w4[3]);
     }
     w += __shfl_xor_sync(0xffffffffu, w, 1);
     w += __shfl_xor_sync(0xffffffffu, w, 2);
     s = 0.0;
-    if (upd) {
-      const double tw = tau * w;
+    {
+      double s4[4] = {0.0, 0.0, 0.0, 0.0};
+      if (upd) {
+        const double tw = tau * w;
 #pragma unroll
-      for (int t = 0; t < QRR_ROWS; ++t) {
-        x[t] = fma(-tw, vw[q + 4 * t], x[t]);
-        const int i = q + 4 * t;
-        if (i > j) s = fma(x[t], x[t], s);
-      }
-    } else if (active && !is_piv) {
+        for (int t = 0; t < QRR_ROWS; ++t) {
+          x[t] = fma(-tw, vw[q + 4 * t], x[t]);
+          const int i = q + 4 * t;
+          if (i > j) s4[t & 3] = fma(x[t], x[t], s4[t & 3]);
+        }
+      } else if (active && !is_piv) {
 #pragma unroll
-      for (int t = 0; t < QRR_ROWS; ++t) {
-        const int i = q + 4 * t;
-        if (i > j) s = fma(x[t], x[t], s);
+        for (int t = 0; t < QRR_ROWS; ++t) {
+          const int i = q + 4 * t;
+          if (i > j) s4[t & 3] = fma(x[t], x[t], s4[t & 3]);
+        }
       }
+      s = (s4[0] + s4[1]) + (s4[2] + s4[3]);
     }
     if (is_piv) {
 #pragma unroll
@@ -541,8 +569,15 @@ cudaError_t qrcp_truncated(cudaStream_t st, const double* B, int ldb, int ell, l
   if (use_reg) {
     void* rargs[] = {(void*)&B,   (void*)&ldb, (void*)&ell, (void*)&n,    (void*)&k,    (void*)&w, (void*)&NB,
                      (void*)&piv, (void*)&Rho, (void*)&ldr, (void*)&gaps, (void*)&info, (void*)&tb};
-    e = cudaLaunchCooperativeKernel(reinterpret_cast<void*>(qrcp_reg_kernel), dim3(NB), dim3(QRR_THREADS), rargs, 0,
-                                    st);
+    const size_t rsmem = (4 * static_cast<size_t>(NB) + static_cast<size_t>(NB) * ell) * 8;
+    static size_t rsmem_set = 0;
+    if (rsmem > rsmem_set) {
+      e = cudaFuncSetAttribute(qrcp_reg_kernel, cudaFuncAttributeMaxDynamicSharedMemorySize, static_cast<int>(rsmem));
+      if (e != cudaSuccess) return e;
+      rsmem_set = rsmem;
+    }
+    e = cudaLaunchCooperativeKernel(reinterpret_cast<void*>(qrcp_reg_kernel), dim3(NB), dim3(QRR_THREADS), rargs,
+                                    rsmem, st);
   } else {
     e = cudaLaunchCooperativeKernel(reinterpret_cast<void*>(qrcp_kernel), dim3(NB), dim3(QR_THREADS), args, smem, st);
   }

@@ -180,9 +180,59 @@ __global__ void __launch_bounds__(TRSM_WARPS * 32)
   }
 }
 
+// k <= 128: U and 1/U_ii staged once per CTA in shared memory (no division, no global reads in
+// the dependent chain); one warp per right-hand side, every lane forms x_i itself from the
+// broadcast b_i, then the lanes update b_0..b_{i-1}.
+constexpr int TRSM2_WARPS = 32;
+__global__ void __launch_bounds__(TRSM2_WARPS * 32, 1)
+    trsm_upper_cols_smem_kernel(const double* __restrict__ U, int ldu, int k, const double* __restrict__ Y,
+                                long long ldy, long long ncols, double* __restrict__ X, long long ldx) {
+  extern __shared__ double sb[];
+  double* Us = sb;               // k x k, column-major, ld k
+  double* rd = Us + k * k;       // 1 / U_ii
+  double* bw = rd + k;           // per-warp right-hand side
+  const int warp = threadIdx.x >> 5, lane = threadIdx.x & 31;
+  for (int idx = threadIdx.x; idx < k * k; idx += blockDim.x) {
+    const int i = idx % k, j = idx / k;
+    Us[idx] = i <= j ? U[i + static_cast<long long>(j) * ldu] : 0.0;
+  }
+  for (int i = threadIdx.x; i < k; i += blockDim.x) rd[i] = 1.0 / U[i + static_cast<long long>(i) * ldu];
+  __syncthreads();
+  double* b = bw + warp * k;
+  for (long long c = blockIdx.x * static_cast<long long>(TRSM2_WARPS) + warp; c < ncols;
+       c += static_cast<long long>(gridDim.x) * TRSM2_WARPS) {
+    for (int i = lane; i < k; i += 32) b[i] = Y[i + c * ldy];
+    __syncwarp();
+    for (int i = k - 1; i >= 0; --i) {
+      const double xi = b[i] * rd[i];
+      const double* ucol = Us + i * k;
+      for (int i2 = lane; i2 < i; i2 += 32) b[i2] = fma(-xi, ucol[i2], b[i2]);
+      __syncwarp();                        // every lane has read b_i
+      if (lane == (i & 31)) b[i] = xi;     // b_i is not read again before the final store
+    }
+    __syncwarp();
+    for (int i = lane; i < k; i += 32) X[i + c * ldx] = b[i];
+    __syncwarp();
+  }
+}
+
 cudaError_t trsm_upper_cols(cudaStream_t st, const double* U, int ldu, int k, const double* Y, long long ldy,
                             long long ncols, double* X, long long ldx) {
   if (ncols <= 0) return cudaSuccess;
+  if (k <= 128) {
+    const size_t smem2 = (static_cast<size_t>(k) * k + k + static_cast<size_t>(TRSM2_WARPS) * k) * 8;
+    static bool attr2 = false;
+    if (!attr2) {
+      cudaError_t e = cudaFuncSetAttribute(trsm_upper_cols_smem_kernel, cudaFuncAttributeMaxDynamicSharedMemorySize,
+                                           static_cast<int>((128 * 128 + 128 + TRSM2_WARPS * 128) * 8));
+      if (e != cudaSuccess) return e;
+      attr2 = true;
+    }
+    const int blocks = static_cast<int>(std::min<long long>((ncols + TRSM2_WARPS - 1) / TRSM2_WARPS, 148LL));
+    trsm_upper_cols_smem_kernel<<<blocks, TRSM2_WARPS * 32, smem2, st>>>(U, ldu, k, Y, ldy, ncols, X, ldx);
+    count_launch();
+    return cudaGetLastError();
+  }
   const size_t smem = static_cast<size_t>(TRSM_WARPS) * k * 8;
   if (smem > 220 * 1024) return cudaErrorInvalidValue;
   static bool attr = false;

@@ -81,13 +81,20 @@ def main():
             run_rs()
             t_rs = timed(run_rs, args.reps)
             err_rs = float(torch.linalg.norm(A[:, perm] - Q @ R) / normA)  # check only
+            rs.reset_profile(h)
+            rs.set_profiling(h, True)
+            for _ in range(args.reps):
+                run_rs()
+            torch.cuda.synchronize()
+            rs.set_profiling(h, False)
+            phases = {nm: round(v["ms"] / args.reps, 4) for nm, v in rs.get_profile(h).items() if v["launches"]}
             rs.destroy(h)
             print(json.dumps({
                 "experiment": "RS vs truncated QP3 (Fig. 7)", "m": m, "n": n, "k": k, "p": p, "q": q,
                 "law": args.law, "rs_ms": round(t_rs, 4), "qp3_ms": round(t_qp3, 4),
                 "speedup_rs_over_qp3": round(t_qp3 / t_rs, 3),
                 "qp3_GBps_trailing_reads": round(8.0 * m * sum(n - j for j in range(k)) / (t_qp3 * 1e6), 1),
-                "err_rs": err_rs, "err_qp3": res / normA}), flush=True)
+                "err_rs": err_rs, "err_qp3": res / normA, "rs_phases_ms": phases}), flush=True)
 
 
 if __name__ == "__main__":

@@ -188,6 +188,10 @@ def test_pipeline_cfg1(q):
     (4000, 500, 150, 10, 0, "exp-k"),     # l = 160 > 128: two M tiles, k > 128
     (6000, 900, 400, 10, 1, "exp-k"),     # cfg5's largest k: l = 410, four M tiles, Cholesky n > 128
     (8000, 1000, 200, 20, 2, "power"),    # cfg3 law and (k, p, q) at reduced m, n
+    # m / 128 >= 8 x 148 tiles: the short-K applies (C1 = L^-1 C, Q1 = X R^-1) run on the persistent
+    # MC kernel (resident operand, balanced triangular fragment / box sets)
+    (160000, 300, 50, 10, 1, "exp-k"),
+    (152000, 400, 100, 10, 1, "exp-k"),   # cfg2/cfg4's (k, p): l = 110, MFW 7 apply, k = 100 factor
 ])
 def test_pipeline_ragged_and_multitile(m, n, k, p, q, law):
     A, _ = make_matrix(m, n, law, k, seed=m + 3 * n)
