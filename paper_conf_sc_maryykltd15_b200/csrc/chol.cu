@@ -495,17 +495,19 @@ RS_DEVINL void chol_tile_step(CholTile<TPT, NTHR>& T, int k, int n, int npad, do
 #pragma unroll
   for (int s2 = 0; s2 < TPT; ++s2) {
     if (!T.has[s2] || 4 * T.TI[s2] + 3 <= k) continue;  // rows of the tile all finished
-    const double2* gpi = reinterpret_cast<const double2*>(&Gp[par][4 * T.TI[s2]]);
-    const double2 gi0 = gpi[0], gi1 = gpi[1];
-    const double ra[4] = {gi0.x * dinv, gi0.y * dinv, gi1.x * dinv, gi1.y * dinv};
-    const double2* src = T.kind[s2] == 0 ? reinterpret_cast<const double2*>(&Gp[par][4 * T.TJ[s2]])
-                                         : reinterpret_cast<const double2*>(&Xp[par][4 * T.TJ[s2]]);
-    const double2 c0 = src[0], c1 = src[1];
-    const double cb[4] = {c0.x, c0.y, c1.x, c1.y};
+    if (T.kind[s2] == 0 || 4 * T.TJ[s2] <= k) {          // (X(k, c) = 0 for c > k: nothing to add)
+      const double2* gpi = reinterpret_cast<const double2*>(&Gp[par][4 * T.TI[s2]]);
+      const double2 gi0 = gpi[0], gi1 = gpi[1];
+      const double ra[4] = {gi0.x * dinv, gi0.y * dinv, gi1.x * dinv, gi1.y * dinv};
+      const double2* src = T.kind[s2] == 0 ? reinterpret_cast<const double2*>(&Gp[par][4 * T.TJ[s2]])
+                                           : reinterpret_cast<const double2*>(&Xp[par][4 * T.TJ[s2]]);
+      const double2 c0 = src[0], c1 = src[1];
+      const double cb[4] = {c0.x, c0.y, c1.x, c1.y};
 #pragma unroll
-    for (int a = 0; a < 4; ++a)
+      for (int a = 0; a < 4; ++a)
 #pragma unroll
-      for (int bb = 0; bb < 4; ++bb) T.v[s2][a][bb] = fma(-ra[a], cb[bb], T.v[s2][a][bb]);
+        for (int bb = 0; bb < 4; ++bb) T.v[s2][a][bb] = fma(-ra[a], cb[bb], T.v[s2][a][bb]);
+    }
     if (T.TI[s2] == ipub) {  // publish row k + 1 = tile row A1
       const int c = 4 * T.TJ[s2];
       if (T.kind[s2] == 0) {
@@ -615,7 +617,11 @@ cudaError_t chol_inv(cudaStream_t st, const double* G, int ldg, int n, int npad,
   static const bool use_tile = getenv("RS_CHOL_BLOCKED") == nullptr;  // development switch
   if (use_tile && n <= CT_MAXN) {
     const int nt = (n + 3) / 4;
-    if (nt * (nt + 1) <= 1024)  // one tile per thread (n <= 124)
+    static const int tpt = [] {  // RS_CHOL_TPT=2: development switch (two tiles per thread)
+      const char* v = getenv("RS_CHOL_TPT");
+      return v ? atoi(v) : 1;
+    }();
+    if (tpt == 1 && nt * (nt + 1) <= 1024)  // one tile per thread (n <= 124)
       chol_tile_kernel<1, 1024><<<1, 1024, 0, st>>>(G, ldg, n, R, ldr, Linv, ldl, info, info_code, npad);
     else
       chol_tile_kernel<2, 576><<<1, 576, 0, st>>>(G, ldg, n, R, ldr, Linv, ldl, info, info_code, npad);

@@ -61,6 +61,18 @@ bool make_tmap3(CUtensorMap* m, const View2D& v, uint32_t nbx) {
 template <int MFW>
 cudaError_t launch_kc_t(cudaStream_t st, dim3 grid, const CUtensorMap& tR, const CUtensorMap& tL, const GemmArgs& a) {
   constexpr int smem = KCSmem<MFW, false>::TOTAL;
+  static const bool pwg = getenv("RS_KC_PWG") != nullptr;  // development switch: producer warpgroup
+  if (pwg) {
+    static bool attr_p = false;
+    if (!attr_p) {
+      cudaError_t e = cudaFuncSetAttribute(kc_gemm_pwg_kernel<MFW>, cudaFuncAttributeMaxDynamicSharedMemorySize, smem);
+      if (e != cudaSuccess) return e;
+      attr_p = true;
+    }
+    kc_gemm_pwg_kernel<MFW><<<grid, KCP_THREADS, smem, st>>>(tR, tL, a);
+    count_launch();
+    return cudaGetLastError();
+  }
   static bool attr_set = false;  // per-instantiation; races are benign (idempotent)
   if (!attr_set) {
     cudaError_t e = cudaFuncSetAttribute(kc_gemm_kernel<MFW>, cudaFuncAttributeMaxDynamicSharedMemorySize, smem);

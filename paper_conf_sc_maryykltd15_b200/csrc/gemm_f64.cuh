@@ -212,6 +212,86 @@ __global__ void __launch_bounds__(GEMM_THREADS, 1)
   kc_store<MFW>(acc, a.out, m0, n0, wn, kk, rowL);
 }
 
+// KC with a dedicated producer warpgroup (warps 8-11; one thread issues, setmaxnreg moves their
+// registers to the MMA warps): the MMA warps never wait on the ring's "empty" barriers, so no
+// MMA warp is coupled to the slowest one at every stage.
+constexpr int KCP_THREADS = GEMM_THREADS + 128;
+constexpr int MCP_PROD_REGS = 40;
+constexpr int MCP_MMA_REGS = 232;  // 4*32*40 + 8*32*232 = 64512 <= 65536
+template <int MFW>
+__global__ void __launch_bounds__(KCP_THREADS, 1)
+    kc_gemm_pwg_kernel(const __grid_constant__ CUtensorMap tmR, const __grid_constant__ CUtensorMap tmL,
+                       const GemmArgs a) {
+  using SM = KCSmem<MFW, false>;
+  constexpr int MT = SM::MT;
+  extern __shared__ unsigned char smem_raw[];
+  unsigned char* smem = align1024(smem_raw);
+  unsigned char* sR = smem;
+  unsigned char* sL = sR + SM::NS * SM::R_BYTES;
+  uint64_t* full = reinterpret_cast<uint64_t*>(sL + SM::NS * SM::L_BYTES);
+  uint64_t* empty = full + SM::NS;
+
+  const int warp = threadIdx.x >> 5, lane = threadIdx.x & 31;
+  const int n0 = blockIdx.x * NT, m0 = blockIdx.y * MT;
+  const long long kb = static_cast<long long>(blockIdx.z) * a.k_chunk;
+  const long long ke = min(a.K, kb + a.k_chunk);
+  const int nk = kb < ke ? static_cast<int>((ke - kb + KT - 1) / KT) : 0;
+
+  if (threadIdx.x == 0) {
+#pragma unroll
+    for (int s = 0; s < SM::NS; ++s) {
+      mbar_init(&full[s], 1);
+      mbar_init(&empty[s], NCONS);
+    }
+    fence_mbar_init();
+  }
+  __syncthreads();
+  if (warp >= NCONS) {
+    asm volatile("setmaxnreg.dec.sync.aligned.u32 %0;\n" ::"n"(MCP_PROD_REGS));
+    if (warp == NCONS && lane == 0) {
+      tma_prefetch_desc(&tmR);
+      tma_prefetch_desc(&tmL);
+      for (int it = 0; it < nk; ++it) {
+        const int s = it % SM::NS;
+        if (it >= SM::NS) mbar_wait(&empty[s], ((it / SM::NS) - 1) & 1);
+        mbar_arrive_expect_tx(&full[s], SM::R_BYTES + SM::L_BYTES_TMA);
+        const int kc = static_cast<int>(kb + static_cast<long long>(it) * KT);
+        tma_load_2d(sR + s * SM::R_BYTES, &tmR, &full[s], kc, n0);
+        tma_load_2d(sL + s * SM::L_BYTES, &tmL, &full[s], kc, m0);
+      }
+    }
+    return;
+  }
+  asm volatile("setmaxnreg.inc.sync.aligned.u32 %0;\n" ::"n"(MCP_MMA_REGS));
+  const int wm = warp >> 2, wn = warp & 3;
+  const int r = lane >> 2, kk = lane & 3;
+  double acc[MFW][4][2];
+#pragma unroll
+  for (int mf = 0; mf < MFW; ++mf)
+#pragma unroll
+    for (int nf = 0; nf < 4; ++nf) acc[mf][nf][0] = acc[mf][nf][1] = 0.0;
+  auto rowL = [&](int mf) {
+    const int mg = wm * MFW + mf;
+    return kc_row(mg >> 1, mg & 1, r);
+  };
+  auto rowR = [&](int nf) {
+    const int ng = wn * 4 + nf;
+    return kc_row(ng >> 1, ng & 1, r);
+  };
+  for (int it = 0; it < nk; ++it) {
+    const int s = it % SM::NS;
+    mbar_wait(&full[s], (it / SM::NS) & 1);
+    const unsigned char* Ls = sL + s * SM::L_BYTES;
+    const unsigned char* Rs = sR + s * SM::R_BYTES;
+    kc_stage_mma<MFW>(
+        acc, [&](int mf, int p) { return *reinterpret_cast<const double2*>(Ls + kc_pair_off(rowL(mf), p, kk)); },
+        [&](int nf, int p) { return *reinterpret_cast<const double2*>(Rs + kc_pair_off(rowR(nf), p, kk)); });
+    __syncwarp();
+    if (lane == 0) mbar_arrive(&empty[s]);
+  }
+  kc_store<MFW>(acc, a.out, m0, n0, wn, kk, rowL);
+}
+
 // ------------------------------------------------------------------------------------------
 // KC family with Omega generated in the tile loader, warp-specialised: warpgroup 0 (4 warps,
 // one per SM sub-partition) runs Philox + RS-BM32 on the INT/FP32 pipes and issues the TMA

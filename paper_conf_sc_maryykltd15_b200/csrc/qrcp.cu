@@ -519,6 +519,246 @@ __global__ void __launch_bounds__(QRR_THREADS, 1)
   }
 }
 
+// ------------------------------------------------------------------------------------------
+// Cluster variant (n <= 16 CTAs x COLS columns, l <= 4 ROWS): the CTAs of ONE thread-block
+// cluster hold the columns in registers as above, and each step's exchange runs through
+// distributed shared memory: every CTA pushes its candidate and candidate column (rows j..l-1)
+// into every peer's shared memory (st.shared::cluster), one cluster barrier, then every CTA
+// scans the NB candidates and forms the reflector from local shared memory.  No global-memory
+// round trips in the step at all (the grid-barrier kernel above pays several per step).
+// ------------------------------------------------------------------------------------------
+constexpr int QRC_MAXNB = 16;
+
+template <int ROWS, int THREADS>
+__global__ void __launch_bounds__(THREADS, 1)
+    qrcp_cluster_kernel(const double* __restrict__ B, int ldb, int ell, long long n, int k, int cols_per,
+                        int64_t* __restrict__ piv, double* __restrict__ Rho, int ldr, double* __restrict__ gaps,
+                        int* info) {
+  constexpr int WARPS = THREADS / 32;
+  const uint32_t blk = cluster_ctarank();
+  const int NB = static_cast<int>(gridDim.x);
+  const int tid = threadIdx.x, warp = tid >> 5, lane = tid & 31;
+  const int mc = tid >> 2, q = tid & 3;
+  const long long c0 = static_cast<long long>(blk) * cols_per;
+  const long long gi = c0 + mc;
+  bool active = mc < cols_per && gi < n;
+  __shared__ Arg s_warg[WARPS];
+  __shared__ double s_wsec[WARPS];
+  __shared__ __align__(16) double s_v[WARPS][4 * ROWS];
+  __shared__ __align__(16) QrCand s_cand[2][QRC_MAXNB];
+  __shared__ __align__(16) double s_stage[4 * ROWS];
+  extern __shared__ __align__(16) double s_dynq[];  // s_col[2][QRC_MAXNB][4 ROWS]
+  double (*s_col)[QRC_MAXNB][4 * ROWS] = reinterpret_cast<double (*)[QRC_MAXNB][4 * ROWS]>(s_dynq);
+
+  double x[ROWS];
+#pragma unroll
+  for (int t = 0; t < ROWS; ++t) {
+    const int i = q + 4 * t;
+    x[t] = (active && i < ell) ? B[i + gi * static_cast<long long>(ldb)] : 0.0;
+  }
+  double s = 0.0;
+  {
+    double s4[4] = {0.0, 0.0, 0.0, 0.0};
+#pragma unroll
+    for (int t = 0; t < ROWS; ++t) s4[t & 3] = fma(x[t], x[t], s4[t & 3]);
+    s = (s4[0] + s4[1]) + (s4[2] + s4[3]);
+  }
+  cluster_sync_all();  // peers' shared memory exists before anyone writes into it
+
+  for (int j = 0; j < k; ++j) {
+    const int par = j & 1;
+    // ---- (A) CTA best / runner-up ----
+    double sc = s;
+    sc += __shfl_xor_sync(0xffffffffu, sc, 1);
+    sc += __shfl_xor_sync(0xffffffffu, sc, 2);
+    {
+      Arg a = (active && q == 0) ? Arg{sc, gi, mc} : Arg{-1.0, -1, -1};
+      double sec = -1.0;
+      warp_top2(a, sec);
+      if (lane == 0) {
+        s_warg[warp] = a;
+        s_wsec[warp] = sec;
+      }
+      __syncthreads();
+      if (warp == 0) {
+        Arg xx = lane < WARPS ? s_warg[lane] : Arg{-1.0, -1, -1};
+        double xs = lane < WARPS ? s_wsec[lane] : -1.0;
+        warp_top2(xx, xs);
+        if (lane == 0) {
+          s_warg[0] = xx;
+          s_wsec[0] = xs;
+        }
+      }
+      __syncthreads();
+    }
+    // the owner stages its rows j..ell-1 locally, then everyone pushes candidate + column to all peers
+    const Arg mine = s_warg[0];
+    if (active && mine.i == gi) {
+#pragma unroll
+      for (int t = 0; t < ROWS; ++t) {
+        const int i = q + 4 * t;
+        if (i >= j && i < ell) s_stage[i] = x[t];
+      }
+    }
+    __syncthreads();
+    {
+      const int len = ell - j;
+      const uint32_t col_base = smem_u32(&s_col[par][blk][0]);
+      for (int e = tid; e < NB * len; e += THREADS) {
+        const int pc = e / len, i = j + (e - pc * len);
+        const uint32_t ra = mapa_shared(col_base + 8u * i, static_cast<uint32_t>(pc));
+        asm volatile("st.shared::cluster.f64 [%0], %1;" ::"r"(ra), "d"(s_stage[i]) : "memory");
+      }
+      if (tid < NB) {
+        const uint32_t cb = mapa_shared(smem_u32(&s_cand[par][blk]), static_cast<uint32_t>(tid));
+        const long long idx = mine.i;
+        asm volatile("st.shared::cluster.v2.f64 [%0], {%1, %2};" ::"r"(cb), "d"(mine.v), "d"(s_wsec[0]) : "memory");
+        asm volatile("st.shared::cluster.s64 [%0], %1;" ::"r"(cb + 16u), "l"(idx) : "memory");
+      }
+    }
+    cluster_sync_all();
+
+    // ---- (B) every warp scans the NB candidates in local shared memory ----
+    Arg g{-1.0, -1, -1};
+    double g2 = -1.0;
+    for (int b = lane; b < NB; b += 32) {
+      const long long ci = s_cand[par][b].idx;
+      const double cb = s_cand[par][b].best;
+      const double cs = s_cand[par][b].second;
+      g2 = fmax(g2, cs);
+      if (better(cb, ci, g.v, g.i)) {
+        if (g.i >= 0) g2 = fmax(g2, g.v);
+        g = Arg{cb, ci, b};
+      } else if (ci >= 0) {
+        g2 = fmax(g2, cb);
+      }
+    }
+    warp_top2(g, g2);
+    const long long gidx = g.i;
+    const int gblk = g.b < 0 ? 0 : g.b;
+    const double* src = &s_col[par][gblk][0];
+    double* vw = s_v[warp];
+    double pv[ROWS / 8];
+    double xs = 0.0, alpha = 0.0;
+#pragma unroll
+    for (int u = 0; u < ROWS / 8; ++u) {
+      const int i = lane + 32 * u;
+      pv[u] = (i >= j && i < ell) ? src[i] : 0.0;
+      if (i > j) xs = fma(pv[u], pv[u], xs);
+      if (i == j) alpha = pv[u];
+    }
+#pragma unroll
+    for (int o = 16; o > 0; o >>= 1) {
+      xs += __shfl_xor_sync(0xffffffffu, xs, o);
+      alpha += __shfl_xor_sync(0xffffffffu, alpha, o);
+    }
+    double tau = 0.0, beta = alpha;
+    if (g.i >= 0 && xs > 0.0) {
+      const double h = sqrt(fma(alpha, alpha, xs));
+      beta = alpha >= 0.0 ? -h : h;
+      tau = (beta - alpha) / beta;
+    }
+    const double den = alpha - beta;
+#pragma unroll
+    for (int u = 0; u < ROWS / 8; ++u) {
+      const int i = lane + 32 * u;
+      vw[i] = (i < j) ? 0.0 : (i == j ? 1.0 : (tau != 0.0 ? pv[u] / den : 0.0));
+    }
+    __syncwarp();
+    if (blk == 0 && tid == 0) {
+      if (g.i < 0 || !(g.v > 0.0)) {
+        if (info) atomicCAS(info, 0, 6 /* RS_ERR_RANK_DEFICIENT */), atomicCAS(info + 1, 0, j + 1);
+      }
+      piv[j] = gidx;
+      const double nb = sqrt(fmax(g.v, 0.0)), ns = sqrt(fmax(g2, 0.0));
+      if (gaps) gaps[j] = nb > 0.0 ? (nb - ns) / nb : 0.0;
+    }
+    // ---- apply H = I - tau v v^T; retire the pivot column; fuse the next residual norm ----
+    const bool is_piv = active && gi == gidx;
+    const bool upd = active && !is_piv && tau != 0.0;
+    double w = 0.0;
+    if (upd) {
+      double w4[4] = {0.0, 0.0, 0.0, 0.0};
+#pragma unroll
+      for (int t = 0; t < ROWS; ++t) w4[t & 3] = fma(vw[q + 4 * t], x[t], w4[t & 3]);
+      w = (w4[0] + w4[1]) + (w4[2] + w4[3]);
+    }
+    w += __shfl_xor_sync(0xffffffffu, w, 1);
+    w += __shfl_xor_sync(0xffffffffu, w, 2);
+    {
+      double s4[4] = {0.0, 0.0, 0.0, 0.0};
+      if (upd) {
+        const double tw = tau * w;
+#pragma unroll
+        for (int t = 0; t < ROWS; ++t) {
+          x[t] = fma(-tw, vw[q + 4 * t], x[t]);
+          const int i = q + 4 * t;
+          if (i > j) s4[t & 3] = fma(x[t], x[t], s4[t & 3]);
+        }
+      } else if (active && !is_piv) {
+#pragma unroll
+        for (int t = 0; t < ROWS; ++t) {
+          const int i = q + 4 * t;
+          if (i > j) s4[t & 3] = fma(x[t], x[t], s4[t & 3]);
+        }
+      }
+      s = (s4[0] + s4[1]) + (s4[2] + s4[3]);
+    }
+    if (is_piv) {
+#pragma unroll
+      for (int t = 0; t < ROWS; ++t) {
+        const int i = q + 4 * t;
+        if (i < k) Rho[i + gi * static_cast<long long>(ldr)] = (i < j) ? x[t] : (i == j ? beta : 0.0);
+      }
+      active = false;
+    }
+    __syncthreads();  // s_warg / s_stage reuse
+  }
+  if (active) {
+#pragma unroll
+    for (int t = 0; t < ROWS; ++t) {
+      const int i = q + 4 * t;
+      if (i < k) Rho[i + gi * static_cast<long long>(ldr)] = x[t];
+    }
+  }
+  cluster_sync_all();  // no CTA leaves while peers may still write its shared memory
+}
+
+template <int ROWS, int THREADS>
+cudaError_t launch_qrcp_cluster(cudaStream_t st, int NB, const double* B, int ldb, int ell, long long n, int k,
+                                int cols_per, int64_t* piv, double* Rho, int ldr, double* gaps, int* info) {
+  constexpr int dsmem = 2 * QRC_MAXNB * 4 * ROWS * 8;
+  static bool attr = false;
+  if (!attr) {
+    cudaError_t e = cudaFuncSetAttribute(qrcp_cluster_kernel<ROWS, THREADS>,
+                                         cudaFuncAttributeNonPortableClusterSizeAllowed, 1);
+    if (e != cudaSuccess) return e;
+    e = cudaFuncSetAttribute(qrcp_cluster_kernel<ROWS, THREADS>, cudaFuncAttributeMaxDynamicSharedMemorySize, dsmem);
+    if (e != cudaSuccess) return e;
+    attr = true;
+  }
+  cudaLaunchConfig_t cfg{};
+  cfg.gridDim = dim3(NB, 1, 1);
+  cfg.blockDim = dim3(THREADS, 1, 1);
+  cfg.dynamicSmemBytes = dsmem;
+  cfg.stream = st;
+  cudaLaunchAttribute at[1];
+  at[0].id = cudaLaunchAttributeClusterDimension;
+  at[0].val.clusterDim.x = NB;
+  at[0].val.clusterDim.y = 1;
+  at[0].val.clusterDim.z = 1;
+  cfg.attrs = at;
+  cfg.numAttrs = 1;
+  int nclusters = 0;
+  cudaError_t e = cudaOccupancyMaxActiveClusters(&nclusters, qrcp_cluster_kernel<ROWS, THREADS>, &cfg);
+  if (e != cudaSuccess || nclusters < 1) {
+    cudaGetLastError();
+    return cudaErrorNotSupported;
+  }
+  return cudaLaunchKernelEx(&cfg, qrcp_cluster_kernel<ROWS, THREADS>, B, ldb, ell, n, k, cols_per, piv, Rho, ldr,
+                            gaps, info);
+}
+
 namespace {
 int qr_ldw(int ell) { return (ell + 11) / 16 * 16 + 4; }  // >= ell, = 4 mod 16 doubles
 size_t qr_smem(int cols, int ell) { return (static_cast<size_t>(cols) * qr_ldw(ell) + ell) * 8; }
@@ -550,9 +790,33 @@ cudaError_t qrcp_truncated(cudaStream_t st, const double* B, int ldb, int ell, l
     if (e != cudaSuccess) return e;
     attr = true;
   }
+  QrWork* w = static_cast<QrWork*>(work);
+  {
+    // cluster path: l <= 64 with <= 160 columns per CTA, or l <= 128 with <= 128, over <= 16 CTAs
+    static const bool no_cluster = getenv("RS_QRCP_NO_CLUSTER") != nullptr;  // development switch
+    const int rows = ell <= 64 ? 16 : 32;
+    const int maxc = rows == 16 ? 160 : 128;
+    const int nbc = static_cast<int>((n + maxc - 1) / maxc);
+    if (!no_cluster && !force_smem && ell <= 128 && nbc <= QRC_MAXNB) {
+      const int cp = static_cast<int>((n + nbc - 1) / nbc);
+      int64_t* pv = reinterpret_cast<int64_t*>(reinterpret_cast<double*>(reinterpret_cast<QrCand*>(w + 1) + 2 * nbc) +
+                                               2 * static_cast<size_t>(nbc) * ell);
+      cudaError_t ec = rows == 16
+                           ? launch_qrcp_cluster<16, 640>(st, nbc, B, ldb, ell, n, k, cp, pv, Rho, ldr, gaps, info)
+                           : launch_qrcp_cluster<32, 512>(st, nbc, B, ldb, ell, n, k, cp, pv, Rho, ldr, gaps, info);
+      if (ec == cudaSuccess) {
+        count_launch();
+        const size_t psmem = static_cast<size_t>(n) * 8;
+        const bool use_smem = psmem <= QR_SMEM_MAX;
+        qrcp_perm_kernel<<<1, 1024, use_smem ? psmem : 0, st>>>(pv, k, n, perm, pv + n, use_smem);
+        count_launch();
+        return cudaGetLastError();
+      }
+      if (ec != cudaErrorNotSupported) return ec;
+    }
+  }
   cudaError_t e = cudaMemsetAsync(work, 0, sizeof(QrWork), st);
   if (e != cudaSuccess) return e;
-  QrWork* w = static_cast<QrWork*>(work);
   QrCand* cand = reinterpret_cast<QrCand*>(w + 1);
   double* candcol = reinterpret_cast<double*>(cand + 2 * NB);
   int64_t* piv = reinterpret_cast<int64_t*>(candcol + 2 * static_cast<size_t>(NB) * ell);
