@@ -71,19 +71,40 @@ RS_DEVINL Arg shfl_arg(const Arg& a, int o) {
   return Arg{__shfl_xor_sync(0xffffffffu, a.v, o), __shfl_xor_sync(0xffffffffu, a.i, o),
              __shfl_xor_sync(0xffffffffu, a.b, o)};
 }
-// warp-wide best and runner-up (value only) of per-lane (best a, runner-up sec)
+// warp-wide best and runner-up (value only) of per-lane (best a, runner-up sec), on REDUX.SYNC:
+// squared norms are >= 0, and non-negative doubles order like their bit patterns, so the argmax
+// is a 64-bit unsigned max taken as (hi word, then lo word among the hi winners), then the lowest
+// original index among the lanes holding that key (ties -> lowest index, as `better`).  Keys are
+// bits + 1 so a valid 0.0 beats "none" (i < 0 / sec < 0, key 0).  7 warp-wide ops instead of 5
+// dependent levels of 7 shuffles plus divergent compares.
+RS_DEVINL unsigned long long top2_key(bool has, double v) {
+  return has ? static_cast<unsigned long long>(__double_as_longlong(v + 0.0)) + 1ull : 0ull;  // -0 -> +0
+}
+RS_DEVINL unsigned long long warp_max_u64(unsigned long long k) {
+  const unsigned hi = static_cast<unsigned>(k >> 32), lo = static_cast<unsigned>(k);
+  const unsigned mhi = __reduce_max_sync(0xffffffffu, hi);
+  const unsigned mlo = __reduce_max_sync(0xffffffffu, hi == mhi ? lo : 0u);
+  return (static_cast<unsigned long long>(mhi) << 32) | mlo;
+}
 RS_DEVINL void warp_top2(Arg& a, double& sec) {
-#pragma unroll
-  for (int o = 16; o > 0; o >>= 1) {
-    const Arg x = shfl_arg(a, o);
-    const double xs = __shfl_xor_sync(0xffffffffu, sec, o);
-    sec = fmax(sec, xs);
-    if (better(x.v, x.i, a.v, a.i)) {
-      if (a.i >= 0) sec = fmax(sec, a.v);
-      a = x;
-    } else if (x.i >= 0) {
-      sec = fmax(sec, x.v);
-    }
+  const bool has = a.i >= 0;
+  const unsigned long long key = top2_key(has, a.v);
+  const unsigned long long mk = warp_max_u64(key);
+  const bool top = has && key == mk;
+  const unsigned mi = __reduce_min_sync(0xffffffffu, top ? static_cast<unsigned>(a.i) : 0xffffffffu);
+  const unsigned win = __ballot_sync(0xffffffffu, top && static_cast<unsigned>(a.i) == mi);
+  const bool me = (win >> (threadIdx.x & 31)) & 1u;
+  // runner-up: every lane's own runner-up and every non-winning lane's best
+  const unsigned long long k2 = max(top2_key(sec >= 0.0, sec), me ? 0ull : key);
+  const unsigned long long m2 = warp_max_u64(k2);
+  sec = m2 ? __longlong_as_double(static_cast<long long>(m2 - 1ull)) : -1.0;
+  if (win) {
+    const int src = __ffs(win) - 1;
+    a.b = __shfl_sync(0xffffffffu, a.b, src);
+    a.v = __longlong_as_double(static_cast<long long>(mk - 1ull));
+    a.i = static_cast<long long>(mi);
+  } else {
+    a = Arg{-1.0, -1, -1};
   }
 }
 
@@ -390,20 +411,40 @@ __global__ void __launch_bounds__(QRR_THREADS, 1)
     QT(2)
 
     // ---- (B) stage all candidates + columns, then every warp scans them in shared memory ----
+    // one flat copy of the NB published columns (rows < j are stale and never read), issued as
+    // batches of independent loads so the step pays about one L2 round trip, not one per element
     {
-      const int len = ell - j;
-      for (int b = tid; b < NB; b += QRR_THREADS) {
-        QrCand cd;
+      constexpr int U = 12;
+      const double* cc = candcol + static_cast<size_t>(par) * NB * ell;
+      const int tot = NB * ell;
+      QrCand cd;
+      const bool mine = tid < NB;
+      if (mine) {
+        cd.best = __ldcg(&cand[par * NB + tid].best);
+        cd.second = __ldcg(&cand[par * NB + tid].second);
+        cd.idx = __ldcg(&cand[par * NB + tid].idx);
+        cd.pad = 0;
+      }
+      for (int e0 = 0; e0 < tot; e0 += U * QRR_THREADS) {
+        double v[U];
+#pragma unroll
+        for (int u = 0; u < U; ++u) {
+          const int e = e0 + u * QRR_THREADS + tid;
+          v[u] = e < tot ? __ldcg(cc + e) : 0.0;
+        }
+#pragma unroll
+        for (int u = 0; u < U; ++u) {
+          const int e = e0 + u * QRR_THREADS + tid;
+          if (e < tot) s_col[e] = v[u];
+        }
+      }
+      if (mine) s_cand[tid] = cd;
+      for (int b = tid + QRR_THREADS; b < NB; b += QRR_THREADS) {  // NB <= 148 < QRR_THREADS: unused
         cd.best = __ldcg(&cand[par * NB + b].best);
         cd.second = __ldcg(&cand[par * NB + b].second);
         cd.idx = __ldcg(&cand[par * NB + b].idx);
         cd.pad = 0;
         s_cand[b] = cd;
-      }
-      const double* cc = candcol + static_cast<size_t>(par) * NB * ell + j;
-      for (int e = tid; e < NB * len; e += QRR_THREADS) {
-        const int b = e / len, i = e - b * len;
-        s_col[b * ell + i] = __ldcg(cc + static_cast<size_t>(b) * ell + i);
       }
     }
     __syncthreads();
@@ -427,7 +468,7 @@ __global__ void __launch_bounds__(QRR_THREADS, 1)
     const int gblk = g.b < 0 ? 0 : g.b;
     // this warp's copy of the pivot column (rows >= j) in shared memory; alpha and
     // xs = ||x_p[j+1:]||^2 by a warp reduction, reflector formed redundantly per warp
-    const double* src = s_col + gblk * ell - j;  // src[i] = row i of the pivot column, i >= j
+    const double* src = s_col + gblk * ell;  // src[i] = row i of the pivot column, i >= j
     double* vw = s_v[warp];
     double pv[QRR_ROWS / 8];
     double xs = 0.0, alpha = 0.0;
@@ -449,11 +490,13 @@ __global__ void __launch_bounds__(QRR_THREADS, 1)
       beta = alpha >= 0.0 ? -h : h;
       tau = (beta - alpha) / beta;
     }
-    const double den = alpha - beta;
+    // v = x / (alpha - beta) as x * (1 / (alpha - beta)): one division on the step's critical path
+    // instead of QRR_ROWS / 8 (differs from the quotient by <= 1 ulp per entry)
+    const double rden = tau != 0.0 ? 1.0 / (alpha - beta) : 0.0;
 #pragma unroll
     for (int u = 0; u < QRR_ROWS / 8; ++u) {
       const int i = lane + 32 * u;
-      vw[i] = (i < j) ? 0.0 : (i == j ? 1.0 : (tau != 0.0 ? pv[u] / den : 0.0));
+      vw[i] = (i < j) ? 0.0 : (i == j ? 1.0 : pv[u] * rden);
     }
     __syncwarp();
     QT(4)
@@ -771,6 +814,7 @@ size_t qrcp_workspace_bytes(int ell, long long n) {
 
 cudaError_t qrcp_truncated(cudaStream_t st, const double* B, int ldb, int ell, long long n, int k, void* work,
                            int64_t* perm, double* Rho, int ldr, double* gaps, int* info, int num_sms) {
+  if (n >= (1LL << 31)) return cudaErrorInvalidValue;  // column indices ride in 32-bit REDUX keys
   static const bool force_smem = getenv("RS_QRCP_SMEM") != nullptr;  // development switch
   const bool use_reg = !force_smem && ell <= 4 * QRR_ROWS && (n + QRR_COLS - 1) / QRR_COLS <= num_sms;
   int cols_per = use_reg ? QRR_COLS : QR_MAX_COLS;
