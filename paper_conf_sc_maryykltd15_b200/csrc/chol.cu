@@ -477,30 +477,51 @@ struct CholTile {
   bool has[TPT];
 };
 
+// Published rows are kept for the whole factorisation in shared memory, packed: row k of G from
+// column 4(k/4) on (the columns any live tile can read), row k of X's accumulators up to column
+// 4(k/4) + 3.  Nothing is written to global memory inside the pivot loop; R and Linv are written
+// once at the end from the packed rows and the per-pivot 1/sqrt(d_k) (coalesced, all threads).
+RS_DEVINL int ct_gofs(int k, int np) {
+  const int b = k >> 2, r = k & 3;
+  return 4 * np * b - 8 * b * (b - 1) + r * (np - 4 * b);
+}
+RS_DEVINL int ct_xofs(int k) {
+  const int b = k >> 2, r = k & 3;
+  return 8 * b * (b + 1) + r * 4 * (b + 1);
+}
+// packed shared memory (doubles) for an np x np problem
+__host__ __device__ constexpr int ct_smem_doubles(int np) {
+  return (4 * np * (np / 4) - 8 * (np / 4) * (np / 4 - 1)) + 8 * (np / 4) * (np / 4 + 1) + np + 8;
+}
+
 // one pivot step k with (k + 1) % 4 == A1 (the tile row that holds row k + 1)
 template <int A1, int TPT, int NTHR>
-RS_DEVINL void chol_tile_step(CholTile<TPT, NTHR>& T, int k, int n, int npad, double (*Gp)[CT_MAXN],
-                              double (*Xp)[CT_MAXN], double* __restrict__ R, int ldr, double* __restrict__ Linv,
-                              int ldl, int* info, int code) {
+RS_DEVINL void chol_tile_step(CholTile<TPT, NTHR>& T, int k, int n, int np, double* Gs, double* Xs, double* s_ri,
+                              int* info, int code) {
   const int tid = threadIdx.x;
-  const int par = k & 1;
-  double d = Gp[par][k];
+  const int k4 = 4 * (k >> 2);
+  const double* Gk = Gs + ct_gofs(k, np) - k4;  // Gk[c] = G(k, c), c >= 4 (k / 4)
+  const double* Xk = Xs + ct_xofs(k);           // Xk[c] = acc(k, c), c < 4 (k / 4) + 4
+  double d = Gk[k];
   if (!(d > 0.0)) {
     if (tid == 0 && info && k < n) atomicCAS(info, 0, code), atomicCAS(info + 1, 0, k + 1);
     d = 1.0;
   }
   const double ri = rsqrt(d);
   const double dinv = ri * ri;
+  if (tid == 0) s_ri[k] = ri;
   const int ipub = (k + 1) >> 2;  // tile row block holding row k + 1
+  double* Gn = Gs + ct_gofs(k + 1, np) - 4 * ipub;
+  double* Xn = Xs + ct_xofs(k + 1);
 #pragma unroll
   for (int s2 = 0; s2 < TPT; ++s2) {
     if (!T.has[s2] || 4 * T.TI[s2] + 3 <= k) continue;  // rows of the tile all finished
     if (T.kind[s2] == 0 || 4 * T.TJ[s2] <= k) {          // (X(k, c) = 0 for c > k: nothing to add)
-      const double2* gpi = reinterpret_cast<const double2*>(&Gp[par][4 * T.TI[s2]]);
+      const double2* gpi = reinterpret_cast<const double2*>(&Gk[4 * T.TI[s2]]);
       const double2 gi0 = gpi[0], gi1 = gpi[1];
       const double ra[4] = {gi0.x * dinv, gi0.y * dinv, gi1.x * dinv, gi1.y * dinv};
-      const double2* src = T.kind[s2] == 0 ? reinterpret_cast<const double2*>(&Gp[par][4 * T.TJ[s2]])
-                                           : reinterpret_cast<const double2*>(&Xp[par][4 * T.TJ[s2]]);
+      const double2* src = T.kind[s2] == 0 ? reinterpret_cast<const double2*>(&Gk[4 * T.TJ[s2]])
+                                           : reinterpret_cast<const double2*>(&Xk[4 * T.TJ[s2]]);
       const double2 c0 = src[0], c1 = src[1];
       const double cb[4] = {c0.x, c0.y, c1.x, c1.y};
 #pragma unroll
@@ -508,32 +529,18 @@ RS_DEVINL void chol_tile_step(CholTile<TPT, NTHR>& T, int k, int n, int npad, do
 #pragma unroll
         for (int bb = 0; bb < 4; ++bb) T.v[s2][a][bb] = fma(-ra[a], cb[bb], T.v[s2][a][bb]);
     }
-    if (T.TI[s2] == ipub) {  // publish row k + 1 = tile row A1
+    if (T.TI[s2] == ipub && k + 1 < np) {  // publish row k + 1 = tile row A1
       const int c = 4 * T.TJ[s2];
       if (T.kind[s2] == 0) {
-        reinterpret_cast<double2*>(&Gp[par ^ 1][c])[0] = make_double2(T.v[s2][A1][0], T.v[s2][A1][1]);
-        reinterpret_cast<double2*>(&Gp[par ^ 1][c])[1] = make_double2(T.v[s2][A1][2], T.v[s2][A1][3]);
+        reinterpret_cast<double2*>(&Gn[c])[0] = make_double2(T.v[s2][A1][0], T.v[s2][A1][1]);
+        reinterpret_cast<double2*>(&Gn[c])[1] = make_double2(T.v[s2][A1][2], T.v[s2][A1][3]);
       } else {
         const int lim = k + 1 - c;  // X(k + 1, c + bb) = 0 for c + bb > k + 1
-        reinterpret_cast<double2*>(&Xp[par ^ 1][c])[0] =
+        reinterpret_cast<double2*>(&Xn[c])[0] =
             make_double2(lim >= 0 ? T.v[s2][A1][0] : 0.0, lim >= 1 ? T.v[s2][A1][1] : 0.0);
-        reinterpret_cast<double2*>(&Xp[par ^ 1][c])[1] =
+        reinterpret_cast<double2*>(&Xn[c])[1] =
             make_double2(lim >= 2 ? T.v[s2][A1][2] : 0.0, lim >= 3 ? T.v[s2][A1][3] : 0.0);
       }
-    }
-  }
-  // row k of R and of Linv = R^{-T}
-  if (k < n) {
-    for (int t = tid; t < npad; t += NTHR) {
-      double rv = 0.0, lv = 0.0;
-      if (t < n) {
-        if (t > k) rv = Gp[par][t] * ri;
-        else if (t == k) rv = d * ri;
-        if (t < k) lv = Xp[par][t] * ri;
-        else if (t == k) lv = ri;
-      }
-      R[k + static_cast<long long>(t) * ldr] = rv;
-      Linv[k + static_cast<long long>(t) * ldl] = lv;
     }
   }
   __syncthreads();
@@ -543,11 +550,13 @@ template <int TPT, int NTHR>
 __global__ void __launch_bounds__(NTHR, 1)
     chol_tile_kernel(const double* __restrict__ G, int ldg, int n, double* __restrict__ R, int ldr,
                      double* __restrict__ Linv, int ldl, int* info, int code, int npad) {
-  __shared__ __align__(16) double Gp[2][CT_MAXN];
-  __shared__ __align__(16) double Xp[2][CT_MAXN];
+  extern __shared__ __align__(16) double ct_smem[];
   const int tid = threadIdx.x;
   const int np = (n + 3) / 4 * 4;
   const int nt = np / 4;  // tile blocks per dimension
+  double* Gs = ct_smem;
+  double* Xs = Gs + ct_gofs(np, np);
+  double* s_ri = Xs + ct_xofs(np);
   CholTile<TPT, NTHR> T;
 #pragma unroll
   for (int s2 = 0; s2 < TPT; ++s2) {
@@ -583,26 +592,28 @@ __global__ void __launch_bounds__(NTHR, 1)
         T.v[s2][a][bb] = x;
       }
   }
-  // row 0; X's rows are published only up to the publishing tile's last column, so both X
-  // buffers start at zero (X(k, c) = 0 for c > k must read as zero)
-  for (int j = tid; j < CT_MAXN; j += NTHR) {
-    Gp[0][j] = j < np ? ((j < n) ? G[static_cast<long long>(j) * ldg] : (j == 0 ? 1.0 : 0.0)) : 0.0;
-    Gp[1][j] = 0.0;
-    Xp[0][j] = j == 0 ? 1.0 : 0.0;
-    Xp[1][j] = 0.0;
-  }
+  // row 0 of G (identity-padded past n) and of X's accumulators (e_0)
+  for (int j = tid; j < np; j += NTHR) Gs[j] = (j < n) ? G[static_cast<long long>(j) * ldg] : (j == 0 ? 1.0 : 0.0);
+  if (tid < 4) Xs[tid] = tid == 0 ? 1.0 : 0.0;
   __syncthreads();
   for (int k = 0; k < np; k += 4) {  // np is a multiple of 4
-    chol_tile_step<1>(T, k, n, npad, Gp, Xp, R, ldr, Linv, ldl, info, code);
-    chol_tile_step<2>(T, k + 1, n, npad, Gp, Xp, R, ldr, Linv, ldl, info, code);
-    chol_tile_step<3>(T, k + 2, n, npad, Gp, Xp, R, ldr, Linv, ldl, info, code);
-    chol_tile_step<0>(T, k + 3, n, npad, Gp, Xp, R, ldr, Linv, ldl, info, code);
+    chol_tile_step<1>(T, k, n, np, Gs, Xs, s_ri, info, code);
+    chol_tile_step<2>(T, k + 1, n, np, Gs, Xs, s_ri, info, code);
+    chol_tile_step<3>(T, k + 2, n, np, Gs, Xs, s_ri, info, code);
+    chol_tile_step<0>(T, k + 3, n, np, Gs, Xs, s_ri, info, code);
   }
-  // zero padding rows n..npad-1
-  for (int idx = tid; idx < (npad - n) * npad; idx += NTHR) {
-    const int kk = n + idx / npad, t = idx % npad;
-    R[kk + static_cast<long long>(t) * ldr] = 0.0;
-    Linv[kk + static_cast<long long>(t) * ldl] = 0.0;
+  // R(k, t) = G(k, t) / sqrt(d_k) (t >= k), Linv(k, t) = acc(k, t) / sqrt(d_k) (t <= k), zero
+  // elsewhere and in the padding; consecutive threads take consecutive rows (column-major)
+  for (int idx = tid; idx < npad * npad; idx += NTHR) {
+    const int kk = idx % npad, t = idx / npad;
+    double rv = 0.0, lv = 0.0;
+    if (kk < n && t < n) {
+      const double ri = s_ri[kk];
+      if (t >= kk) rv = Gs[ct_gofs(kk, np) - 4 * (kk >> 2) + t] * ri;
+      if (t <= kk) lv = Xs[ct_xofs(kk) + t] * ri;
+    }
+    R[kk + static_cast<long long>(t) * ldr] = rv;
+    Linv[kk + static_cast<long long>(t) * ldl] = lv;
   }
 }
 
@@ -621,10 +632,21 @@ cudaError_t chol_inv(cudaStream_t st, const double* G, int ldg, int n, int npad,
       const char* v = getenv("RS_CHOL_TPT");
       return v ? atoi(v) : 1;
     }();
+    static bool attr_t = false;
+    constexpr int ct_max_smem = ct_smem_doubles(CT_MAXN) * 8;
+    if (!attr_t) {
+      cudaError_t e = cudaFuncSetAttribute(chol_tile_kernel<1, 1024>, cudaFuncAttributeMaxDynamicSharedMemorySize,
+                                           ct_max_smem);
+      if (e == cudaSuccess)
+        e = cudaFuncSetAttribute(chol_tile_kernel<2, 576>, cudaFuncAttributeMaxDynamicSharedMemorySize, ct_max_smem);
+      if (e != cudaSuccess) return e;
+      attr_t = true;
+    }
+    const size_t ct_smem = static_cast<size_t>(ct_smem_doubles(4 * nt)) * 8;
     if (tpt == 1 && nt * (nt + 1) <= 1024)  // one tile per thread (n <= 124)
-      chol_tile_kernel<1, 1024><<<1, 1024, 0, st>>>(G, ldg, n, R, ldr, Linv, ldl, info, info_code, npad);
+      chol_tile_kernel<1, 1024><<<1, 1024, ct_smem, st>>>(G, ldg, n, R, ldr, Linv, ldl, info, info_code, npad);
     else
-      chol_tile_kernel<2, 576><<<1, 576, 0, st>>>(G, ldg, n, R, ldr, Linv, ldl, info, info_code, npad);
+      chol_tile_kernel<2, 576><<<1, 576, ct_smem, st>>>(G, ldg, n, R, ldr, Linv, ldl, info, info_code, npad);
   } else if (n <= smem_max_n && n <= CH_SMEM_MAX_N) {
     const int np = (n + CB - 1) / CB * CB;
     const size_t smem = static_cast<size_t>(np) * (np + 1) * 8;

@@ -563,6 +563,250 @@ __global__ void __launch_bounds__(QRR_THREADS, 1)
 }
 
 // ------------------------------------------------------------------------------------------
+// Flag-synchronised variant of the register kernel (the default for l <= 128, n <= 148 x COLS).
+// No grid barrier and no bulk staging: per step each CTA publishes ONE record -- its best column's
+// squared norm, the runner-up, the index, and the dlarfg reflector of that column (beta, tau,
+// 1 / (alpha - beta), formed by the column's owner lanes BEFORE the exchange, off the critical
+// path of every other CTA) -- written with a release store of the sequence number j + 1 last.
+// Every CTA acquires the NB records (one L2 round trip after the last publication), picks the
+// same global pivot (largest norm, ties -> lowest original index), and each warp reads only the
+// winning column and its reflector (a second, small round trip).  LPC lanes own one column (rows
+// q + LPC t): LPC = 8 halves the FP64 FMA work per SM of the trailing update when n <= 148 x 64.
+// Records and columns are double-buffered by step parity: a CTA can only overwrite slot `par`
+// at step j + 2 after every CTA has published step j + 1, i.e. finished reading step j.
+// ------------------------------------------------------------------------------------------
+struct QrRec {
+  double best;             // squared residual norm of the CTA's best active column (-1 if none)
+  double second;           // runner-up in the CTA (-1 if none)
+  long long idx;           // original column index (-1 if none)
+  unsigned long long seq;  // j + 1 once the record of step j (and its column) is published
+};
+constexpr int QRF_CST = 132;  // published column stride: rows 0..127, then beta, tau, 1/(alpha - beta)
+constexpr int QRF_MAXNB = 148;
+
+RS_DEVINL unsigned long long ld_acquire_u64(const unsigned long long* p) {
+  unsigned long long v;
+  asm volatile("ld.acquire.gpu.global.u64 %0, [%1];" : "=l"(v) : "l"(p) : "memory");
+  return v;
+}
+RS_DEVINL void st_release_u64(unsigned long long* p, unsigned long long v) {
+  asm volatile("st.release.gpu.global.u64 [%0], %1;" ::"l"(p), "l"(v) : "memory");
+}
+
+template <int LPC>
+__global__ void __launch_bounds__(QRR_THREADS, 1)
+    qrcp_flag_kernel(const double* __restrict__ B, int ldb, int ell, long long n, int k, QrRec* rec,
+                     double* candcol, int NB, int64_t* __restrict__ piv, double* __restrict__ Rho, int ldr,
+                     double* __restrict__ gaps, int* info, long long* tbuf, unsigned int* counter) {
+  constexpr int COLS = QRR_THREADS / LPC;
+  constexpr int RPL = 128 / LPC;  // rows per lane (l <= 128)
+  constexpr int NW = QRR_THREADS / 32;
+  const int blk = blockIdx.x;
+  const int tid = threadIdx.x, warp = tid >> 5, lane = tid & 31;
+  const int mc = tid / LPC, q = tid % LPC;
+  const unsigned gmask = ((1u << LPC) - 1u) << (lane & ~(LPC - 1));  // my column's lanes
+  const long long gi = static_cast<long long>(blk) * COLS + mc;
+  bool active = gi < n;
+  __shared__ Arg s_warg[NW];
+  __shared__ double s_wsec[NW];
+  __shared__ QrRec s_rec[QRF_MAXNB];
+  __shared__ double s_v[NW][128];
+
+  double x[RPL];
+#pragma unroll
+  for (int t = 0; t < RPL; ++t) {
+    const int i = q + LPC * t;
+    x[t] = (active && i < ell) ? B[i + gi * static_cast<long long>(ldb)] : 0.0;
+  }
+  double s = 0.0;  // residual norm^2 (my rows) over rows >= j
+#pragma unroll
+  for (int t = 0; t < RPL; ++t) s = fma(x[t], x[t], s);
+
+#define QT(ph) \
+  if (tbuf && blk == 0 && tid == 0) tbuf[j * 8 + (ph)] = clock64();
+  for (int j = 0; j < k; ++j) {
+    const int par = j & 1;
+    QT(0)
+    // ---- (A) CTA best / runner-up, the winner's owner lanes publish column + reflector ----
+    double sc = s;
+#pragma unroll
+    for (int o = 1; o < LPC; o <<= 1) sc += __shfl_xor_sync(0xffffffffu, sc, o);
+    {
+      Arg a = (active && q == 0) ? Arg{sc, gi, mc} : Arg{-1.0, -1, -1};
+      double sec = -1.0;
+      warp_top2(a, sec);
+      if (lane == 0) {
+        s_warg[warp] = a;
+        s_wsec[warp] = sec;
+      }
+    }
+    __syncthreads();
+    if (warp == 0) {
+      Arg xx = lane < NW ? s_warg[lane] : Arg{-1.0, -1, -1};
+      double xs = lane < NW ? s_wsec[lane] : -1.0;
+      warp_top2(xx, xs);
+      __syncwarp();
+      if (lane == 0) {
+        s_warg[0] = xx;
+        s_wsec[0] = xs;
+      }
+    }
+    __syncthreads();
+    QT(1)
+    {
+      const Arg cw = s_warg[0];
+      QrRec* myrec = rec + par * NB + blk;
+      if (cw.i < 0) {  // nothing left in this CTA: publish an empty record
+        if (tid == 0) {
+          myrec->best = -1.0;
+          myrec->second = s_wsec[0];
+          myrec->idx = -1;
+          if (!counter) st_release_u64(&myrec->seq, static_cast<unsigned long long>(j + 1));
+        }
+      } else if (active && cw.i == gi) {
+        double* dst = candcol + (static_cast<size_t>(par) * NB + blk) * QRF_CST;
+        double ap = 0.0, xp = 0.0;
+#pragma unroll
+        for (int t = 0; t < RPL; ++t) {
+          const int i = q + LPC * t;
+          if (i >= j && i < ell) dst[i] = x[t];
+          if (i == j) ap = x[t];
+          if (i > j) xp = fma(x[t], x[t], xp);
+        }
+#pragma unroll
+        for (int o = 1; o < LPC; o <<= 1) {
+          ap += __shfl_xor_sync(gmask, ap, o);  // one nonzero term
+          xp += __shfl_xor_sync(gmask, xp, o);
+        }
+        __syncwarp(gmask);  // the group's column stores are ordered before the release below
+        if (q == 0) {
+          double beta = ap, tau = 0.0, rden = 0.0;
+          if (xp > 0.0) {  // dlarfg: H = I when the part below the diagonal is zero
+            const double h = sqrt(fma(ap, ap, xp));
+            beta = ap >= 0.0 ? -h : h;
+            tau = (beta - ap) / beta;
+            rden = 1.0 / (ap - beta);
+          }
+          dst[128] = beta;
+          dst[129] = tau;
+          dst[130] = rden;
+          myrec->best = cw.v;
+          myrec->second = s_wsec[0];
+          myrec->idx = cw.i;
+          if (!counter) st_release_u64(&myrec->seq, static_cast<unsigned long long>(j + 1));
+        }
+      }
+    }
+    // ---- (B) acquire every CTA's record of step j, pick the global pivot ----
+    // counter != NULL: one grid barrier (one poller per CTA) instead of NB pollers per CTA
+    if (counter) grid_sync_count(counter, static_cast<unsigned int>(j + 1) * NB);
+    if (tid < NB) {
+      const QrRec* r = rec + par * NB + tid;
+      if (!counter)
+        while (ld_acquire_u64(&r->seq) < static_cast<unsigned long long>(j + 1)) {
+        }
+      QrRec cd;
+      cd.best = __ldcg(&r->best);
+      cd.second = __ldcg(&r->second);
+      cd.idx = __ldcg(&r->idx);
+      cd.seq = 0;
+      s_rec[tid] = cd;
+    }
+    __syncthreads();
+    QT(2)
+    Arg g{-1.0, -1, -1};
+    double g2 = -1.0;
+    for (int b = lane; b < NB; b += 32) {
+      const long long ci = s_rec[b].idx;
+      const double cb = s_rec[b].best;
+      g2 = fmax(g2, s_rec[b].second);
+      if (better(cb, ci, g.v, g.i)) {
+        if (g.i >= 0) g2 = fmax(g2, g.v);
+        g = Arg{cb, ci, b};
+      } else if (ci >= 0) {
+        g2 = fmax(g2, cb);
+      }
+    }
+    warp_top2(g, g2);
+    QT(3)
+    // ---- the winner's column (rows >= j) and reflector, straight from L2, per warp ----
+    const double* src = candcol + (static_cast<size_t>(par) * NB + (g.b < 0 ? 0 : g.b)) * QRF_CST;
+    double pv[4];
+#pragma unroll
+    for (int u = 0; u < 4; ++u) {
+      const int i = lane + 32 * u;
+      pv[u] = (g.i >= 0 && i >= j && i < ell) ? __ldcg(src + i) : 0.0;
+    }
+    const double beta = g.i >= 0 ? __ldcg(src + 128) : 0.0;
+    const double tau = g.i >= 0 ? __ldcg(src + 129) : 0.0;
+    const double rden = g.i >= 0 ? __ldcg(src + 130) : 0.0;
+    double* vw = s_v[warp];
+#pragma unroll
+    for (int u = 0; u < 4; ++u) {
+      const int i = lane + 32 * u;
+      vw[i] = (i < j) ? 0.0 : (i == j ? 1.0 : pv[u] * rden);
+    }
+    __syncwarp();
+    QT(4)
+    const long long gidx = g.i;
+    if (blk == 0 && tid == 0) {
+      if (g.i < 0 || !(g.v > 0.0)) {
+        if (info) atomicCAS(info, 0, 6 /* RS_ERR_RANK_DEFICIENT */), atomicCAS(info + 1, 0, j + 1);
+      }
+      piv[j] = gidx;
+      const double nb = sqrt(fmax(g.v, 0.0)), ns = sqrt(fmax(g2, 0.0));
+      if (gaps) gaps[j] = nb > 0.0 ? (nb - ns) / nb : 0.0;
+    }
+    // ---- apply H = I - tau v v^T; retire the pivot column; fuse the next residual norm ----
+    const bool is_piv = active && gi == gidx;
+    const bool upd = active && !is_piv && tau != 0.0;
+    double w = 0.0;
+    if (upd) {
+      double w4[4] = {0.0, 0.0, 0.0, 0.0};
+#pragma unroll
+      for (int t = 0; t < RPL; ++t) w4[t & 3] = fma(vw[q + LPC * t], x[t], w4[t & 3]);
+      w = (w4[0] + w4[1]) + (w4[2] + w4[3]);
+    }
+#pragma unroll
+    for (int o = 1; o < LPC; o <<= 1) w += __shfl_xor_sync(0xffffffffu, w, o);
+    {
+      double s4[4] = {0.0, 0.0, 0.0, 0.0};
+      if (upd) {
+        const double tw = tau * w;
+#pragma unroll
+        for (int t = 0; t < RPL; ++t) {
+          x[t] = fma(-tw, vw[q + LPC * t], x[t]);
+          if (q + LPC * t > j) s4[t & 3] = fma(x[t], x[t], s4[t & 3]);
+        }
+      } else if (active && !is_piv) {
+#pragma unroll
+        for (int t = 0; t < RPL; ++t)
+          if (q + LPC * t > j) s4[t & 3] = fma(x[t], x[t], s4[t & 3]);
+      }
+      s = (s4[0] + s4[1]) + (s4[2] + s4[3]);
+    }
+    if (is_piv) {
+#pragma unroll
+      for (int t = 0; t < RPL; ++t) {
+        const int i = q + LPC * t;
+        if (i < k) Rho[i + gi * static_cast<long long>(ldr)] = (i < j) ? x[t] : (i == j ? beta : 0.0);
+      }
+      active = false;
+    }
+    QT(5)
+    QT(6)
+  }
+#undef QT
+  if (active) {
+#pragma unroll
+    for (int t = 0; t < RPL; ++t) {
+      const int i = q + LPC * t;
+      if (i < k) Rho[i + gi * static_cast<long long>(ldr)] = x[t];
+    }
+  }
+}
+
+// ------------------------------------------------------------------------------------------
 // Cluster variant (n <= 16 CTAs x COLS columns, l <= 4 ROWS): the CTAs of ONE thread-block
 // cluster hold the columns in registers as above, and each step's exchange runs through
 // distributed shared memory: every CTA pushes its candidate and candidate column (rows j..l-1)
@@ -809,7 +1053,9 @@ size_t qr_smem(int cols, int ell) { return (static_cast<size_t>(cols) * qr_ldw(e
 
 size_t qrcp_workspace_bytes(int ell, long long n) {
   const int NB = 1024;  // upper bound on blocks
-  return sizeof(QrWork) + 2 * NB * sizeof(QrCand) + 2 * static_cast<size_t>(NB) * ell * 8 + 2 * n * 8 + 256;
+  // the flag kernel uses QrRec records and QRF_CST-strided columns in the same region
+  return sizeof(QrWork) + 2 * NB * sizeof(QrCand) + 2 * static_cast<size_t>(NB) * std::max(ell, QRF_CST) * 8 +
+         2 * n * 8 + 256;
 }
 
 cudaError_t qrcp_truncated(cudaStream_t st, const double* B, int ldb, int ell, long long n, int k, void* work,
@@ -859,17 +1105,65 @@ cudaError_t qrcp_truncated(cudaStream_t st, const double* B, int ldb, int ell, l
       if (ec != cudaErrorNotSupported) return ec;
     }
   }
+  // RS_QRCP_TIMING=1: per-phase cycle counts of CTA 0 printed to stderr (development aid)
+  static long long* tbuf = nullptr;
+  static const bool timing = getenv("RS_QRCP_TIMING") != nullptr;
+  if (timing && !tbuf && cudaMalloc(&tbuf, 8 * 8 * 1024) != cudaSuccess) tbuf = nullptr;
+  long long* tb = (timing && k <= 1024) ? tbuf : nullptr;
+  auto report = [&](const char* what, int nb, int cols) {
+    if (!tb) return;
+    static long long h[8 * 1024];
+    cudaStreamSynchronize(st);
+    cudaMemcpy(h, tb, 8 * 8 * static_cast<size_t>(k), cudaMemcpyDeviceToHost);
+    double acc[7] = {0};
+    for (int j = 1; j < k; ++j)
+      for (int p = 0; p < 6; ++p) acc[p] += static_cast<double>(h[j * 8 + p + 1] - h[j * 8 + p]);
+    for (int j = 1; j < k; ++j) acc[6] += static_cast<double>(h[j * 8] - h[(j - 1) * 8 + 6]);
+    fprintf(stderr,
+            "QRCP %s NB=%d cols=%d cycles/step: p0-1=%.0f p1-2=%.0f p2-3=%.0f p3-4=%.0f p4-5=%.0f p5-6=%.0f "
+            "tail=%.0f\n",
+            what, nb, cols, acc[0] / (k - 1), acc[1] / (k - 1), acc[2] / (k - 1), acc[3] / (k - 1), acc[4] / (k - 1),
+            acc[5] / (k - 1), acc[6] / (k - 1));
+  };
+  {
+    // flag-synchronised register kernel: 8 lanes per column when n <= NBmax x 64, else 4
+    static const bool barrier_kernel = getenv("RS_QRCP_BARRIER") != nullptr;  // development switch
+    const int nbmax = std::min(num_sms, QRF_MAXNB);
+    const int nb8 = static_cast<int>((n + 63) / 64), nb4 = static_cast<int>((n + 127) / 128);
+    static const bool force4 = getenv("RS_QRCP_LPC4") != nullptr;  // development switch
+    const int lpc = (nb8 <= nbmax && !force4) ? 8 : (nb4 <= nbmax ? 4 : 0);
+    if (!barrier_kernel && !force_smem && ell <= 128 && lpc) {
+      const int nbf = lpc == 8 ? nb8 : nb4;
+      QrRec* rec = reinterpret_cast<QrRec*>(w + 1);
+      double* ccol = reinterpret_cast<double*>(rec + 2 * nbf);
+      int64_t* pv = reinterpret_cast<int64_t*>(ccol + 2 * static_cast<size_t>(nbf) * QRF_CST);
+      cudaError_t e = cudaMemsetAsync(work, 0, sizeof(QrWork) + 2 * static_cast<size_t>(nbf) * sizeof(QrRec), st);
+      if (e != cudaSuccess) return e;
+      static const bool poll_records = getenv("RS_QRCP_POLL") != nullptr;  // development switch
+      unsigned int* counter = poll_records ? nullptr : &w->count;
+      void* fargs[] = {(void*)&B,   (void*)&ldb, (void*)&ell, (void*)&n,   (void*)&k,    (void*)&rec,
+                       (void*)&ccol, (void*)&nbf, (void*)&pv, (void*)&Rho, (void*)&ldr, (void*)&gaps,
+                       (void*)&info, (void*)&tb, (void*)&counter};
+      e = lpc == 8 ? cudaLaunchCooperativeKernel(reinterpret_cast<void*>(qrcp_flag_kernel<8>), dim3(nbf),
+                                                 dim3(QRR_THREADS), fargs, 0, st)
+                   : cudaLaunchCooperativeKernel(reinterpret_cast<void*>(qrcp_flag_kernel<4>), dim3(nbf),
+                                                 dim3(QRR_THREADS), fargs, 0, st);
+      if (e != cudaSuccess) return e;
+      count_launch();
+      const size_t psmem = static_cast<size_t>(n) * 8;
+      const bool use_smem = psmem <= QR_SMEM_MAX;
+      qrcp_perm_kernel<<<1, 1024, use_smem ? psmem : 0, st>>>(pv, k, n, perm, pv + n, use_smem);
+      count_launch();
+      report(poll_records ? "poll" : "flag", nbf, QRR_THREADS / lpc);
+      return cudaGetLastError();
+    }
+  }
   cudaError_t e = cudaMemsetAsync(work, 0, sizeof(QrWork), st);
   if (e != cudaSuccess) return e;
   QrCand* cand = reinterpret_cast<QrCand*>(w + 1);
   double* candcol = reinterpret_cast<double*>(cand + 2 * NB);
   int64_t* piv = reinterpret_cast<int64_t*>(candcol + 2 * static_cast<size_t>(NB) * ell);
   int64_t* gpos = piv + n;
-  // RS_QRCP_TIMING=1: per-phase cycle counts of CTA 0 printed to stderr (development aid)
-  static long long* tbuf = nullptr;
-  static const bool timing = getenv("RS_QRCP_TIMING") != nullptr;
-  if (timing && !tbuf && cudaMalloc(&tbuf, 8 * 8 * 1024) != cudaSuccess) tbuf = nullptr;
-  long long* tb = (timing && k <= 1024) ? tbuf : nullptr;
   void* args[] = {(void*)&B,   (void*)&ldb, (void*)&ell, (void*)&n,    (void*)&k,  (void*)&w,
                   (void*)&NB,  (void*)&cols_per, (void*)&ldw, (void*)&piv, (void*)&Rho, (void*)&ldr,
                   (void*)&gaps, (void*)&info, (void*)&tb};
@@ -894,20 +1188,7 @@ cudaError_t qrcp_truncated(cudaStream_t st, const double* B, int ldb, int ell, l
   const bool use_smem = psmem <= QR_SMEM_MAX;
   qrcp_perm_kernel<<<1, 1024, use_smem ? psmem : 0, st>>>(piv, k, n, perm, gpos, use_smem);
   count_launch();
-  if (tb) {
-    static long long h[8 * 1024];
-    cudaStreamSynchronize(st);
-    cudaMemcpy(h, tb, 8 * 8 * static_cast<size_t>(k), cudaMemcpyDeviceToHost);
-    double acc[7] = {0};
-    for (int j = 1; j < k; ++j)
-      for (int p = 0; p < 6; ++p) acc[p] += static_cast<double>(h[j * 8 + p + 1] - h[j * 8 + p]);
-    for (int j = 1; j < k; ++j) acc[6] += static_cast<double>(h[j * 8] - h[(j - 1) * 8 + 6]);
-    fprintf(stderr,
-            "QRCP NB=%d cols=%d cycles/step: p0-1=%.0f p1-2=%.0f p2-3=%.0f p3-4=%.0f p4-5=%.0f p5-6=%.0f "
-            "tail=%.0f\n",
-            NB, cols_per, acc[0] / (k - 1), acc[1] / (k - 1), acc[2] / (k - 1), acc[3] / (k - 1), acc[4] / (k - 1),
-            acc[5] / (k - 1), acc[6] / (k - 1));
-  }
+  report(use_reg ? "barrier" : "smem", NB, cols_per);
   return cudaGetLastError();
 }
 

@@ -1,0 +1,60 @@
+// Probe: time the register-tile Cholesky + inverse kernel alone (n = 100, 110, 128).
+// nvcc -gencode arch=compute_100a,code=sm_100a -O3 -I../paper_conf_sc_maryykltd15_b200/csrc chol_bench.cu
+#include <cstdio>
+#include <vector>
+
+#include "../paper_conf_sc_maryykltd15_b200/csrc/chol.cu"
+
+namespace rs {
+void count_launch() {}
+}  // namespace rs
+
+int main() {
+  for (int n : {100, 110, 128}) {
+    const int npad = (n + 15) / 16 * 16;
+    std::vector<double> G(static_cast<size_t>(n) * n);
+    unsigned s = 12345;
+    std::vector<double> X(static_cast<size_t>(n) * 2 * n);
+    for (auto& v : X) {
+      s = s * 1664525u + 1013904223u;
+      v = (s >> 8) * (1.0 / 16777216.0) - 0.5;
+    }
+    for (int i = 0; i < n; ++i)
+      for (int j = 0; j < n; ++j) {
+        double a = 0;
+        for (int t = 0; t < 2 * n; ++t) a += X[i + t * n] * X[j + t * n];
+        G[i + j * n] = a + (i == j ? 0.1 : 0.0);
+      }
+    double *dG, *dR, *dL;
+    int* info;
+    cudaMalloc(&dG, G.size() * 8);
+    cudaMalloc(&dR, npad * npad * 8);
+    cudaMalloc(&dL, npad * npad * 8);
+    cudaMalloc(&info, 16);
+    cudaMemset(info, 0, 16);
+    cudaMemcpy(dG, G.data(), G.size() * 8, cudaMemcpyHostToDevice);
+    const int np = (n + 3) / 4 * 4;
+    const size_t smem = rs::ct_smem_doubles(np) * 8;
+    cudaFuncSetAttribute(rs::chol_tile_kernel<1, 1024>, cudaFuncAttributeMaxDynamicSharedMemorySize,
+                         rs::ct_smem_doubles(128) * 8);
+    {
+      const int exp = 0;
+      cudaEvent_t e0, e1;
+      cudaEventCreate(&e0);
+      cudaEventCreate(&e1);
+      const int reps = 200;
+      for (int r = 0; r < 10; ++r)
+        rs::chol_tile_kernel<1, 1024><<<1, 1024, smem>>>(dG, n, n, dR, npad, dL, npad, info, 5, npad);
+      cudaEventRecord(e0);
+      for (int r = 0; r < reps; ++r)
+        rs::chol_tile_kernel<1, 1024><<<1, 1024, smem>>>(dG, n, n, dR, npad, dL, npad, info, 5, npad);
+      cudaEventRecord(e1);
+      cudaEventSynchronize(e1);
+      float ms = 0;
+      cudaEventElapsedTime(&ms, e0, e1);
+      printf("{\"n\":%d,\"exp\":%d,\"us\":%.2f,\"err\":\"%s\"}\n", n, exp, 1e3 * ms / reps,
+             cudaGetErrorString(cudaGetLastError()));
+    }
+  }
+  return 0;
+}

@@ -215,6 +215,19 @@ def test_pipeline_ragged_and_multitile(m, n, k, p, q, law):
     _compare(A, k, p, q)
 
 
+@pytest.mark.parametrize("m,n,k,p,q", [
+    (2000, 5000, 100, 10, 0),   # cfg2/cfg4's n, k, p: 8 lanes per column, 79 CTAs
+    (1500, 5000, 60, 10, 1),   # (n % m != 0: a Gaussian U, no tied column norms)
+    (600, 9500, 30, 10, 0),     # n > 148 x 64: 4 lanes per column, 75 CTAs
+])
+def test_pipeline_wide_n_grid_qrcp(m, n, k, p, q):
+    """n > 2048: the truncated QRCP runs on the flag-synchronised grid kernel (not the single-
+    cluster one).  A = (n x m matrix with the exp-k law)^T: same singular values, cheap to build."""
+    At, _ = make_matrix(n, m, "exp-k", k, seed=m + 3 * n)
+    A = np.asfortranarray(At.T)
+    _compare(A, k, p, q)
+
+
 def test_pipeline_is_bitwise_deterministic():
     A, _ = make_matrix(5000, 400, "exp-k", 30, seed=5)
     g1 = _run_gpu(A, 30, 10, 1)
