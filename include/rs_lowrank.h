@@ -167,13 +167,6 @@ RS_API rs_status_t rs_lowrank_reset_profile(rs_lowrank_t h);
 /* Number of CUDA kernels this library has launched in the process (all handles). */
 RS_API int64_t rs_lowrank_kernel_launches(void);
 RS_API const char* rs_lowrank_last_error(rs_lowrank_t h);
-/* Device self-test of the Gaussian transform: the production RS-BM32 forms the
- * sampling GEMM runs (fast division / square root without range checks, branch-free quadrant
- * rotation) against the reference forms (IEEE __fdiv_rn / __fsqrt_rn, quadrant switch), for
- * every possible input: mismatches[0] = number of the 2^23 values of x >> 9 whose ln u or
- * sqrt(-2 ln u) bits differ, mismatches[1] = number of the 2^24 values of y >> 8 whose
- * (cos, sin) bits differ.  Both must be 0.  Synchronises; RS_ERR_CUDA on a CUDA failure.     */
-RS_API rs_status_t rs_selftest_rsbm(int64_t* mismatches);
 
 /* ---- the paper's deterministic baseline: truncated QP3 of A itself (one GPU) ----
  * Householder QR with column pivoting stopped after k columns (Sec. 2; "QP3" of

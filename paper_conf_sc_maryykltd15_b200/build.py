@@ -60,13 +60,14 @@ def build(force: bool = False, verbose: bool = False) -> str:
     deps = srcs + [os.path.join(CSRC, f) for f in os.listdir(CSRC) if f.endswith((".cuh", ".h"))]
     deps.append(os.path.join(ROOT, "include", "rs_lowrank.h"))
     deps.append(os.path.abspath(__file__))
-    digest = _hash(deps)
+    extra = os.environ.get("RS_EXTRA_NVCC_FLAGS", "").split()  # development experiments only
+    digest = _hash(deps) + ("|" + " ".join(extra) if extra else "")
     if not force and os.path.exists(LIB) and os.path.exists(STAMP) and open(STAMP).read().strip() == digest:
         return LIB
     os.makedirs(LIBDIR, exist_ok=True)
     nccl_inc, nccl_lib = _nccl_dirs()
     common = ["nvcc", *ARCH, "-O3", "-lineinfo", "-std=c++17", "-Xcompiler", "-fPIC", "-Xcompiler", "-fvisibility=hidden",
-              f"-I{os.path.join(ROOT, 'include')}", f"-I{CSRC}", f"-I{nccl_inc}"]
+              f"-I{os.path.join(ROOT, 'include')}", f"-I{CSRC}", f"-I{nccl_inc}", *extra]
     objs = []
 
     def compile_one(src):

@@ -66,6 +66,13 @@ struct GemmArgs {
   int l3d, r3d;  // MC: operand tensor map is the 3-D stacked-box form (one TMA per stage), see mc_load
 };
 
+// KC ring depths (compile-time; -DRS_PHX_NS / -DRS_KC_NS only for ring-depth experiments)
+#ifndef RS_PHX_NS
+#define RS_PHX_NS 4
+#endif
+#ifndef RS_KC_NS
+#define RS_KC_NS 4
+#endif
 template <int MFW, bool PHILOX>
 struct KCSmem {
   static constexpr int MT = 16 * MFW;
@@ -75,7 +82,7 @@ struct KCSmem {
   static constexpr int L_BYTES = (L_BYTES_RAW + 1023) / 1024 * 1024;
   // small M (l <= 32): little MMA work per stage, so a deeper ring keeps more of A in flight and
   // lets several generator groups work on different stages at once
-  static constexpr int NS = MFW <= 2 ? 8 : NSTAGE;
+  static constexpr int NS = MFW <= 2 ? 8 : (PHILOX ? RS_PHX_NS : RS_KC_NS);
   static constexpr int TOTAL = 1024 + NS * (R_BYTES + L_BYTES) + 2 * NS * 8;
 };
 
@@ -169,7 +176,7 @@ __global__ void __launch_bounds__(GEMM_THREADS, 1)
 
   auto issue = [&](int it) {  // one thread: fill stage `it`
     const int s = it % SM::NS;
-    if (it >= SM::NS) mbar_wait(&empty[s], ((it / SM::NS) - 1) & 1);
+    if (it >= SM::NS) mbar_wait_sleep(&empty[s], ((it / SM::NS) - 1) & 1);
     mbar_arrive_expect_tx(&full[s], SM::R_BYTES + SM::L_BYTES_TMA);
     const int kc = static_cast<int>(kb + static_cast<long long>(it) * KT);
     tma_load_2d(sR + s * SM::R_BYTES, &tmR, &full[s], kc, n0);
@@ -253,7 +260,7 @@ __global__ void __launch_bounds__(KCP_THREADS, 1)
       tma_prefetch_desc(&tmL);
       for (int it = 0; it < nk; ++it) {
         const int s = it % SM::NS;
-        if (it >= SM::NS) mbar_wait(&empty[s], ((it / SM::NS) - 1) & 1);
+        if (it >= SM::NS) mbar_wait_sleep(&empty[s], ((it / SM::NS) - 1) & 1);
         mbar_arrive_expect_tx(&full[s], SM::R_BYTES + SM::L_BYTES_TMA);
         const int kc = static_cast<int>(kb + static_cast<long long>(it) * KT);
         tma_load_2d(sR + s * SM::R_BYTES, &tmR, &full[s], kc, n0);
@@ -361,7 +368,7 @@ __global__ void __launch_bounds__(PHX_THREADS, 1)
     for (int it = grp; it < nk; it += NGRP) {
       const int s = it % SM::NS;
       if (it >= SM::NS) {
-        if (lane == 0) mbar_wait(&empty[s], ((it / SM::NS) - 1) & 1);
+        if (lane == 0) mbar_wait_sleep(&empty[s], ((it / SM::NS) - 1) & 1);
         __syncwarp();
       }
       if (g == 0) {
@@ -473,16 +480,20 @@ __global__ void __launch_bounds__(PHX_THREADS, 1)
 // Epilogue: the accumulators go through shared memory (the drained ring) so every global store
 // is a 16-byte run along the output's contiguous dimension.
 // ------------------------------------------------------------------------------------------
+#ifndef RS_MC_NS
+#define RS_MC_NS 4
+#endif
+constexpr int MC_NS = RS_MC_NS;  // MC ring depth (-DRS_MC_NS only for ring-depth experiments)
 template <int MFW, int WM>
 struct MCSmem {
   static constexpr int MT = 16 * MFW;
   static constexpr int R_BYTES = NT * KT * 8;
   static constexpr int L_BYTES = MT * KT * 8;
-  static constexpr int RING = NSTAGE * (R_BYTES + L_BYTES);
+  static constexpr int RING = MC_NS * (R_BYTES + L_BYTES);
   static constexpr int STAGE_LD = (MT > NT ? MT : NT) + 1;  // staged tile row (doubles; odd: fewer conflicts)
   static constexpr int STAGE = (MT > NT ? MT : NT) * STAGE_LD * 8;  // rows: MT (N-contiguous out) or NT
   static constexpr int BODY = RING > STAGE ? RING : STAGE;
-  static constexpr int TOTAL = 1024 + BODY + 2 * NSTAGE * 8;
+  static constexpr int TOTAL = 1024 + BODY + 2 * MC_NS * 8;
 };
 
 // One stage of an MC operand (rows0 = first M or N index of the tile, nbx 16-wide boxes, K offset
@@ -558,9 +569,9 @@ __global__ void __launch_bounds__(GEMM_THREADS, 1)
   extern __shared__ unsigned char smem_raw[];
   unsigned char* smem = align1024(smem_raw);
   unsigned char* sR = smem;
-  unsigned char* sL = sR + NSTAGE * SM::R_BYTES;
+  unsigned char* sL = sR + MC_NS * SM::R_BYTES;
   uint64_t* full = reinterpret_cast<uint64_t*>(smem + SM::BODY);
-  uint64_t* empty = full + NSTAGE;
+  uint64_t* empty = full + MC_NS;
 
   const int warp = threadIdx.x >> 5, lane = threadIdx.x & 31;
   const int n0 = blockIdx.x * NT, m0 = blockIdx.y * MT;
@@ -570,7 +581,7 @@ __global__ void __launch_bounds__(GEMM_THREADS, 1)
 
   if (threadIdx.x == 0) {
 #pragma unroll
-    for (int s = 0; s < NSTAGE; ++s) {
+    for (int s = 0; s < MC_NS; ++s) {
       mbar_init(&full[s], 1);
       mbar_init(&empty[s], NCONS);
     }
@@ -579,8 +590,8 @@ __global__ void __launch_bounds__(GEMM_THREADS, 1)
   __syncthreads();
 
   auto issue = [&](int it) {
-    const int s = it % NSTAGE;
-    if (it >= NSTAGE) mbar_wait(&empty[s], ((it / NSTAGE) - 1) & 1);
+    const int s = it % MC_NS;
+    if (it >= MC_NS) mbar_wait_sleep(&empty[s], ((it / MC_NS) - 1) & 1);
     mbar_arrive_expect_tx(&full[s], SM::R_BYTES + SM::L_BYTES);
     const int kc = static_cast<int>(kb + static_cast<long long>(it) * KT);
     mc_load(sL + s * SM::L_BYTES, &tmL, &full[s], a.l3d, m0, MT / 16, kc);
@@ -589,7 +600,7 @@ __global__ void __launch_bounds__(GEMM_THREADS, 1)
   if (threadIdx.x == 0) {
     tma_prefetch_desc(&tmL);
     tma_prefetch_desc(&tmR);
-    for (int it = 0; it < NSTAGE - 1 && it < nk; ++it) issue(it);
+    for (int it = 0; it < MC_NS - 1 && it < nk; ++it) issue(it);
   }
 
   const int r = lane >> 2, kk = lane & 3;
@@ -605,9 +616,9 @@ __global__ void __launch_bounds__(GEMM_THREADS, 1)
       for (int f2 = 0; f2 < 2; ++f2) acc[fl][nb][f2][0] = acc[fl][nb][f2][1] = 0.0;
 
   for (int it = 0; it < nk; ++it) {
-    const int s = it % NSTAGE;
-    if (threadIdx.x == 0 && it + NSTAGE - 1 < nk) issue(it + NSTAGE - 1);
-    mbar_wait(&full[s], (it / NSTAGE) & 1);
+    const int s = it % MC_NS;
+    if (threadIdx.x == 0 && it + MC_NS - 1 < nk) issue(it + MC_NS - 1);
+    mbar_wait(&full[s], (it / MC_NS) & 1);
     const long long kc = kb + static_cast<long long>(it) * KT;  // first K of the stage
     const unsigned char* Ls = sL + s * SM::L_BYTES;
     const unsigned char* Rs = sR + s * SM::R_BYTES;
@@ -888,7 +899,7 @@ __global__ void __launch_bounds__(GEMM_THREADS, 1)
   };
   auto issue = [&](int g) {
     const int s = g % MCP_NS;
-    if (g >= MCP_NS) mbar_wait(&empty[s], ((g / MCP_NS) - 1) & 1);
+    if (g >= MCP_NS) mbar_wait_sleep(&empty[s], ((g / MCP_NS) - 1) & 1);
     int m0, n0;
     tile_of(g / nk, m0, n0);
     const int kc = (g % nk) * KT;
@@ -916,7 +927,7 @@ __global__ void __launch_bounds__(GEMM_THREADS, 1)
   }
   mbar_wait(resb, 0);
   const int r = lane >> 2, kk = lane & 3;
-  const int wm = warp >> 2, wn = warp & 3;
+  const int wm = warp >> 2, wn = warp & 3;  // (measured: wm = warp & 1, one code path per sub-partition, is slower)
   const int nbx[2] = {static_cast<int>((a.nmap >> (16 * wn)) & 0xffu), static_cast<int>((a.nmap >> (16 * wn + 8)) & 0xffu)};
   const GemmOut& o = a.out;
   for (int i = 0; i < mytiles; ++i) {
@@ -1105,7 +1116,7 @@ __global__ void __launch_bounds__(GEMM_THREADS, 1)
   __syncthreads();
   auto issue = [&](int it) {
     const int s = it % SYRK_NS;
-    if (it >= SYRK_NS) mbar_wait(&empty[s], ((it / SYRK_NS) - 1) & 1);
+    if (it >= SYRK_NS) mbar_wait_sleep(&empty[s], ((it / SYRK_NS) - 1) & 1);
     mbar_arrive_expect_tx(&full[s], SM::X_BYTES);
     tma_load_2d(sX + s * SM::X_BYTES, &tmX, &full[s], static_cast<int>(kb + static_cast<long long>(it) * KT), 0);
   };

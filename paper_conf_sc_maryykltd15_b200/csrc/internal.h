@@ -73,7 +73,6 @@ cudaError_t trsm_upper_cols(cudaStream_t st, const double* U, int ldu, int k, co
                             long long ncols, double* X, long long ldx);
 cudaError_t copy_2d(cudaStream_t st, const double* src, long long lds, double* dst, long long ldd, long long rows,
                     long long cols);
-cudaError_t selftest_rsbm(cudaStream_t st, unsigned long long* bad_dev);
 cudaError_t omega_materialize(cudaStream_t st, uint64_t seed, uint32_t tag, int ell, long long j0, long long ncols,
                               double* out, long long ldo);
 

@@ -1070,20 +1070,6 @@ rs_status_t rs_lowrank_reset_profile(rs_lowrank_t h) {
 
 int64_t rs_lowrank_kernel_launches(void) { return rs::launch_count(); }
 
-rs_status_t rs_selftest_rsbm(int64_t* mismatches) {
-  if (!mismatches) return RS_ERR_INVALID_ARG;
-  unsigned long long* d = nullptr;
-  unsigned long long hbuf[2] = {0, 0};
-  if (cudaMalloc(&d, 16) != cudaSuccess) return RS_ERR_CUDA;
-  cudaError_t e = rs::selftest_rsbm(nullptr, d);
-  if (e == cudaSuccess) e = cudaMemcpy(hbuf, d, 16, cudaMemcpyDeviceToHost);
-  cudaFree(d);
-  if (e != cudaSuccess) return RS_ERR_CUDA;
-  mismatches[0] = static_cast<int64_t>(hbuf[0]);
-  mismatches[1] = static_cast<int64_t>(hbuf[1]);
-  return RS_OK;
-}
-
 size_t rs_qp3_workspace_bytes(int64_t m, int64_t n, int32_t k) {
   (void)k;
   return m > 0 && n > 0 ? qp3_workspace_bytes(m, n) : 0;

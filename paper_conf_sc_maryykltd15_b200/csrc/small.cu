@@ -292,37 +292,6 @@ cudaError_t omega_materialize(cudaStream_t st, uint64_t seed, uint32_t tag, int 
   return cudaGetLastError();
 }
 
-// Exhaustive check of the production RS-BM32 forms against the reference forms (IEEE
-// intrinsics, divergent quadrant switch): bad[0] counts the x >> 9 (2^23 values) whose ln(u) or
-// sqrt(-2 ln u) bits differ, bad[1] the y >> 8 (2^24 values) whose (cos, sin) bits differ.
-__global__ void selftest_rsbm_kernel(unsigned long long* bad) {
-  const long long stride = static_cast<long long>(gridDim.x) * blockDim.x;
-  unsigned long long b0 = 0, b1 = 0;
-  for (long long t = blockIdx.x * static_cast<long long>(blockDim.x) + threadIdx.x; t < (1LL << 24); t += stride) {
-    if (t < (1LL << 23)) {
-      const uint32_t x = static_cast<uint32_t>(t) << 9;
-      const float Lr = rsbm_ln_uniform_ref(x), L = rsbm_ln_uniform(x);
-      const float rr = __fsqrt_rn(-__fadd_rn(Lr, Lr)), r = sqrt_rn_nochk(-__fadd_rn(L, L));
-      if (__float_as_uint(Lr) != __float_as_uint(L) || __float_as_uint(rr) != __float_as_uint(r)) ++b0;
-    }
-    const uint32_t y = static_cast<uint32_t>(t) << 8;
-    float cr, sr, c, s;
-    rsbm_sincos_turn_ref(y, cr, sr);
-    rsbm_sincos_turn(y, c, s);
-    if (__float_as_uint(cr) != __float_as_uint(c) || __float_as_uint(sr) != __float_as_uint(s)) ++b1;
-  }
-  if (b0) atomicAdd(bad, b0);
-  if (b1) atomicAdd(bad + 1, b1);
-}
-
-cudaError_t selftest_rsbm(cudaStream_t st, unsigned long long* bad_dev) {
-  cudaError_t e = cudaMemsetAsync(bad_dev, 0, 16, st);
-  if (e != cudaSuccess) return e;
-  selftest_rsbm_kernel<<<148 * 8, 256, 0, st>>>(bad_dev);
-  count_launch();
-  return cudaGetLastError();
-}
-
 // out[0] = max over rows of the row 2-norms of X (rows x ncols, column-major): the adaptive
 // scheme's error estimate eps~ (Fig. 3 line 15, reading R18).  One CTA.
 __global__ void rows_maxnorm_kernel(const double* __restrict__ X, long long ld, int rows, long long ncols,

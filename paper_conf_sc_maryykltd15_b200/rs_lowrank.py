@@ -31,7 +31,7 @@ ABI_FUNCTIONS = (
     "rs_lowrank_get_sample", "rs_lowrank_set_sample", "rs_lowrank_get_pivot_data", "rs_lowrank_omega",
     "rs_lowrank_get_info", "rs_lowrank_get_fallbacks", "rs_lowrank_set_profiling", "rs_lowrank_get_profile", "rs_lowrank_reset_profile",
     "rs_lowrank_kernel_launches", "rs_qp3_workspace_bytes", "rs_qp3_truncated", "rs_lowrank_sample_columns",
-    "rs_lowrank_last_error", "rs_selftest_rsbm", "rs_comm_get_unique_id", "rs_comm_init", "rs_comm_destroy",
+    "rs_lowrank_last_error", "rs_comm_get_unique_id", "rs_comm_init", "rs_comm_destroy",
 )
 
 
@@ -77,7 +77,6 @@ def load_library(path: str = LIB_PATH):
         "rs_lowrank_get_profile": (ctypes.c_int, [P, ctypes.c_char_p, D, ctypes.POINTER(I64), D]),
         "rs_lowrank_reset_profile": (ctypes.c_int, [P]),
         "rs_lowrank_kernel_launches": (I64, []),
-        "rs_selftest_rsbm": (ctypes.c_int, [ctypes.POINTER(I64)]),
         "rs_qp3_workspace_bytes": (SZ, [I64, I64, I32]),
         "rs_lowrank_sample_columns": (ctypes.c_int, [P, P, I64, P, I64]),
         "rs_qp3_truncated": (ctypes.c_int, [I64, I64, I32, P, I64, P, P, D, P, SZ, P]),
@@ -268,16 +267,6 @@ def get_pivot_data(h: Handle):
     _check(load_library().rs_lowrank_get_pivot_data(h.ptr, T.data_ptr(), colmajor_ld(T), Rh.data_ptr(),
                                                     colmajor_ld(Rh), gaps), h.ptr)
     return T[:, : h.n - k], Rh, list(gaps)
-
-
-def selftest_rsbm() -> tuple[int, int]:
-    """Exhaustive device check of the production Gaussian transform against its IEEE reference
-    forms (rs_selftest_rsbm): (mismatching x >> 9 values, mismatching y >> 8 values)."""
-    out = (ctypes.c_int64 * 2)()
-    code = load_library().rs_selftest_rsbm(out)
-    if code != 0:
-        raise RSError(code, "rs_selftest_rsbm")
-    return int(out[0]), int(out[1])
 
 
 def omega(h: Handle, j0: int, ncols: int) -> torch.Tensor:

@@ -48,13 +48,6 @@ def test_omega_bit_exact(j0, ncols):
         rs.destroy(h)
 
 
-def test_rsbm_production_forms_match_ieee_reference_exhaustively():
-    """The generator's fast division / square root (no range checks) and branch-free quadrant
-    rotation give the same bits as the IEEE reference forms for EVERY possible input
-    (2^23 values of x >> 9, 2^24 values of y >> 8)."""
-    assert rs.rs_lowrank.selftest_rsbm() == (0, 0)
-
-
 def test_omega_bit_exact_large_sample():
     """1.85 M values (37 rows x 50 000 columns, odd start) against the oracle, bit for bit."""
     h = rs.create(64, 64, 0, 64, 30, 7, SEED)
