@@ -67,6 +67,10 @@ typedef enum {
   RS_ERR_NOT_CONVERGED = 9   /* adaptive sampling reached l_max before eps~ <= eps */
 } rs_status_t;
 
+/* In-place sum over the ranks of `count` doubles at device pointer `buf`, ordered on
+ * `cuda_stream` (cudaStream_t); returns 0 on success.  See rs_lowrank_set_allreduce_hook. */
+typedef int (*rs_allreduce_fn)(void* ctx, double* buf, int64_t count, void* cuda_stream);
+
 /* Bytes of device workspace rs_lowrank_create needs for these sizes (no device access). */
 RS_API size_t rs_lowrank_workspace_bytes(int64_t m_local, int64_t n, int32_t k, int32_t p, int32_t nranks);
 
@@ -167,6 +171,17 @@ RS_API rs_status_t rs_lowrank_reset_profile(rs_lowrank_t h);
 /* Number of CUDA kernels this library has launched in the process (all handles). */
 RS_API int64_t rs_lowrank_kernel_launches(void);
 RS_API const char* rs_lowrank_last_error(rs_lowrank_t h);
+/* Replace NCCL by a caller-supplied allreduce for this handle (the reductions of the
+ * 1-D row distribution are sums of B (l x n) and of the l x l / k x k Gram matrices).  Used to run
+ * several ranks' handles in ONE process on ONE GPU (the multi-rank parity tests), or to plug in
+ * another transport.  nranks / rank: this handle's place in the row partition (create's
+ * m_local / row_offset must match it); fn is called from the pipeline calls, on the calling host
+ * thread, every time the multi-GPU path reduces (same order on every rank); it must return after
+ * the sum is enqueued on (or completed before) cuda_stream.  Only directly after create and only
+ * on a handle created without an NCCL communicator; RS_ERR_BAD_STATE otherwise.  A nonzero
+ * return from fn fails the pipeline call with RS_ERR_NCCL.                                    */
+RS_API rs_status_t rs_lowrank_set_allreduce_hook(rs_lowrank_t h, int32_t nranks, int32_t rank, rs_allreduce_fn fn,
+                                                 void* ctx);
 
 /* ---- the paper's deterministic baseline: truncated QP3 of A itself (one GPU) ----
  * Householder QR with column pivoting stopped after k columns (Sec. 2; "QP3" of

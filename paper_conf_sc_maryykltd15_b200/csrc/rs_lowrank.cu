@@ -105,6 +105,8 @@ struct rs_lowrank_s {
   cudaStream_t st;
   ncclComm_t comm;
   int nranks, rank, sms;
+  rs_allreduce_fn ar_fn = nullptr;  // rs_lowrank_set_allreduce_hook: replaces NCCL for this handle
+  void* ar_ctx = nullptr;
   Layout L;
   char* ws;
   double *B, *Bt, *B1, *C, *C1, *part, *G, *Rf, *Linv, *cholw, *Rho, *Rhat, *T, *Q1, *R1, *R2, *Rbar, *gaps;
@@ -195,6 +197,11 @@ void drain_profile(rs_lowrank_t h) {
 }
 
 rs_status_t allreduce(rs_lowrank_t h, double* buf, long long count) {
+  if (h->ar_fn && h->nranks > 1 && count > 0) {
+    Scope sc(h, "comm", 0.0);
+    if (h->ar_fn(h->ar_ctx, buf, count, h->st) != 0) return fail(h, RS_ERR_NCCL, "allreduce hook failed");
+    return RS_OK;
+  }
   if (!h->comm || h->nranks <= 1 || count <= 0) return RS_OK;
   Scope sc(h, "comm", 0.0);
   RS_NCCL(h, ncclAllReduce(buf, buf, static_cast<size_t>(count), ncclDouble, ncclSum, h->comm, h->st));
@@ -1069,6 +1076,19 @@ rs_status_t rs_lowrank_reset_profile(rs_lowrank_t h) {
 }
 
 int64_t rs_lowrank_kernel_launches(void) { return rs::launch_count(); }
+
+rs_status_t rs_lowrank_set_allreduce_hook(rs_lowrank_t h, int32_t nranks, int32_t rank, rs_allreduce_fn fn,
+                                          void* ctx) {
+  if (!h) return RS_ERR_INVALID_ARG;
+  if (h->state != ST_CREATED) return fail(h, RS_ERR_BAD_STATE, "set_allreduce_hook must follow create");
+  if (h->comm) return fail(h, RS_ERR_BAD_STATE, "handle already has an NCCL communicator");
+  if (nranks < 1 || rank < 0 || rank >= nranks || (nranks > 1 && !fn)) return RS_ERR_INVALID_ARG;
+  h->ar_fn = fn;
+  h->ar_ctx = ctx;
+  h->nranks = nranks;
+  h->rank = rank;
+  return RS_OK;
+}
 
 size_t rs_qp3_workspace_bytes(int64_t m, int64_t n, int32_t k) {
   (void)k;

@@ -31,8 +31,12 @@ ABI_FUNCTIONS = (
     "rs_lowrank_get_sample", "rs_lowrank_set_sample", "rs_lowrank_get_pivot_data", "rs_lowrank_omega",
     "rs_lowrank_get_info", "rs_lowrank_get_fallbacks", "rs_lowrank_set_profiling", "rs_lowrank_get_profile", "rs_lowrank_reset_profile",
     "rs_lowrank_kernel_launches", "rs_qp3_workspace_bytes", "rs_qp3_truncated", "rs_lowrank_sample_columns",
-    "rs_lowrank_last_error", "rs_comm_get_unique_id", "rs_comm_init", "rs_comm_destroy",
+    "rs_lowrank_last_error", "rs_lowrank_set_allreduce_hook", "rs_comm_get_unique_id", "rs_comm_init", "rs_comm_destroy",
 )
+
+
+# rs_allreduce_fn: int (*)(void* ctx, double* buf, int64_t count, void* cuda_stream)
+ALLREDUCE_FN = ctypes.CFUNCTYPE(ctypes.c_int, ctypes.c_void_p, ctypes.c_void_p, ctypes.c_int64, ctypes.c_void_p)
 
 
 class RSError(RuntimeError):
@@ -77,6 +81,7 @@ def load_library(path: str = LIB_PATH):
         "rs_lowrank_get_profile": (ctypes.c_int, [P, ctypes.c_char_p, D, ctypes.POINTER(I64), D]),
         "rs_lowrank_reset_profile": (ctypes.c_int, [P]),
         "rs_lowrank_kernel_launches": (I64, []),
+        "rs_lowrank_set_allreduce_hook": (ctypes.c_int, [P, I32, I32, ALLREDUCE_FN, P]),
         "rs_qp3_workspace_bytes": (SZ, [I64, I64, I32]),
         "rs_lowrank_sample_columns": (ctypes.c_int, [P, P, I64, P, I64]),
         "rs_qp3_truncated": (ctypes.c_int, [I64, I64, I32, P, I64, P, P, D, P, SZ, P]),
@@ -267,6 +272,24 @@ def get_pivot_data(h: Handle):
     _check(load_library().rs_lowrank_get_pivot_data(h.ptr, T.data_ptr(), colmajor_ld(T), Rh.data_ptr(),
                                                     colmajor_ld(Rh), gaps), h.ptr)
     return T[:, : h.n - k], Rh, list(gaps)
+
+
+def set_allreduce_hook(h: Handle, nranks: int, rank: int, fn) -> None:
+    """Route this handle's reductions through `fn(buf_ptr, count, stream_ptr) -> None` instead of
+    NCCL (rs_lowrank_set_allreduce_hook).  The ctypes callback is kept alive on the handle."""
+    def _cb(ctx, buf, count, stream):
+        try:
+            fn(int(buf), int(count), int(stream) if stream else 0)
+            return 0
+        except Exception:  # noqa: BLE001 -- reported to the library as a failed reduction
+            import traceback
+
+            traceback.print_exc()
+            return 1
+
+    cb = ALLREDUCE_FN(_cb)
+    h._ar_cb = cb
+    _check(load_library().rs_lowrank_set_allreduce_hook(h.ptr, nranks, rank, cb, None), h.ptr)
 
 
 def omega(h: Handle, j0: int, ncols: int) -> torch.Tensor:
