@@ -5,6 +5,7 @@ N handles' device buffers instead of NCCL.  Every CUDA kernel of the N > 1 code 
 as it does under NCCL; only the transport differs.  Results are compared with the CPU oracle
 (same tolerances as tests/test_gpu_parity.py) and with the single-rank GPU run."""
 
+import os
 import threading
 
 import numpy as np
@@ -24,6 +25,7 @@ from paper_conf_sc_maryykltd15_b200.partition import row_split  # noqa: E402
 from synth.matrices import make_matrix  # noqa: E402
 
 SEED = 0x5C15
+_OVERLAP = os.environ.get("RS_MR_OVERLAP") == "1"  # debugging: let the ranks' kernels overlap
 
 
 @pytest.fixture(scope="module", autouse=True)
@@ -64,7 +66,8 @@ class InProcessAllreduce:
             stream.synchronize()
             self.bufs[rank] = (buf, count)
             self.calls[rank] += 1
-            self.token.release()
+            if not _OVERLAP:
+                self.token.release()
             self.barrier.wait()
             if rank == 0:
                 counts = {c for _, c in self.bufs}
@@ -80,7 +83,8 @@ class InProcessAllreduce:
                     v.copy_(src)
                 torch.cuda.synchronize()
             self.barrier.wait()
-            self.token.acquire()
+            if not _OVERLAP:
+                self.token.acquire()
 
         return fn
 
@@ -93,7 +97,8 @@ def _run_ranks(A, nranks, k, p, q):
     dev = torch.device("cuda", 0)
 
     def work(r):
-        comm.token.acquire()
+        if not _OVERLAP:
+            comm.token.acquire()
         try:
             torch.cuda.set_device(dev)
             r0, r1 = row_split(m, nranks, r)
@@ -121,7 +126,8 @@ def _run_ranks(A, nranks, k, p, q):
             errs[r] = e
             comm.barrier.abort()
         finally:
-            comm.token.release()
+            if not _OVERLAP:
+                comm.token.release()
 
     ts = [threading.Thread(target=work, args=(r,)) for r in range(nranks)]
     for t in ts:
