@@ -635,15 +635,22 @@ cudaError_t chol_inv(cudaStream_t st, const double* G, int ldg, int n, int npad,
     static bool attr_t = false;
     constexpr int ct_max_smem = ct_smem_doubles(CT_MAXN) * 8;
     if (!attr_t) {
-      cudaError_t e = cudaFuncSetAttribute(chol_tile_kernel<1, 1024>, cudaFuncAttributeMaxDynamicSharedMemorySize,
-                                           ct_max_smem);
-      if (e == cudaSuccess)
-        e = cudaFuncSetAttribute(chol_tile_kernel<2, 576>, cudaFuncAttributeMaxDynamicSharedMemorySize, ct_max_smem);
+      cudaError_t e = cudaSuccess;
+      for (auto fn : {chol_tile_kernel<1, 256>, chol_tile_kernel<1, 512>, chol_tile_kernel<1, 1024>,
+                      chol_tile_kernel<2, 576>})
+        if (e == cudaSuccess) e = cudaFuncSetAttribute(fn, cudaFuncAttributeMaxDynamicSharedMemorySize, ct_max_smem);
       if (e != cudaSuccess) return e;
       attr_t = true;
     }
     const size_t ct_smem = static_cast<size_t>(ct_smem_doubles(4 * nt)) * 8;
-    if (tpt == 1 && nt * (nt + 1) <= 1024)  // one tile per thread (n <= 124)
+    // one tile per thread, in the smallest CTA that holds all nt (nt + 1) tiles: idle warps would
+    // still take part in every pivot's barrier
+    const int tiles = nt * (nt + 1);
+    if (tpt == 1 && tiles <= 256)  // n <= 60 (adaptive blocks, Fig. 7's k = 54)
+      chol_tile_kernel<1, 256><<<1, 256, ct_smem, st>>>(G, ldg, n, R, ldr, Linv, ldl, info, info_code, npad);
+    else if (tpt == 1 && tiles <= 512)  // n <= 88 (l = 64)
+      chol_tile_kernel<1, 512><<<1, 512, ct_smem, st>>>(G, ldg, n, R, ldr, Linv, ldl, info, info_code, npad);
+    else if (tpt == 1 && tiles <= 1024)  // n <= 124
       chol_tile_kernel<1, 1024><<<1, 1024, ct_smem, st>>>(G, ldg, n, R, ldr, Linv, ldl, info, info_code, npad);
     else
       chol_tile_kernel<2, 576><<<1, 576, ct_smem, st>>>(G, ldg, n, R, ldr, Linv, ldl, info, info_code, npad);

@@ -10,7 +10,7 @@ void count_launch() {}
 }  // namespace rs
 
 int main() {
-  for (int n : {100, 110, 128}) {
+  for (int n : {54, 64, 100, 110}) {
     const int npad = (n + 15) / 16 * 16;
     std::vector<double> G(static_cast<size_t>(n) * n);
     unsigned s = 12345;
@@ -35,24 +35,28 @@ int main() {
     cudaMemcpy(dG, G.data(), G.size() * 8, cudaMemcpyHostToDevice);
     const int np = (n + 3) / 4 * 4;
     const size_t smem = rs::ct_smem_doubles(np) * 8;
-    cudaFuncSetAttribute(rs::chol_tile_kernel<1, 1024>, cudaFuncAttributeMaxDynamicSharedMemorySize,
-                         rs::ct_smem_doubles(128) * 8);
-    {
-      const int exp = 0;
+    for (auto fn : {rs::chol_tile_kernel<1, 256>, rs::chol_tile_kernel<1, 512>, rs::chol_tile_kernel<1, 1024>})
+      cudaFuncSetAttribute(fn, cudaFuncAttributeMaxDynamicSharedMemorySize, rs::ct_smem_doubles(128) * 8);
+    const int tiles = (np / 4) * (np / 4 + 1);
+    for (int nthr : {256, 512, 1024}) {
+      if (tiles > nthr) continue;
       cudaEvent_t e0, e1;
       cudaEventCreate(&e0);
       cudaEventCreate(&e1);
       const int reps = 200;
-      for (int r = 0; r < 10; ++r)
-        rs::chol_tile_kernel<1, 1024><<<1, 1024, smem>>>(dG, n, n, dR, npad, dL, npad, info, 5, npad);
+      auto launch = [&] {
+        if (nthr == 256) rs::chol_tile_kernel<1, 256><<<1, 256, smem>>>(dG, n, n, dR, npad, dL, npad, info, 5, npad);
+        else if (nthr == 512) rs::chol_tile_kernel<1, 512><<<1, 512, smem>>>(dG, n, n, dR, npad, dL, npad, info, 5, npad);
+        else rs::chol_tile_kernel<1, 1024><<<1, 1024, smem>>>(dG, n, n, dR, npad, dL, npad, info, 5, npad);
+      };
+      for (int r = 0; r < 10; ++r) launch();
       cudaEventRecord(e0);
-      for (int r = 0; r < reps; ++r)
-        rs::chol_tile_kernel<1, 1024><<<1, 1024, smem>>>(dG, n, n, dR, npad, dL, npad, info, 5, npad);
+      for (int r = 0; r < reps; ++r) launch();
       cudaEventRecord(e1);
       cudaEventSynchronize(e1);
       float ms = 0;
       cudaEventElapsedTime(&ms, e0, e1);
-      printf("{\"n\":%d,\"exp\":%d,\"us\":%.2f,\"err\":\"%s\"}\n", n, exp, 1e3 * ms / reps,
+      printf("{\"n\":%d,\"threads\":%d,\"us\":%.2f,\"err\":\"%s\"}\n", n, nthr, 1e3 * ms / reps,
              cudaGetErrorString(cudaGetLastError()));
     }
   }
