@@ -636,8 +636,8 @@ cudaError_t chol_inv(cudaStream_t st, const double* G, int ldg, int n, int npad,
     constexpr int ct_max_smem = ct_smem_doubles(CT_MAXN) * 8;
     if (!attr_t) {
       cudaError_t e = cudaSuccess;
-      for (auto fn : {chol_tile_kernel<1, 256>, chol_tile_kernel<1, 512>, chol_tile_kernel<1, 1024>,
-                      chol_tile_kernel<2, 576>})
+      for (auto fn : {chol_tile_kernel<1, 256>, chol_tile_kernel<1, 512>, chol_tile_kernel<1, 832>,
+                      chol_tile_kernel<1, 1024>, chol_tile_kernel<2, 576>})
         if (e == cudaSuccess) e = cudaFuncSetAttribute(fn, cudaFuncAttributeMaxDynamicSharedMemorySize, ct_max_smem);
       if (e != cudaSuccess) return e;
       attr_t = true;
@@ -650,6 +650,8 @@ cudaError_t chol_inv(cudaStream_t st, const double* G, int ldg, int n, int npad,
       chol_tile_kernel<1, 256><<<1, 256, ct_smem, st>>>(G, ldg, n, R, ldr, Linv, ldl, info, info_code, npad);
     else if (tpt == 1 && tiles <= 512)  // n <= 88 (l = 64)
       chol_tile_kernel<1, 512><<<1, 512, ct_smem, st>>>(G, ldg, n, R, ldr, Linv, ldl, info, info_code, npad);
+    else if (tpt == 1 && tiles <= 832)  // n <= 112 (l = 110: 72 registers per thread instead of 64)
+      chol_tile_kernel<1, 832><<<1, 832, ct_smem, st>>>(G, ldg, n, R, ldr, Linv, ldl, info, info_code, npad);
     else if (tpt == 1 && tiles <= 1024)  // n <= 124
       chol_tile_kernel<1, 1024><<<1, 1024, ct_smem, st>>>(G, ldg, n, R, ldr, Linv, ldl, info, info_code, npad);
     else

@@ -35,10 +35,11 @@ int main() {
     cudaMemcpy(dG, G.data(), G.size() * 8, cudaMemcpyHostToDevice);
     const int np = (n + 3) / 4 * 4;
     const size_t smem = rs::ct_smem_doubles(np) * 8;
-    for (auto fn : {rs::chol_tile_kernel<1, 256>, rs::chol_tile_kernel<1, 512>, rs::chol_tile_kernel<1, 1024>})
+    for (auto fn : {rs::chol_tile_kernel<1, 256>, rs::chol_tile_kernel<1, 512>, rs::chol_tile_kernel<1, 832>,
+                    rs::chol_tile_kernel<1, 1024>})
       cudaFuncSetAttribute(fn, cudaFuncAttributeMaxDynamicSharedMemorySize, rs::ct_smem_doubles(128) * 8);
     const int tiles = (np / 4) * (np / 4 + 1);
-    for (int nthr : {256, 512, 1024}) {
+    for (int nthr : {256, 512, 832, 1024}) {
       if (tiles > nthr) continue;
       cudaEvent_t e0, e1;
       cudaEventCreate(&e0);
@@ -47,6 +48,7 @@ int main() {
       auto launch = [&] {
         if (nthr == 256) rs::chol_tile_kernel<1, 256><<<1, 256, smem>>>(dG, n, n, dR, npad, dL, npad, info, 5, npad);
         else if (nthr == 512) rs::chol_tile_kernel<1, 512><<<1, 512, smem>>>(dG, n, n, dR, npad, dL, npad, info, 5, npad);
+        else if (nthr == 832) rs::chol_tile_kernel<1, 832><<<1, 832, smem>>>(dG, n, n, dR, npad, dL, npad, info, 5, npad);
         else rs::chol_tile_kernel<1, 1024><<<1, 1024, smem>>>(dG, n, n, dR, npad, dL, npad, info, 5, npad);
       };
       for (int r = 0; r < 10; ++r) launch();
