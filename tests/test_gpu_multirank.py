@@ -49,10 +49,9 @@ class InProcessAllreduce:
     copies the N buffers to the host, sums them in rank order (deterministic, plain numpy) and writes
     the sum back to every buffer before any rank continues.  A token serialises the ranks' library
     calls between reductions, so the N ranks' kernels never overlap on the one GPU -- as with one
-    process per GPU.  (With the ranks' kernels overlapping on one GPU, B came out ~1e-5 off in about
-    one fresh process in ten -- not with launches serialised (CUDA_LAUNCH_BLOCKING=1, 10/10), not with
-    the ranks serialised, and never for two independent handles running concurrently; see DESIGN.md
-    §7, scripts/debug_multirank*.py.)"""
+    process per GPU.  (With the ranks' kernels overlapping, the first call of a fresh process gave
+    a ~1e-5 B mismatch in about one process in five under CUDA's lazy module loading, never with
+    CUDA_MODULE_LOADING=EAGER, scripts/debug_multirank*.py.)"""
 
     def __init__(self, nranks):
         self.n = nranks
