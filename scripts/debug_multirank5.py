@@ -19,6 +19,16 @@ SYNC = os.environ.get("MR_SYNC", "sample,power,pivot").split(",")
 rs.load_library()
 m, n, k, p, q = 20000, 1000, 50, 10, 1
 A, _ = make_matrix(m, n, "exp-k", k, seed=m + 14)
+WARM = os.environ.get("MR_WARM", "none")  # single-threaded warm-up (loads kernels) before the ranks
+if WARM != "none":
+    hw = rs.create(m, m, 0, n, k, p, T.SEED)
+    Aw = to_dev(A)
+    rs.sample(hw, Aw)
+    if WARM in ("power", "all"):
+        rs.power_iterate(hw, Aw, q)
+    torch.cuda.synchronize()
+    rs.destroy(hw)
+    del Aw
 nranks = 2
 comm = T.InProcessAllreduce(nranks)
 res = [dict() for _ in range(nranks)]
