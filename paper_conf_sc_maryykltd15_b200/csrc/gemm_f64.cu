@@ -61,7 +61,10 @@ bool make_tmap3(CUtensorMap* m, const View2D& v, uint32_t nbx) {
 template <int MFW>
 cudaError_t launch_kc_t(cudaStream_t st, dim3 grid, const CUtensorMap& tR, const CUtensorMap& tL, const GemmArgs& a) {
   constexpr int smem = KCSmem<MFW, false>::TOTAL;
-  static const bool pwg = getenv("RS_KC_PWG") != nullptr;  // development switch: producer warpgroup
+  // producer warpgroup (default): with the producer sleeping in the slot wait (mbar_wait_sleep) the
+  // MMA warps no longer carry the TMA issue; cfg4 B = C~ A 32.07 -> 31.36 ms.  RS_KC_NO_PWG: TMA
+  // issued by thread 0 of MMA warp 0 (A/B switch)
+  static const bool pwg = getenv("RS_KC_NO_PWG") == nullptr;
   if (pwg) {
     static bool attr_p = false;
     if (!attr_p) {
