@@ -148,6 +148,19 @@ cudaError_t launch_mc_wm(cudaStream_t st, dim3 grid, const CUtensorMap& tL, cons
     }
     attr_set = true;
   }
+  // dense 1x8 products (C = B~ A^T): dedicated producer warpgroup; RS_MC_NO_PWG: A/B switch
+  static const bool pwg = getenv("RS_MC_NO_PWG") == nullptr;
+  if (WM == 1 && a.tri == 0 && pwg) {
+    static bool attr_p = false;
+    if (!attr_p) {
+      cudaError_t e = cudaFuncSetAttribute(mc_gemm_pwg_kernel<MFW, WM, 0>, cudaFuncAttributeMaxDynamicSharedMemorySize, smem);
+      if (e != cudaSuccess) return e;
+      attr_p = true;
+    }
+    mc_gemm_pwg_kernel<MFW, WM, 0><<<grid, KCP_THREADS, smem, st>>>(tL, tR, a);
+    count_launch();
+    return cudaGetLastError();
+  }
   if (a.tri == 1)
     mc_gemm_kernel<MFW, WM, 1><<<grid, GEMM_THREADS, smem, st>>>(tL, tR, a);
   else if (a.tri == 2)

@@ -701,6 +701,155 @@ __global__ void __launch_bounds__(GEMM_THREADS, 1)
   }
 }
 
+// MC with a dedicated producer warpgroup (warps 8-11, as kc_gemm_pwg_kernel): the MMA warps never
+// carry the TMA issue; the epilogue synchronises the 8 MMA warps with a named barrier.
+template <int MFW, int WM, int TRI>
+__global__ void __launch_bounds__(KCP_THREADS, 1)
+    mc_gemm_pwg_kernel(const __grid_constant__ CUtensorMap tmL, const __grid_constant__ CUtensorMap tmR,
+                   const GemmArgs a) {
+  using SM = MCSmem<MFW, WM>;
+  constexpr int MT = SM::MT;
+  constexpr int NFR = WM == 1 ? 2 * MFW : MFW;  // 8-row M fragments per warp
+  constexpr int NB = WM == 1 ? 1 : 2;            // N boxes per warp
+  extern __shared__ unsigned char smem_raw[];
+  unsigned char* smem = align1024(smem_raw);
+  unsigned char* sR = smem;
+  unsigned char* sL = sR + MC_NS * SM::R_BYTES;
+  uint64_t* full = reinterpret_cast<uint64_t*>(smem + SM::BODY);
+  uint64_t* empty = full + MC_NS;
+
+  const int warp = threadIdx.x >> 5, lane = threadIdx.x & 31;
+  const int n0 = blockIdx.x * NT, m0 = blockIdx.y * MT;
+  const long long kb = static_cast<long long>(blockIdx.z) * a.k_chunk;
+  const long long ke = min(a.K, kb + a.k_chunk);
+  const int nk = kb < ke ? static_cast<int>((ke - kb + KT - 1) / KT) : 0;
+
+  if (threadIdx.x == 0) {
+#pragma unroll
+    for (int s = 0; s < MC_NS; ++s) {
+      mbar_init(&full[s], 1);
+      mbar_init(&empty[s], NCONS);
+    }
+    fence_mbar_init();
+  }
+  __syncthreads();
+
+  auto issue = [&](int it) {
+    const int s = it % MC_NS;
+    if (it >= MC_NS) mbar_wait_sleep(&empty[s], ((it / MC_NS) - 1) & 1);
+    mbar_arrive_expect_tx(&full[s], SM::R_BYTES + SM::L_BYTES);
+    const int kc = static_cast<int>(kb + static_cast<long long>(it) * KT);
+    mc_load(sL + s * SM::L_BYTES, &tmL, &full[s], a.l3d, m0, MT / 16, kc);
+    mc_load(sR + s * SM::R_BYTES, &tmR, &full[s], a.r3d, n0, NT / 16, kc);
+  };
+  if (warp >= NCONS) {
+    asm volatile("setmaxnreg.dec.sync.aligned.u32 %0;\n" ::"n"(MCP_PROD_REGS));
+    if (warp == NCONS && lane == 0) {
+      tma_prefetch_desc(&tmL);
+      tma_prefetch_desc(&tmR);
+      for (int it = 0; it < nk; ++it) issue(it);
+    }
+    return;
+  }
+  asm volatile("setmaxnreg.inc.sync.aligned.u32 %0;\n" ::"n"(MCP_MMA_REGS));
+
+  const int r = lane >> 2, kk = lane & 3;
+  const int wm = WM == 1 ? 0 : warp >> 2;
+  const int nbox0 = WM == 1 ? warp : 2 * (warp & 3);  // first N box of this warp
+  const int phi0 = wm * NFR;                          // first M fragment of this warp
+  double acc[NFR][NB][2][2];
+#pragma unroll
+  for (int fl = 0; fl < NFR; ++fl)
+#pragma unroll
+    for (int nb = 0; nb < NB; ++nb)
+#pragma unroll
+      for (int f2 = 0; f2 < 2; ++f2) acc[fl][nb][f2][0] = acc[fl][nb][f2][1] = 0.0;
+
+  for (int it = 0; it < nk; ++it) {
+    const int s = it % MC_NS;
+    mbar_wait(&full[s], (it / MC_NS) & 1);
+    const long long kc = kb + static_cast<long long>(it) * KT;  // first K of the stage
+    const unsigned char* Ls = sL + s * SM::L_BYTES;
+    const unsigned char* Rs = sR + s * SM::R_BYTES;
+    // compile-time fragment sets: the dense path has no per-box branches
+    if (WM == 1 || wm == 0)
+      mc_stage<NFR, 0, NB, TRI>(acc, Ls, Rs, nbox0, r, kk, kc, m0, n0);
+    else
+      mc_stage<NFR, NFR, NB, TRI>(acc, Ls, Rs, nbox0, r, kk, kc, m0, n0);
+    __syncwarp();
+    if (lane == 0) mbar_arrive(&empty[s]);
+  }
+
+  // ---- epilogue: stage the MT x NT tile in shared memory, then coalesced 16-byte stores ----
+  const GemmOut& o = a.out;
+  double* base = o.ptr + static_cast<long long>(blockIdx.z) * o.split_stride;
+  const bool n_contig = o.ld_n == 1, m_contig = o.ld_m == 1;
+  if (!n_contig && !m_contig) {  // generic strides: direct stores
+#pragma unroll
+    for (int fl = 0; fl < NFR; ++fl) {
+      const int phi = phi0 + fl;
+      const long long gm = m0 + 16 * (phi >> 1) + 2 * r + (phi & 1);
+      if (gm >= o.m_store) continue;
+#pragma unroll
+      for (int nb = 0; nb < NB; ++nb)
+#pragma unroll
+        for (int f2 = 0; f2 < 2; ++f2)
+#pragma unroll
+          for (int e = 0; e < 2; ++e) {
+            const long long gn = n0 + 16 * (nbox0 + nb) + 2 * (2 * kk + e) + f2;
+            if (gn < o.n_store) gemm_put(base + gm * o.ld_m + gn * o.ld_n, acc[fl][nb][f2][e], o.mode);
+          }
+    }
+    return;
+  }
+  named_bar_sync(1, GEMM_THREADS);  // every MMA warp is done with the ring
+  double* st = reinterpret_cast<double*>(smem);
+  // n_contig: st[m * LDS + n] (rows along N); else st[n * LDS + m] (rows along M)
+  constexpr int LDS = SM::STAGE_LD;
+#pragma unroll
+  for (int fl = 0; fl < NFR; ++fl) {
+    const int phi = phi0 + fl;
+    const int lm = 16 * (phi >> 1) + 2 * r + (phi & 1);
+#pragma unroll
+    for (int nb = 0; nb < NB; ++nb)
+#pragma unroll
+      for (int f2 = 0; f2 < 2; ++f2)
+#pragma unroll
+        for (int e = 0; e < 2; ++e) {
+          const int ln = 16 * (nbox0 + nb) + 2 * (2 * kk + e) + f2;
+          st[n_contig ? lm * LDS + ln : ln * LDS + lm] = acc[fl][nb][f2][e];
+        }
+  }
+  named_bar_sync(1, GEMM_THREADS);
+  // rows of the staged tile: n_contig -> MT rows of NT; else NT rows of MT
+  const int nrows = n_contig ? MT : NT, rowlen = n_contig ? NT : MT;
+  const long long row0 = n_contig ? m0 : n0, col0 = n_contig ? n0 : m0;
+  const long long row_lim = n_contig ? o.m_store : o.n_store, col_lim = n_contig ? o.n_store : o.m_store;
+  const long long ld_row = n_contig ? o.ld_m : o.ld_n;
+  const int pairs = rowlen / 2;
+  for (int idx = threadIdx.x; idx < nrows * pairs; idx += GEMM_THREADS) {
+    const int lr = idx / pairs, lc = 2 * (idx - lr * pairs);
+    const long long gr = row0 + lr, gc = col0 + lc;
+    if (gr >= row_lim || gc >= col_lim) continue;
+    double* p = base + gr * ld_row + gc;
+    const double v0 = st[lr * LDS + lc], v1 = st[lr * LDS + lc + 1];
+    if (gc + 1 < col_lim && (reinterpret_cast<uintptr_t>(p) & 15) == 0) {
+      double2* p2 = reinterpret_cast<double2*>(p);
+      if (o.mode) {
+        double2 c = *p2;
+        c.x -= v0;
+        c.y -= v1;
+        *p2 = c;
+      } else {
+        *p2 = make_double2(v0, v1);
+      }
+    } else {
+      gemm_put(p, v0, o.mode);
+      if (gc + 1 < col_lim) gemm_put(p + 1, v1, o.mode);
+    }
+  }
+}
+
 // ------------------------------------------------------------------------------------------
 // Persistent MC for the short-K products (K <= 128: C1 = L^{-1} C, Q1 = X R^{-1}): a CTA has
 // only ceil(K/16) stages of work per tile, so one tile per CTA leaves the TMA round trip and the
