@@ -15,6 +15,9 @@ extraction of the SC15 paper), with the section / figure / equation named.
 
 Modules
 -------
+``gemm``     the oracle's own fixed-order matrix product (plain C loop nest in
+             ``csrc/gemm.c``, every output summed in increasing k; SURVEY
+             §8(c) c-1 step 2) -- every product of the oracle goes through it.
 ``philox``   Philox4x32-10 and the RS-BM32 Gaussian transform,
              i.e. the PRNG(l, m) of Fig. 2(b) line 2.
 ``linalg``   Householder QR (sign-normalised), truncated QRCP with recomputed
@@ -27,4 +30,4 @@ the paper prints, closed forms, brute force or an independent library routine
 (LAPACK via numpy/scipy, used in tests only).  See DESIGN.md §4 for the list.
 """
 
-from . import philox, linalg, pipeline  # noqa: F401
+from . import gemm, philox, linalg, pipeline  # noqa: F401

@@ -2,14 +2,16 @@
 
 TEST INFRASTRUCTURE ONLY (see oracle/__init__.py).  Plain numpy, float64,
 one column / one pivot step at a time, in the order the paper's algorithms
-(and the LAPACK routines it names) perform them.  ``np.linalg.norm`` and ``@``
-are used as library primitives for single steps (a 2-norm, a matrix-vector or
-outer product); nothing is blocked, fused or reordered.
+(and the LAPACK routines it names) perform them.  Vector-matrix products go
+through the oracle's own fixed-order GEMM (``oracle.gemm.matmul``); 2-norms are
+sqrt(sum of squares); nothing is blocked, fused or reordered.
 """
 
 from __future__ import annotations
 
 import numpy as np
+
+from .gemm import matmul
 
 
 class RankDeficientError(ValueError):
@@ -25,7 +27,7 @@ def dlarfg(x: np.ndarray):
     """
     x = np.asarray(x, dtype=np.float64)
     alpha = float(x[0])
-    xnorm = float(np.linalg.norm(x[1:])) if x.size > 1 else 0.0
+    xnorm = float(np.sqrt(np.sum(x[1:] * x[1:]))) if x.size > 1 else 0.0
     v = np.zeros_like(x)
     v[0] = 1.0
     if xnorm == 0.0:
@@ -51,7 +53,7 @@ def householder_qr(X: np.ndarray):
     for j in range(n):
         beta, tau, v = dlarfg(A[j:, j])
         if tau != 0.0 and j + 1 < n:
-            w = v @ A[j:, j + 1:]
+            w = matmul(v, A[j:, j + 1:])
             A[j:, j + 1:] -= tau * np.outer(v, w)
         A[j, j] = beta
         A[j + 1:, j] = 0.0
@@ -63,7 +65,7 @@ def householder_qr(X: np.ndarray):
     for j in reversed(range(n)):          # Q = H_0 H_1 ... H_{n-1} [I; 0]
         v, tau = vs[j], taus[j]
         if tau != 0.0:
-            w = v @ Q[j:, :]
+            w = matmul(v, Q[j:, :])
             Q[j:, :] -= tau * np.outer(v, w)
     d = np.where(np.diag(R) < 0.0, -1.0, 1.0)
     return Q * d[None, :], R * d[:, None]
@@ -116,7 +118,7 @@ def qrcp_truncated(B: np.ndarray, k: int, *, return_trailing: bool = False):
             perm[[j, p]] = perm[[p, j]]
         beta, tau, v = dlarfg(W[j:, j])
         if tau != 0.0 and j + 1 < n:
-            w = v @ W[j:, j + 1:]
+            w = matmul(v, W[j:, j + 1:])
             W[j:, j + 1:] -= tau * np.outer(v, w)
         W[j, j] = beta
         W[j + 1:, j] = 0.0
@@ -134,6 +136,6 @@ def back_substitution(U: np.ndarray, Y: np.ndarray) -> np.ndarray:
     k = U.shape[0]
     for i in reversed(range(k)):
         if i + 1 < k:
-            X[i] -= U[i, i + 1:] @ X[i + 1:]
+            X[i] -= matmul(U[i, i + 1:], X[i + 1:])
         X[i] /= U[i, i]
     return X
