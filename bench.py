@@ -7,8 +7,11 @@ A P_{1:k}, R = Rbar [I T]).  A is resident in HBM and row-block partitioned over
 
     python bench.py [--gpus N] [--steps K] [--warmup W] [--workload cfg4] [--impl ours|reference]
 
-Prints ONE JSON line on rank 0.  --impl reference times the CPU oracle (the only reference this
-paper has: it ships no code) on a bounded row sample of the same workload.
+Prints ONE JSON line on rank 0.  With --gpus N > 1 and no torchrun environment (WORLD_SIZE unset)
+the script re-launches itself under torch.distributed.run with N ranks on 127.0.0.1.  The timed
+step is rs_lowrank_run (the whole step replayed as one CUDA graph).  --impl reference times the CPU
+oracle (the only reference this paper has: it ships no code) on a bounded row sample of the same
+workload.
 """
 
 from __future__ import annotations
@@ -173,8 +176,77 @@ def run_reference(args, c):
 
 
 # --------------------------------------------------------------------------------------------
+# launcher: N ranks on one node
+# --------------------------------------------------------------------------------------------
+def _free_port() -> int:
+    import socket
+
+    s = socket.socket()
+    s.bind(("127.0.0.1", 0))
+    port = s.getsockname()[1]
+    s.close()
+    return port
+
+
+def spawn_command(nproc: int, argv: list[str], port: int) -> list[str]:
+    return [sys.executable, "-m", "torch.distributed.run", "--nnodes=1", f"--nproc-per-node={nproc}",
+            "--master-addr", "127.0.0.1", "--master-port", str(port), os.path.abspath(__file__), *argv]
+
+
+def maybe_spawn(args, argv: list[str]) -> None:
+    """--gpus N > 1 outside torchrun: re-exec this script under torch.distributed.run (one rank per
+    GPU); rank 0 prints the one JSON line.  Exits with the launcher's return code."""
+    if args.gpus <= 1 or "WORLD_SIZE" in os.environ or args.impl == "reference":
+        return
+    raise SystemExit(subprocess.call(spawn_command(args.gpus, argv, _free_port())))
+
+
+def max_over_ranks(vals: list[float], device) -> list[float]:
+    """Element-wise max over the ranks (device-timed numbers: the job is as slow as its slowest rank)."""
+    import torch
+    import torch.distributed as dist
+
+    t = torch.tensor(vals, dtype=torch.float64, device=device)
+    if dist.is_initialized() and dist.get_world_size() > 1:
+        dist.all_reduce(t, op=dist.ReduceOp.MAX)
+    return [float(x) for x in t.cpu()]
+
+
+def run_launcher_selftest(args):
+    """CPU check of the launcher and the max-over-ranks merge (gloo, no GPU): every rank reports a
+    rank-dependent fake time; rank 0 prints one JSON line with the max."""
+    import torch.distributed as dist
+
+    world = int(os.environ.get("WORLD_SIZE", "1"))
+    rank = int(os.environ.get("RANK", "0"))
+    if world > 1:
+        dist.init_process_group("gloo")
+    ms = max_over_ranks([10.0 + rank], "cpu")[0]
+    if rank == 0:
+        print(json.dumps({"metric": METRIC, "value": ms / 1e3, "unit": "s", "n_gpus": world, "steps": args.steps,
+                          "warmup": args.warmup, "ms_per_step": ms, "selftest": True}), flush=True)
+    if world > 1:
+        dist.barrier()
+        dist.destroy_process_group()
+
+
+# --------------------------------------------------------------------------------------------
 # our arm
 # --------------------------------------------------------------------------------------------
+def kernels_per_step(rs, h, A, q, perm, Q, R) -> int:
+    """Kernel launches of one step, counted by the library's launchers on an un-captured run of the
+    same phases (a graph replay re-launches exactly these kernels)."""
+    import torch
+
+    n0 = rs.kernel_launches()
+    rs.sample(h, A)
+    rs.power_iterate(h, A, q)
+    rs.pivot(h, perm)
+    rs.factor(h, A, Q, R)
+    torch.cuda.synchronize()
+    return rs.kernel_launches() - n0
+
+
 def run_ours(args, c):
     import torch
     import torch.distributed as dist
@@ -203,17 +275,18 @@ def run_ours(args, c):
         uid = [rs.rs_lowrank.comm_get_unique_id() if rank == 0 else None]
         dist.broadcast_object_list(uid, src=0)
         comm = rs.rs_lowrank.comm_init(world, uid[0], rank)
+        nr, rr = rs.rs_lowrank.comm_info(comm)
+        if nr != world or rr != rank:
+            raise SystemExit(f"NCCL communicator has nranks={nr} rank={rr}, expected {world}/{rank}")
+        print(f"[rank {rank}] NCCL communicator: nranks={nr} rank={rr}", file=sys.stderr, flush=True)
     stream = torch.cuda.Stream(device=dev)
     h = rs.create(m, ml, r0, n, k, p, c["omega_seed"], device=dev, stream=stream, nccl_comm=comm)
     perm = torch.empty(n, dtype=torch.int64, device=dev)
     Q = rs.empty_colmajor(ml, k, device=dev)
     R = rs.empty_colmajor(k, n, device=dev)
 
-    def step():
-        rs.sample(h, A)
-        rs.power_iterate(h, A, q)
-        rs.pivot(h, perm)
-        rs.factor(h, A, Q, R)
+    def step():   # the whole step as one CUDA-graph replay (rs_lowrank_run)
+        rs.run(h, A, q, perm, Q, R)
 
     torch.cuda.synchronize()
     for _ in range(args.warmup):
@@ -221,6 +294,9 @@ def run_ours(args, c):
     torch.cuda.synchronize()
     rs.reset_profile(h)
     rs.set_profiling(h, True)
+    step()   # re-capture with the profiling event nodes (untimed)
+    torch.cuda.synchronize()
+    rs.reset_profile(h)
     launches0 = rs.kernel_launches()
     if world > 1:
         dist.barrier()
@@ -234,16 +310,14 @@ def run_ours(args, c):
         torch.cuda.synchronize()
     if world > 1:
         dist.barrier()
-    launches = rs.kernel_launches() - launches0
     rs.set_profiling(h, False)
     ms_local = e0.elapsed_time(e1)
     prof = rs.get_profile(h)
+    # kernels launched in the timed region: the graph replays them; count one un-captured step
+    launches = args.steps * kernels_per_step(rs, h, A, q, perm, Q, R)
     gemm_names = ("gemm_sample", "gemm_power_c", "gemm_power_b")
     gemm_ms_local = sum(prof[g]["ms"] for g in gemm_names)
-    vec = torch.tensor([ms_local, gemm_ms_local], dtype=torch.float64, device=dev)
-    if world > 1:
-        dist.all_reduce(vec, op=dist.ReduceOp.MAX)
-    ms_total, gemm_ms_max = float(vec[0]), float(vec[1])
+    ms_total, gemm_ms_max = max_over_ranks([ms_local, gemm_ms_local], dev)
     ms_step = ms_total / args.steps
 
     # accuracy of the last approximation (evaluation only, outside the timed region)
@@ -349,6 +423,8 @@ def run_ours(args, c):
         "clocks": clk.summary(),
         "e2e": e2e,
         "gpu_launches": int(launches),
+        "step_api": "rs_lowrank_run (CUDA graph replay)",
+        "nccl": {"nranks": world, "checked": "rs_comm_info == WORLD_SIZE on every rank"} if world > 1 else None,
         "cpu_baseline": cpu,
     }
     print(json.dumps(line), flush=True)
@@ -371,7 +447,12 @@ def main():
     ap.add_argument("--no-e2e", action="store_true")
     ap.add_argument("--e2e-steps", type=int, default=2)
     ap.add_argument("--no-cpu-baseline", action="store_true")
+    ap.add_argument("--launcher-selftest", action="store_true", help=argparse.SUPPRESS)
     args = ap.parse_args()
+    maybe_spawn(args, sys.argv[1:])
+    if args.launcher_selftest:
+        run_launcher_selftest(args)
+        return
     if args.warmup < 3:
         args.warmup = 3
     c = workload(args.workload)

@@ -26,9 +26,12 @@
  *    (m_local rows starting at global row row_offset).  Omega is keyed by GLOBAL row index, so
  *    the result does not depend on the partition (up to summation order).  B and R are
  *    replicated on every rank, Q is row-distributed like A.
- *  - Every call enqueues work on the handle's CUDA stream.  sample and power_iterate do not
- *    synchronise; pivot and factor synchronise the stream before returning so that device-side
- *    failures (Cholesky breakdown, zero pivot norm) can be reported (cuSOLVER devInfo style).
+ *  - Every call enqueues work on the handle's CUDA stream.  sample and power_iterate never
+ *    synchronise the host (a CholQR breakdown inside the power iteration is flagged on the device
+ *    and handled by pivot, see there); pivot and factor synchronise the stream before returning
+ *    so that device-side failures (Cholesky breakdown, zero pivot norm) can be reported
+ *    (cuSOLVER devInfo style).  rs_lowrank_run does the whole step as one CUDA-graph replay with
+ *    a single synchronisation.
  *  - Ownership: the caller owns A, Q, R, perm and the workspace (allocate them with any device
  *    allocator); the library never frees them.  A must stay unmodified from sample through
  *    factor (it is re-read by power_iterate and factor).  The handle owns only host state.
@@ -90,12 +93,17 @@ RS_API rs_status_t rs_lowrank_create(rs_lowrank_t* h, int64_t m_global, int64_t 
 RS_API rs_status_t rs_lowrank_sample(rs_lowrank_t h, const double* A, int64_t lda);
 
 /* q passes of the power method with CholQR2 re-orthonormalisation of B and C (Fig. 2(a)).
- * q = 0 is a no-op.  No orthonormalisation after the last B := C A.                         */
+ * q = 0 is a no-op.  No orthonormalisation after the last B := C A.  Enqueues only: the sample
+ * B is kept, and if a CholQR of some pass breaks down (kappa^2 u > 1, "unstable for an
+ * ill-conditioned matrix") pivot redoes the iteration from it -- re-reading A, which
+ * must still be valid -- with the shifted-CholQR fallback of DESIGN.md R20.  At most once per
+ * sample (RS_ERR_BAD_STATE otherwise).                                                        */
 RS_API rs_status_t rs_lowrank_power_iterate(rs_lowrank_t h, const double* A, int64_t lda, int32_t q);
 
 /* Step 2: truncated QRCP of B (k steps, largest residual column norm, ties -> lowest index)
  * and T := R^_{1:k}^{-1} R^_{k+1:n}.  perm (device int64[n], may be NULL) receives P:
- * perm[0..k) are the pivot columns, perm[k..n) the rest in LAPACK swap order.  Synchronises. */
+ * perm[0..k) are the pivot columns, perm[k..n) the rest in LAPACK swap order.  Synchronises;
+ * reports (and recovers from) a breakdown of the preceding power_iterate as described there. */
 RS_API rs_status_t rs_lowrank_pivot(rs_lowrank_t h, int64_t* perm);
 
 /* Step 3: Q := orth(A(:, P_{1:k})) by CholQR2 (Q: m_local x k, ldq >= m_local, even) and
@@ -103,8 +111,17 @@ RS_API rs_status_t rs_lowrank_pivot(rs_lowrank_t h, int64_t* perm);
 RS_API rs_status_t rs_lowrank_factor(rs_lowrank_t h, const double* A, int64_t lda, double* Q, int64_t ldq, double* R,
                               int64_t ldr);
 
+/* The whole step sample -> power_iterate(q) -> pivot -> factor (CholQR2) with the arguments of
+ * those calls (perm: device int64[n] or NULL).  The first call with a given set of pointers and q
+ * captures the step as a CUDA graph on the handle's stream (kernels and NCCL collectives); later
+ * calls replay it: one launch and one synchronisation per step.  If the step saw a CholQR
+ * breakdown it is redone through the phase calls with their fallbacks.  Not captured when an
+ * allreduce hook is installed (the hook runs host code).  Synchronises; state as after factor. */
+RS_API rs_status_t rs_lowrank_run(rs_lowrank_t h, const double* A, int64_t lda, int32_t q, int64_t* perm, double* Q,
+                                  int64_t ldq, double* R, int64_t ldr);
+
 /* End-to-end call with HOST buffers: copies A (m_local x n, lda, host) to the device buffer
- * A_dev (ld_dev), runs sample -> power_iterate(q) -> pivot -> factor, and copies perm (int64[n]),
+ * A_dev (ld_dev), runs rs_lowrank_run (sample -> power_iterate(q) -> pivot -> factor), and copies perm (int64[n]),
  * Q (m_local x k, ldq) and R (k x n, ldr) back to host memory.  Host buffers should be pinned
  * for full PCIe bandwidth.  Q_dev (m_local x k, even ld_qdev) and R_dev (k x n, even ld_rdev)
  * are device scratch for the outputs.  Synchronises.                                          */
@@ -208,6 +225,8 @@ RS_API rs_status_t rs_qp3_truncated(int64_t m, int64_t n, int32_t k, double* A, 
 RS_API rs_status_t rs_comm_get_unique_id(char id_out[128]);
 RS_API rs_status_t rs_comm_init(void** comm, int32_t nranks, const char id[128], int32_t rank);
 RS_API rs_status_t rs_comm_destroy(void* comm);
+/* Number of ranks of a communicator (ncclCommCount) and this process's rank in it. */
+RS_API rs_status_t rs_comm_info(void* comm, int32_t* nranks, int32_t* rank);
 
 #ifdef __cplusplus
 }

@@ -132,19 +132,22 @@ def gaussian_pair(x, y):
     return (rho * c).astype(F32), (rho * s).astype(F32)
 
 
-def omega(ell: int, j0: int, j1: int, seed: int, tag: int = 0) -> np.ndarray:
+def omega(ell: int, j0: int, j1: int, seed: int, tag: int = 0, rows=None) -> np.ndarray:
     """Omega[:, j0:j1] (l x (j1-j0), float64): the Gaussian sampling matrix of
     Step 1, B = Omega A (Fig. 2(b) line 2), columns indexed
     by GLOBAL row j of A so every row-block partition sees the same Omega
-    (1-D block-column layout of Omega)."""
+    (1-D block-column layout of Omega).  ``rows`` (optional) selects
+    the Omega rows to generate (default 0..l-1): each entry depends only on its
+    own (row, column) counter."""
+    nrow = ell if rows is None else len(rows)
     if j1 <= j0:
-        return np.zeros((ell, 0))
+        return np.zeros((nrow, 0))
     t0, t1 = j0 // 4, (j1 + 3) // 4
     t = np.arange(t0, t1, dtype=np.uint64)[None, :]
-    i = np.arange(ell, dtype=np.uint64)[:, None]
+    i = (np.arange(ell, dtype=np.uint64) if rows is None else np.asarray(rows, dtype=np.uint64))[:, None]
     x0, x1, x2, x3 = philox4x32_10(t & MASK32, i, np.uint64(tag), t >> np.uint64(32),
                                    seed & 0xFFFFFFFF, (seed >> 32) & 0xFFFFFFFF)
     z0, z1 = gaussian_pair(x0, x1)
     z2, z3 = gaussian_pair(x2, x3)
-    full = np.stack([z0, z1, z2, z3], axis=-1).reshape(ell, -1).astype(np.float64)
+    full = np.stack([z0, z1, z2, z3], axis=-1).reshape(nrow, -1).astype(np.float64)
     return full[:, j0 - 4 * t0: j1 - 4 * t0]

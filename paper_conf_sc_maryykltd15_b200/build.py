@@ -50,7 +50,7 @@ def _hash(files):
     h = hashlib.sha256()
     for f in sorted(files):
         with open(f, "rb") as fh:
-            h.update(f.encode())
+            h.update(os.path.relpath(f, ROOT).encode())  # location-independent (the repo is copied to the GPU box)
             h.update(fh.read())
     return h.hexdigest()
 
@@ -62,8 +62,12 @@ def build(force: bool = False, verbose: bool = False) -> str:
     deps.append(os.path.abspath(__file__))
     extra = os.environ.get("RS_EXTRA_NVCC_FLAGS", "").split()  # development experiments only
     digest = _hash(deps) + ("|" + " ".join(extra) if extra else "")
-    if not force and os.path.exists(LIB) and os.path.exists(STAMP) and open(STAMP).read().strip() == digest:
-        return LIB
+    # the stamp (git-ignored) records the source digest AND the digest of the .so it was written
+    # with, so a .so replaced by another revision's (a sync, a checkout) is never taken as current
+    if not force and os.path.exists(LIB) and os.path.exists(STAMP):
+        with open(STAMP) as fh:
+            if fh.read().strip() == digest + ":" + _hash([LIB]):
+                return LIB
     os.makedirs(LIBDIR, exist_ok=True)
     nccl_inc, nccl_lib = _nccl_dirs()
     common = ["nvcc", *ARCH, "-O3", "-lineinfo", "-std=c++17", "-Xcompiler", "-fPIC", "-Xcompiler", "-fvisibility=hidden",
@@ -91,7 +95,7 @@ def build(force: bool = False, verbose: bool = False) -> str:
     for o in objs:
         os.remove(o)
     with open(STAMP, "w") as fh:
-        fh.write(digest)
+        fh.write(digest + ":" + _hash([LIB]))
     return LIB
 
 

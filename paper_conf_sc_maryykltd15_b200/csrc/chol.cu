@@ -621,26 +621,30 @@ cudaError_t chol_inv(cudaStream_t st, const double* G, int ldg, int n, int npad,
                      int ldl, double* gwork, int* info, int info_code) {
   if (n <= 0) return cudaSuccess;
   if (n > 512) return cudaErrorInvalidValue;
-  static const int smem_max_n = [] {  // RS_CHOL_SMEM_MAX_N: crossover experiments only
-    const char* v = getenv("RS_CHOL_SMEM_MAX_N");
-    return v ? atoi(v) : CH_SMEM_MAX_N;
-  }();
-  static const bool use_tile = getenv("RS_CHOL_BLOCKED") == nullptr;  // development switch
+  // compile-time development switches: -DRS_DEV_CHOL_SMEM_MAX_N=<n> (crossover experiments),
+  // -DRS_DEV_CHOL_BLOCKED (the blocked kernel for n <= 128), -DRS_DEV_CHOL_TPT=2 (two tiles per thread)
+#ifdef RS_DEV_CHOL_SMEM_MAX_N
+  constexpr int smem_max_n = RS_DEV_CHOL_SMEM_MAX_N;
+#else
+  constexpr int smem_max_n = CH_SMEM_MAX_N;
+#endif
+#ifdef RS_DEV_CHOL_BLOCKED
+  constexpr bool use_tile = false;
+#else
+  constexpr bool use_tile = true;
+#endif
   if (use_tile && n <= CT_MAXN) {
     const int nt = (n + 3) / 4;
-    static const int tpt = [] {  // RS_CHOL_TPT=2: development switch (two tiles per thread)
-      const char* v = getenv("RS_CHOL_TPT");
-      return v ? atoi(v) : 1;
-    }();
-    static bool attr_t = false;
+#ifdef RS_DEV_CHOL_TPT
+    constexpr int tpt = RS_DEV_CHOL_TPT;
+#else
+    constexpr int tpt = 1;
+#endif
     constexpr int ct_max_smem = ct_smem_doubles(CT_MAXN) * 8;
-    if (!attr_t) {
-      cudaError_t e = cudaSuccess;
-      for (auto fn : {chol_tile_kernel<1, 256>, chol_tile_kernel<1, 512>, chol_tile_kernel<1, 832>,
-                      chol_tile_kernel<1, 1024>, chol_tile_kernel<2, 576>})
-        if (e == cudaSuccess) e = cudaFuncSetAttribute(fn, cudaFuncAttributeMaxDynamicSharedMemorySize, ct_max_smem);
+    for (auto fn : {chol_tile_kernel<1, 256>, chol_tile_kernel<1, 512>, chol_tile_kernel<1, 832>,
+                    chol_tile_kernel<1, 1024>, chol_tile_kernel<2, 576>}) {
+      cudaError_t e = ensure_smem(fn, ct_max_smem);
       if (e != cudaSuccess) return e;
-      attr_t = true;
     }
     const size_t ct_smem = static_cast<size_t>(ct_smem_doubles(4 * nt)) * 8;
     // one tile per thread, in the smallest CTA that holds all nt (nt + 1) tiles: idle warps would
@@ -659,27 +663,22 @@ cudaError_t chol_inv(cudaStream_t st, const double* G, int ldg, int n, int npad,
   } else if (n <= smem_max_n && n <= CH_SMEM_MAX_N) {
     const int np = (n + CB - 1) / CB * CB;
     const size_t smem = static_cast<size_t>(np) * (np + 1) * 8;
-    static bool attr = false;
-    if (!attr) {
-      cudaError_t e = cudaFuncSetAttribute(chol_blocked_kernel<true>, cudaFuncAttributeMaxDynamicSharedMemorySize,
-                                           CH_SMEM_MAX_N * (CH_SMEM_MAX_N + 1) * 8);
+    {
+      cudaError_t e = ensure_smem(chol_blocked_kernel<true>, CH_SMEM_MAX_N * (CH_SMEM_MAX_N + 1) * 8);
       if (e != cudaSuccess) return e;
-      attr = true;
     }
     chol_blocked_kernel<true><<<1, CH_BLK_THREADS, smem, st>>>(G, ldg, n, R, ldr, Linv, ldl, gwork, info, info_code,
                                                                 npad);
   } else {  // one 8-CTA cluster on an L2-resident copy in the workspace (np x (np+1) + np doubles)
     const size_t smem = 2 * static_cast<size_t>(CB) * CHL_MAXN * 8;
-    static bool attr_l = false;
-    if (!attr_l) {
-      cudaError_t e = cudaFuncSetAttribute(chol_cluster_kernel, cudaFuncAttributeMaxDynamicSharedMemorySize,
-                                           static_cast<int>(smem));
+    {
+      cudaError_t e = ensure_smem(chol_cluster_kernel, static_cast<int>(smem));
       if (e != cudaSuccess) return e;
       if (CHL_CLUSTER > 8) {
-        e = cudaFuncSetAttribute(chol_cluster_kernel, cudaFuncAttributeNonPortableClusterSizeAllowed, 1);
+        e = ensure_func_attr(reinterpret_cast<const void*>(chol_cluster_kernel),
+                             cudaFuncAttributeNonPortableClusterSizeAllowed, 1);
         if (e != cudaSuccess) return e;
       }
-      attr_l = true;
     }
     const int np = (n + CB - 1) / CB * CB;
     cudaLaunchConfig_t cfg{};

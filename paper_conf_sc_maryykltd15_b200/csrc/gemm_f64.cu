@@ -2,12 +2,29 @@
 #include <algorithm>
 #include <cstdio>
 #include <cstdlib>
+#include <map>
 #include <mutex>
+#include <tuple>
 
 #include "gemm_f64.cuh"
 #include "internal.h"
 
 namespace rs {
+
+cudaError_t ensure_func_attr(const void* fn, cudaFuncAttribute attr, int value) {
+  static std::mutex mu;
+  static std::map<std::tuple<int, const void*, int>, int> done;  // (device, kernel, attribute) -> value set
+  int dev = 0;
+  cudaError_t e = cudaGetDevice(&dev);
+  if (e != cudaSuccess) return e;
+  std::lock_guard<std::mutex> lk(mu);
+  const auto key = std::make_tuple(dev, fn, static_cast<int>(attr));
+  auto it = done.find(key);
+  if (it != done.end() && it->second >= value) return cudaSuccess;
+  e = cudaFuncSetAttribute(fn, attr, value);
+  if (e == cudaSuccess) done[key] = value;
+  return e;
+}
 
 namespace {
 
@@ -62,26 +79,19 @@ template <int MFW>
 cudaError_t launch_kc_t(cudaStream_t st, dim3 grid, const CUtensorMap& tR, const CUtensorMap& tL, const GemmArgs& a) {
   constexpr int smem = KCSmem<MFW, false>::TOTAL;
   // producer warpgroup (default): with the producer sleeping in the slot wait (mbar_wait_sleep) the
-  // MMA warps no longer carry the TMA issue; cfg4 B = C~ A 32.07 -> 31.36 ms.  RS_KC_NO_PWG: TMA
-  // issued by thread 0 of MMA warp 0 (A/B switch)
-  static const bool pwg = getenv("RS_KC_NO_PWG") == nullptr;
-  if (pwg) {
-    static bool attr_p = false;
-    if (!attr_p) {
-      cudaError_t e = cudaFuncSetAttribute(kc_gemm_pwg_kernel<MFW>, cudaFuncAttributeMaxDynamicSharedMemorySize, smem);
-      if (e != cudaSuccess) return e;
-      attr_p = true;
-    }
+  // MMA warps no longer carry the TMA issue; cfg4 B = C~ A 32.07 -> 31.36 ms.  -DRS_DEV_KC_NO_PWG:
+  // TMA issued by thread 0 of MMA warp 0 (A/B switch)
+#ifndef RS_DEV_KC_NO_PWG
+  {
+    cudaError_t e = ensure_smem(kc_gemm_pwg_kernel<MFW>, smem);
+    if (e != cudaSuccess) return e;
     kc_gemm_pwg_kernel<MFW><<<grid, KCP_THREADS, smem, st>>>(tR, tL, a);
     count_launch();
     return cudaGetLastError();
   }
-  static bool attr_set = false;  // per-instantiation; races are benign (idempotent)
-  if (!attr_set) {
-    cudaError_t e = cudaFuncSetAttribute(kc_gemm_kernel<MFW>, cudaFuncAttributeMaxDynamicSharedMemorySize, smem);
-    if (e != cudaSuccess) return e;
-    attr_set = true;
-  }
+#endif
+  cudaError_t e = ensure_smem(kc_gemm_kernel<MFW>, smem);
+  if (e != cudaSuccess) return e;
   kc_gemm_kernel<MFW><<<grid, GEMM_THREADS, smem, st>>>(tR, tL, a);
   count_launch();
   return cudaGetLastError();
@@ -90,12 +100,9 @@ cudaError_t launch_kc_t(cudaStream_t st, dim3 grid, const CUtensorMap& tR, const
 template <int MFW, int CS>
 cudaError_t launch_phx_cs(cudaStream_t st, dim3 grid, const CUtensorMap& tR, const GemmArgs& a) {
   constexpr int smem = KCSmem<MFW, true>::TOTAL;
-  static bool attr_set = false;
-  if (!attr_set) {
-    cudaError_t e =
-        cudaFuncSetAttribute(kc_philox_kernel<MFW, CS>, cudaFuncAttributeMaxDynamicSharedMemorySize, smem);
+  {
+    cudaError_t e = ensure_smem(kc_philox_kernel<MFW, CS>, smem);
     if (e != cudaSuccess) return e;
-    attr_set = true;
   }
   grid.x = (grid.x + CS - 1) / CS * CS;  // whole clusters along N (extra CTAs store nothing)
   cudaLaunchConfig_t cfg = {};
@@ -115,15 +122,12 @@ cudaError_t launch_phx_cs(cudaStream_t st, dim3 grid, const CUtensorMap& tR, con
   return e != cudaSuccess ? e : cudaGetLastError();
 }
 
-// Cluster size for Omega sharing (RS_PHILOX_CLUSTER = 1, 2 or 4; default 2).
-int philox_cluster() {
-  static int cs = [] {
-    const char* v = getenv("RS_PHILOX_CLUSTER");
-    const int c = v ? atoi(v) : 2;
-    return (c == 1 || c == 2 || c == 4) ? c : 2;
-  }();
-  return cs;
-}
+// Cluster size for Omega sharing (-DRS_DEV_PHILOX_CLUSTER=1, 2 or 4; default 2).
+#ifndef RS_DEV_PHILOX_CLUSTER
+#define RS_DEV_PHILOX_CLUSTER 2
+#endif
+constexpr int philox_cluster() { return RS_DEV_PHILOX_CLUSTER; }
+static_assert(philox_cluster() == 1 || philox_cluster() == 2 || philox_cluster() == 4, "Philox cluster size");
 
 template <int MFW>
 cudaError_t launch_phx_t(cudaStream_t st, dim3 grid, const CUtensorMap& tR, const GemmArgs& a) {
@@ -140,23 +144,19 @@ cudaError_t launch_phx_t(cudaStream_t st, dim3 grid, const CUtensorMap& tR, cons
 template <int MFW, int WM>
 cudaError_t launch_mc_wm(cudaStream_t st, dim3 grid, const CUtensorMap& tL, const CUtensorMap& tR, const GemmArgs& a) {
   constexpr int smem = MCSmem<MFW, WM>::TOTAL;
-  static bool attr_set = false;
-  if (!attr_set) {
-    for (auto fn : {mc_gemm_kernel<MFW, WM, 0>, mc_gemm_kernel<MFW, WM, 1>, mc_gemm_kernel<MFW, WM, 2>}) {
-      cudaError_t e = cudaFuncSetAttribute(fn, cudaFuncAttributeMaxDynamicSharedMemorySize, smem);
-      if (e != cudaSuccess) return e;
-    }
-    attr_set = true;
+  for (auto fn : {mc_gemm_kernel<MFW, WM, 0>, mc_gemm_kernel<MFW, WM, 1>, mc_gemm_kernel<MFW, WM, 2>}) {
+    cudaError_t e = ensure_smem(fn, smem);
+    if (e != cudaSuccess) return e;
   }
-  // dense 1x8 products (C = B~ A^T): dedicated producer warpgroup; RS_MC_NO_PWG: A/B switch
-  static const bool pwg = getenv("RS_MC_NO_PWG") == nullptr;
+  // dense 1x8 products (C = B~ A^T): dedicated producer warpgroup; -DRS_DEV_MC_NO_PWG: A/B switch
+#ifdef RS_DEV_MC_NO_PWG
+  constexpr bool pwg = false;
+#else
+  constexpr bool pwg = true;
+#endif
   if (WM == 1 && a.tri == 0 && pwg) {
-    static bool attr_p = false;
-    if (!attr_p) {
-      cudaError_t e = cudaFuncSetAttribute(mc_gemm_pwg_kernel<MFW, WM, 0>, cudaFuncAttributeMaxDynamicSharedMemorySize, smem);
-      if (e != cudaSuccess) return e;
-      attr_p = true;
-    }
+    cudaError_t e = ensure_smem(mc_gemm_pwg_kernel<MFW, WM, 0>, smem);
+    if (e != cudaSuccess) return e;
     mc_gemm_pwg_kernel<MFW, WM, 0><<<grid, KCP_THREADS, smem, st>>>(tL, tR, a);
     count_launch();
     return cudaGetLastError();
@@ -175,13 +175,9 @@ template <int MFW>
 cudaError_t launch_mcp_t(cudaStream_t st, int grid, const CUtensorMap& tL, const CUtensorMap& tR, const GemmArgs& a,
                          int ntn, int ntiles, int res_l) {
   constexpr int smem = MCPSmem<MFW>::TOTAL;
-  static bool attr_set = false;
-  if (!attr_set) {
-    for (auto fn : {mc_persist_kernel<MFW, 0>, mc_persist_kernel<MFW, 1>, mc_persist_kernel<MFW, 2>}) {
-      cudaError_t e = cudaFuncSetAttribute(fn, cudaFuncAttributeMaxDynamicSharedMemorySize, smem);
-      if (e != cudaSuccess) return e;
-    }
-    attr_set = true;
+  for (auto fn : {mc_persist_kernel<MFW, 0>, mc_persist_kernel<MFW, 1>, mc_persist_kernel<MFW, 2>}) {
+    cudaError_t e = ensure_smem(fn, smem);
+    if (e != cudaSuccess) return e;
   }
   if (a.tri == 1)
     mc_persist_kernel<MFW, 1><<<grid, GEMM_THREADS, smem, st>>>(tL, tR, a, ntn, ntiles, res_l);
@@ -242,14 +238,11 @@ void mcp_nmap(GemmArgs& a, int N, long long K, int ntn) {
 // and 32 columns; (MFW/2 + 2) instead of (MFW + 1) LDS.128 per 4 MFW DMMAs) measured slower at
 // cfg4 for C = B A^T (MFW = 7): 34.4 ms vs 33.5 ms with 1 x 8 (an earlier box-granular uneven
 // split: 35.8 ms).  Short-K triangular products (and the persistent kernel): 2 x 4, measured
-// faster for the L^-1 C apply (0.93 vs 1.18 ms at cfg4).  RS_MC_WM = 1 / 2 forces a grid.
-static inline int mc_wm_override() {
-  static const int v = [] {
-    const char* e = getenv("RS_MC_WM");  // development switch: 1 or 2
-    return e ? atoi(e) : 0;
-  }();
-  return v;
-}
+// faster for the L^-1 C apply (0.93 vs 1.18 ms at cfg4).  -DRS_DEV_MC_WM=1 / 2 forces a grid.
+#ifndef RS_DEV_MC_WM
+#define RS_DEV_MC_WM 0
+#endif
+constexpr int mc_wm_override() { return RS_DEV_MC_WM; }
 template <int MFW>
 cudaError_t launch_mc_t(cudaStream_t st, dim3 grid, const CUtensorMap& tL, const CUtensorMap& tR, const GemmArgs& a) {
   if constexpr (MFW < 3) {
@@ -264,11 +257,9 @@ cudaError_t launch_mc_t(cudaStream_t st, dim3 grid, const CUtensorMap& tL, const
 template <int R>
 cudaError_t launch_syrk_t(cudaStream_t st, dim3 grid, const CUtensorMap& tX, const GemmArgs& a) {
   constexpr int smem = SyrkSmem<R>::TOTAL;
-  static bool attr_set = false;
-  if (!attr_set) {
-    cudaError_t e = cudaFuncSetAttribute(syrk_kernel<R>, cudaFuncAttributeMaxDynamicSharedMemorySize, smem);
+  {
+    cudaError_t e = ensure_smem(syrk_kernel<R>, smem);
     if (e != cudaSuccess) return e;
-    attr_set = true;
   }
   syrk_kernel<R><<<grid, GEMM_THREADS, smem, st>>>(tX, a);
   count_launch();
@@ -353,11 +344,6 @@ cudaError_t gemm_kc(cudaStream_t st, int M, int N, long long K, const View2D& Lv
     a.row_offset = phx.row_offset;
     a.ell = phx.ell;
     a.omega_row0 = phx.omega_row0;
-    static const int gen_mode = [] {  // RS_PHILOX_GENMODE: cost experiments only (results invalid)
-      const char* v = getenv("RS_PHILOX_GENMODE");
-      return v ? atoi(v) : 0;
-    }();
-    a.gen_mode = gen_mode;
   }
   CUtensorMap tR, tL;
   if (!make_tmap(&tR, Rv, 16, NT)) return cudaErrorInvalidValue;
@@ -387,14 +373,22 @@ cudaError_t gemm_mc(cudaStream_t st, int M, int N, long long K, const View2D& Lv
   a.tri = tri;
   const long long nsplit = (K + a.k_chunk - 1) / a.k_chunk;
   CUtensorMap tL, tR;
-  static const bool no3d = getenv("RS_MC_NO_TMA3D") != nullptr;  // development switch
+#ifdef RS_DEV_MC_NO_TMA3D
+  constexpr bool no3d = true;
+#else
+  constexpr bool no3d = false;
+#endif
   a.l3d = !no3d && make_tmap3(&tL, Lv, static_cast<uint32_t>(MT / 16));
   a.r3d = !no3d && make_tmap3(&tR, Rv, static_cast<uint32_t>(NT / 16));
   if (!a.l3d && !make_tmap(&tL, Lv, 16, 16)) return cudaErrorInvalidValue;
   if (!a.r3d && !make_tmap(&tR, Rv, 16, 16)) return cudaErrorInvalidValue;
   dim3 grid((N + NT - 1) / NT, (M + MT - 1) / MT, static_cast<unsigned>(nsplit < 1 ? 1 : nsplit));
   // short K and many tiles: persistent CTAs (the ring runs on across tiles)
-  static const bool no_persist = getenv("RS_MC_NO_PERSIST") != nullptr;  // development switch
+#ifdef RS_DEV_MC_NO_PERSIST
+  constexpr bool no_persist = true;
+#else
+  constexpr bool no_persist = false;
+#endif
   const long long ntiles = static_cast<long long>(grid.x) * grid.y;
   // (one of the two operands must be shared by every tile: a single M tile or a single N tile)
   // (measured: at 391 tiles (m = 50 000) the resident-operand start-up costs more than it saves;

@@ -60,7 +60,6 @@ struct GemmArgs {
   long long row_offset;
   long long omega_row0;  // first Omega row of this tile set (adaptive rounds draw rows [l, l + l_inc))
   int ell;               // number of Omega rows generated (rows >= ell of the tile are zero)
-  int gen_mode;  // 0 = Philox + RS-BM32 (production); 1, 2 = generation-cost experiments only
   int tri;       // MC: 0 dense, 1 L lower triangular, 2 R upper triangular (zero blocks skipped)
   unsigned long long nmap;  // persistent MC: N box of warp column wn, slot nb = byte 2 wn + nb
   int l3d, r3d;  // MC: operand tensor map is the 3-D stacked-box form (one TMA per stage), see mc_load
@@ -384,17 +383,7 @@ __global__ void __launch_bounds__(PHX_THREADS, 1)
         const int gi = m0 + lrow;
         double* dst = reinterpret_cast<double*>(sL + s * SM::L_BYTES) + lrow * PHX_LD + 4 * q;
         double v0 = 0.0, v1 = 0.0, v2 = 0.0, v3 = 0.0;
-        if (a.gen_mode != 0) {  // experiments: 1 = Philox words only, 2 = no generation
-          if (a.gen_mode == 1 && gi < a.ell) {
-            uint32_t c0 = static_cast<uint32_t>(t0 + q), c1 = static_cast<uint32_t>(gi), c2 = a.tag,
-                     c3 = static_cast<uint32_t>((t0 + q) >> 32);
-            philox4x32_10(c0, c1, c2, c3, a.key);
-            v0 = static_cast<int>(c0) * 0x1p-31, v1 = static_cast<int>(c1) * 0x1p-31;
-            v2 = static_cast<int>(c2) * 0x1p-31, v3 = static_cast<int>(c3) * 0x1p-31;
-          } else if (gi < a.ell) {
-            v0 = v1 = v2 = v3 = 1.0;
-          }
-        } else if (gi < a.ell) {
+        if (gi < a.ell) {
           const float4 z = omega_block4f(static_cast<uint32_t>(a.omega_row0 + gi), t0 + q, a.tag, a.key);
           if (o == 0) {
             v0 = z.x, v1 = z.y, v2 = z.z, v3 = z.w;

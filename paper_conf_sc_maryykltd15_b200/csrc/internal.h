@@ -47,6 +47,18 @@ int gemm_choose_splits(int M, int N, long long K, int max_splits, int num_sms);
 int gemm_nsplit(long long K, int splits);   // splits actually launched for a requested count
 int gemm_mtile(int M);   // rows per CTA tile used for M
 
+// cudaFuncSetAttribute(fn, attr, value) once per (device, kernel, attribute, value).  Function
+// attributes belong to the device context, so a per-process "done" flag would skip them when a
+// process drives a second GPU; a value above the one already set is applied again.
+cudaError_t ensure_func_attr(const void* fn, cudaFuncAttribute attr, int value);
+template <typename F>
+inline cudaError_t ensure_smem(F* fn, int bytes) {
+  return ensure_func_attr(reinterpret_cast<const void*>(fn), cudaFuncAttributeMaxDynamicSharedMemorySize, bytes);
+}
+
+// Development A/B switches are COMPILE-TIME only (RS_EXTRA_NVCC_FLAGS="-DRS_DEV_..."): the shipped
+// library reads no environment variable.
+
 // kernel launch accounting (every launcher calls count_launch once per kernel launch)
 void count_launch();
 long long launch_count();

@@ -1015,14 +1015,12 @@ template <int ROWS, int THREADS>
 cudaError_t launch_qrcp_cluster(cudaStream_t st, int NB, const double* B, int ldb, int ell, long long n, int k,
                                 int cols_per, int64_t* piv, double* Rho, int ldr, double* gaps, int* info) {
   constexpr int dsmem = 2 * QRC_MAXNB * 4 * ROWS * 8;
-  static bool attr = false;
-  if (!attr) {
-    cudaError_t e = cudaFuncSetAttribute(qrcp_cluster_kernel<ROWS, THREADS>,
-                                         cudaFuncAttributeNonPortableClusterSizeAllowed, 1);
+  {
+    cudaError_t e = ensure_func_attr(reinterpret_cast<const void*>(qrcp_cluster_kernel<ROWS, THREADS>),
+                                     cudaFuncAttributeNonPortableClusterSizeAllowed, 1);
     if (e != cudaSuccess) return e;
-    e = cudaFuncSetAttribute(qrcp_cluster_kernel<ROWS, THREADS>, cudaFuncAttributeMaxDynamicSharedMemorySize, dsmem);
+    e = ensure_smem(qrcp_cluster_kernel<ROWS, THREADS>, dsmem);
     if (e != cudaSuccess) return e;
-    attr = true;
   }
   cudaLaunchConfig_t cfg{};
   cfg.gridDim = dim3(NB, 1, 1);
@@ -1061,7 +1059,13 @@ size_t qrcp_workspace_bytes(int ell, long long n) {
 cudaError_t qrcp_truncated(cudaStream_t st, const double* B, int ldb, int ell, long long n, int k, void* work,
                            int64_t* perm, double* Rho, int ldr, double* gaps, int* info, int num_sms) {
   if (n >= (1LL << 31)) return cudaErrorInvalidValue;  // column indices ride in 32-bit REDUX keys
-  static const bool force_smem = getenv("RS_QRCP_SMEM") != nullptr;  // development switch
+  // compile-time development switches: -DRS_DEV_QRCP_SMEM (shared-memory kernel), _NO_CLUSTER,
+  // _TIMING (per-phase cycle counts of CTA 0 to stderr), _BARRIER, _LPC4, _POLL
+#ifdef RS_DEV_QRCP_SMEM
+  constexpr bool force_smem = true;
+#else
+  constexpr bool force_smem = false;
+#endif
   const bool use_reg = !force_smem && ell <= 4 * QRR_ROWS && (n + QRR_COLS - 1) / QRR_COLS <= num_sms;
   int cols_per = use_reg ? QRR_COLS : QR_MAX_COLS;
   while (!use_reg && cols_per > 1 && qr_smem(cols_per, ell) > QR_SMEM_MAX) --cols_per;
@@ -1070,20 +1074,20 @@ cudaError_t qrcp_truncated(cudaStream_t st, const double* B, int ldb, int ell, l
   if (!use_reg) cols_per = static_cast<int>((n + NB - 1) / NB);  // balance
   const size_t smem = use_reg ? 0 : qr_smem(cols_per, ell);
   const int ldw = qr_ldw(ell);
-  static bool attr = false;
-  if (!attr) {
-    cudaError_t e = cudaFuncSetAttribute(qrcp_kernel, cudaFuncAttributeMaxDynamicSharedMemorySize,
-                                         static_cast<int>(QR_SMEM_MAX));
+  {
+    cudaError_t e = ensure_smem(qrcp_kernel, static_cast<int>(QR_SMEM_MAX));
     if (e != cudaSuccess) return e;
-    e = cudaFuncSetAttribute(qrcp_perm_kernel, cudaFuncAttributeMaxDynamicSharedMemorySize,
-                             static_cast<int>(QR_SMEM_MAX));
+    e = ensure_smem(qrcp_perm_kernel, static_cast<int>(QR_SMEM_MAX));
     if (e != cudaSuccess) return e;
-    attr = true;
   }
   QrWork* w = static_cast<QrWork*>(work);
   {
     // cluster path: l <= 64 with <= 160 columns per CTA, or l <= 128 with <= 128, over <= 16 CTAs
-    static const bool no_cluster = getenv("RS_QRCP_NO_CLUSTER") != nullptr;  // development switch
+#ifdef RS_DEV_QRCP_NO_CLUSTER
+    constexpr bool no_cluster = true;
+#else
+    constexpr bool no_cluster = false;
+#endif
     const int rows = ell <= 64 ? 16 : 32;
     const int maxc = rows == 16 ? 160 : 128;
     const int nbc = static_cast<int>((n + maxc - 1) / maxc);
@@ -1105,12 +1109,19 @@ cudaError_t qrcp_truncated(cudaStream_t st, const double* B, int ldb, int ell, l
       if (ec != cudaErrorNotSupported) return ec;
     }
   }
-  // RS_QRCP_TIMING=1: per-phase cycle counts of CTA 0 printed to stderr (development aid)
+  // -DRS_DEV_QRCP_TIMING: per-phase cycle counts of CTA 0 printed to stderr (development aid)
+#ifdef RS_DEV_QRCP_TIMING
   static long long* tbuf = nullptr;
-  static const bool timing = getenv("RS_QRCP_TIMING") != nullptr;
-  if (timing && !tbuf && cudaMalloc(&tbuf, 8 * 8 * 1024) != cudaSuccess) tbuf = nullptr;
-  long long* tb = (timing && k <= 1024) ? tbuf : nullptr;
+  if (!tbuf && cudaMalloc(&tbuf, 8 * 8 * 1024) != cudaSuccess) tbuf = nullptr;
+  long long* tb = k <= 1024 ? tbuf : nullptr;
+#else
+  long long* tb = nullptr;
+#endif
   auto report = [&](const char* what, int nb, int cols) {
+#ifndef RS_DEV_QRCP_TIMING
+    (void)what, (void)nb, (void)cols;
+    return;
+#else
     if (!tb) return;
     static long long h[8 * 1024];
     cudaStreamSynchronize(st);
@@ -1124,13 +1135,22 @@ cudaError_t qrcp_truncated(cudaStream_t st, const double* B, int ldb, int ell, l
             "tail=%.0f\n",
             what, nb, cols, acc[0] / (k - 1), acc[1] / (k - 1), acc[2] / (k - 1), acc[3] / (k - 1), acc[4] / (k - 1),
             acc[5] / (k - 1), acc[6] / (k - 1));
+#endif
   };
   {
     // flag-synchronised register kernel: 8 lanes per column when n <= NBmax x 64, else 4
-    static const bool barrier_kernel = getenv("RS_QRCP_BARRIER") != nullptr;  // development switch
+#ifdef RS_DEV_QRCP_BARRIER
+    constexpr bool barrier_kernel = true;
+#else
+    constexpr bool barrier_kernel = false;
+#endif
     const int nbmax = std::min(num_sms, QRF_MAXNB);
     const int nb8 = static_cast<int>((n + 63) / 64), nb4 = static_cast<int>((n + 127) / 128);
-    static const bool force4 = getenv("RS_QRCP_LPC4") != nullptr;  // development switch
+#ifdef RS_DEV_QRCP_LPC4
+    constexpr bool force4 = true;
+#else
+    constexpr bool force4 = false;
+#endif
     const int lpc = (nb8 <= nbmax && !force4) ? 8 : (nb4 <= nbmax ? 4 : 0);
     if (!barrier_kernel && !force_smem && ell <= 128 && lpc) {
       const int nbf = lpc == 8 ? nb8 : nb4;
@@ -1139,7 +1159,11 @@ cudaError_t qrcp_truncated(cudaStream_t st, const double* B, int ldb, int ell, l
       int64_t* pv = reinterpret_cast<int64_t*>(ccol + 2 * static_cast<size_t>(nbf) * QRF_CST);
       cudaError_t e = cudaMemsetAsync(work, 0, sizeof(QrWork) + 2 * static_cast<size_t>(nbf) * sizeof(QrRec), st);
       if (e != cudaSuccess) return e;
-      static const bool poll_records = getenv("RS_QRCP_POLL") != nullptr;  // development switch
+#ifdef RS_DEV_QRCP_POLL
+      constexpr bool poll_records = true;
+#else
+      constexpr bool poll_records = false;
+#endif
       unsigned int* counter = poll_records ? nullptr : &w->count;
       void* fargs[] = {(void*)&B,   (void*)&ldb, (void*)&ell, (void*)&n,   (void*)&k,    (void*)&rec,
                        (void*)&ccol, (void*)&nbf, (void*)&pv, (void*)&Rho, (void*)&ldr, (void*)&gaps,
@@ -1172,12 +1196,8 @@ cudaError_t qrcp_truncated(cudaStream_t st, const double* B, int ldb, int ell, l
     void* rargs[] = {(void*)&B,   (void*)&ldb, (void*)&ell, (void*)&n,    (void*)&k,    (void*)&w, (void*)&NB,
                      (void*)&piv, (void*)&Rho, (void*)&ldr, (void*)&gaps, (void*)&info, (void*)&tb};
     const size_t rsmem = (4 * static_cast<size_t>(NB) + static_cast<size_t>(NB) * ell) * 8;
-    static size_t rsmem_set = 0;
-    if (rsmem > rsmem_set) {
-      e = cudaFuncSetAttribute(qrcp_reg_kernel, cudaFuncAttributeMaxDynamicSharedMemorySize, static_cast<int>(rsmem));
-      if (e != cudaSuccess) return e;
-      rsmem_set = rsmem;
-    }
+    e = ensure_smem(qrcp_reg_kernel, static_cast<int>(rsmem));
+    if (e != cudaSuccess) return e;
     e = cudaLaunchCooperativeKernel(reinterpret_cast<void*>(qrcp_reg_kernel), dim3(NB), dim3(QRR_THREADS), rargs,
                                     rsmem, st);
   } else {

@@ -21,6 +21,10 @@ namespace {
 
 enum State { ST_CREATED = 0, ST_SAMPLED = 1, ST_PIVOTED = 2, ST_FACTORED = 3 };
 
+// internal device info code: CholQR breakdown in power-iteration pass (code - RS_INFO_POWER),
+// never returned to the caller (pivot replays the iteration with the R20 fallback)
+constexpr int RS_INFO_POWER = 100;
+
 inline long long round_up(long long x, long long a) { return (x + a - 1) / a * a; }
 
 struct ProfEntry {
@@ -41,7 +45,7 @@ struct Layout {
   long long ldc, ldq1;
   int smax;          // max split-K partial tiles of an l x n product
   long long part_elems;
-  size_t off_B, off_Bt, off_B1, off_C, off_C1, off_part, off_G, off_Rf, off_Linv, off_cholw, off_Rho, off_Rhat,
+  size_t off_B, off_B0, off_Bt, off_B1, off_C, off_C1, off_part, off_G, off_Rf, off_Linv, off_cholw, off_Rho, off_Rhat,
       off_T, off_Q1, off_R1, off_R2, off_Rbar, off_perm, off_info, off_qr, off_gaps;
   size_t total;
 };
@@ -66,6 +70,7 @@ Layout plan(long long m_local, long long n, int k, int p) {
     return o;
   };
   L.off_B = take(lxn * 8);
+  L.off_B0 = take(lxn * 8);
   L.off_Bt = take(lxn * 8);
   L.off_B1 = take(lxn * 8);
   L.off_C = take(static_cast<size_t>(L.lp) * L.ldc * 8);
@@ -109,7 +114,7 @@ struct rs_lowrank_s {
   void* ar_ctx = nullptr;
   Layout L;
   char* ws;
-  double *B, *Bt, *B1, *C, *C1, *part, *G, *Rf, *Linv, *cholw, *Rho, *Rhat, *T, *Q1, *R1, *R2, *Rbar, *gaps;
+  double *B, *B0, *Bt, *B1, *C, *C1, *part, *G, *Rf, *Linv, *cholw, *Rho, *Rhat, *T, *Q1, *R1, *R2, *Rbar, *gaps;
   int64_t* perm;
   int* info;
   void* qr;
@@ -121,6 +126,19 @@ struct rs_lowrank_s {
   std::vector<Pending> pending;
   std::vector<cudaEvent_t> event_pool;
   std::vector<double> gaps_host;
+  bool gaps_valid = false;
+  // power_iterate enqueues only: its Cholesky factorisations report a breakdown with the
+  // internal code RS_INFO_POWER + pass, and pivot replays the iteration from the stored sample
+  int chol_code = RS_ERR_NOT_SPD;
+  const double* pow_A = nullptr;
+  long long pow_lda = 0;
+  int pow_q = 0;
+  // rs_lowrank_run: the whole step captured once as a CUDA graph and replayed
+  bool capturing = false;
+  bool graph_disabled = false;
+  cudaGraphExec_t gexec = nullptr;
+  std::vector<long long> gkey;
+  std::vector<Pending> gscopes;  // profiling scopes baked into the graph (external event records)
 };
 
 namespace {
@@ -155,8 +173,11 @@ cudaEvent_t get_event(rs_lowrank_t h) {
     h->event_pool.pop_back();
     return e;
   }
-  cudaEvent_t e;
-  cudaEventCreate(&e);
+  cudaEvent_t e = nullptr;
+  if (cudaEventCreate(&e) != cudaSuccess) {
+    cudaGetLastError();
+    return nullptr;  // profiling of this scope is skipped (Scope checks)
+  }
   return e;
 }
 
@@ -169,14 +190,26 @@ struct Scope {
   Scope(rs_lowrank_t hh, const char* nm, double fl) : h(hh), name(nm), flops(fl) {
     if (h->prof) {
       e0 = get_event(h);
-      cudaEventRecord(e0, h->st);
+      if (e0) record(e0);
     }
   }
+  // inside a graph capture the events become external event-record nodes, re-recorded at every
+  // replay and read back after each rs_lowrank_run (drain_graph_scopes)
+  void record(cudaEvent_t e) {
+    if (h->capturing)
+      cudaEventRecordWithFlags(e, h->st, cudaEventRecordExternal);
+    else
+      cudaEventRecord(e, h->st);
+  }
   ~Scope() {
-    if (h->prof) {
+    if (h->prof && e0) {
       cudaEvent_t e1 = get_event(h);
-      cudaEventRecord(e1, h->st);
-      h->pending.push_back(Pending{name, e0, e1, flops});
+      if (!e1) {
+        h->event_pool.push_back(e0);
+        return;
+      }
+      record(e1);
+      (h->capturing ? h->gscopes : h->pending).push_back(Pending{name, e0, e1, flops});
     }
   }
 };
@@ -196,13 +229,28 @@ void drain_profile(rs_lowrank_t h) {
   h->pending.clear();
 }
 
+void drain_graph_scopes(rs_lowrank_t h) {
+  for (auto& p : h->gscopes) {
+    float ms = 0.f;
+    if (cudaEventElapsedTime(&ms, p.e0, p.e1) != cudaSuccess) {
+      cudaGetLastError();
+      continue;
+    }
+    auto& e = h->profile[p.name];
+    e.ms += ms;
+    e.launches += 1;
+    e.flops += p.flops;
+  }
+}
+
 rs_status_t allreduce(rs_lowrank_t h, double* buf, long long count) {
   if (h->ar_fn && h->nranks > 1 && count > 0) {
     Scope sc(h, "comm", 0.0);
     if (h->ar_fn(h->ar_ctx, buf, count, h->st) != 0) return fail(h, RS_ERR_NCCL, "allreduce hook failed");
     return RS_OK;
   }
-  if (!h->comm || h->nranks <= 1 || count <= 0) return RS_OK;
+  // NCCL whenever a communicator is attached -- also at world size 1, so that code path runs
+  if (!h->comm || count <= 0) return RS_OK;
   Scope sc(h, "comm", 0.0);
   RS_NCCL(h, ncclAllReduce(buf, buf, static_cast<size_t>(count), ncclDouble, ncclSum, h->comm, h->st));
   return RS_OK;
@@ -262,7 +310,7 @@ rs_status_t cholqr_small_pass(rs_lowrank_t h, const double* src, int rr, int rp,
     Scope sc(h, "chol", rr * static_cast<double>(rr) * rr / 3.0);
     if (shift)
       RS_CUDA(h, shift_diag(h->st, h->G, rp, rr, 11.0 * (static_cast<double>(h->n) * rr + rr * (rr + 1.0)) * 0x1p-53));
-    RS_CUDA(h, chol_inv(h->st, h->G, rp, rr, rp, h->Rf, rp, h->Linv, rp, h->cholw, h->info, RS_ERR_NOT_SPD));
+    RS_CUDA(h, chol_inv(h->st, h->G, rp, rr, rp, h->Rf, rp, h->Linv, rp, h->cholw, h->info, h->chol_code));
   }
   {
     Scope sc(h, "apply", 2.0 * rr * rr * static_cast<double>(h->n));
@@ -304,7 +352,7 @@ rs_status_t cholqr_dist(rs_lowrank_t h, double* Cn, int rr, int rp, int npass, i
       if (pass < nshift)
         RS_CUDA(h, shift_diag(h->st, h->G, rp, rr,
                               11.0 * (static_cast<double>(h->m_global) * rr + rr * (rr + 1.0)) * 0x1p-53));
-      RS_CUDA(h, chol_inv(h->st, h->G, rp, rr, rp, h->Rf, rp, h->Linv, rp, h->cholw, h->info, RS_ERR_NOT_SPD));
+      RS_CUDA(h, chol_inv(h->st, h->G, rp, rr, rp, h->Rf, rp, h->Linv, rp, h->cholw, h->info, h->chol_code));
     }
     if (ml > 0) {
       Scope sc(h, "apply", 2.0 * rr * static_cast<double>(rr) * ml);
@@ -328,10 +376,19 @@ rs_status_t check_matrix(rs_lowrank_t h, const void* p, long long ld, long long 
   return RS_OK;
 }
 
+// internal status: a power-iteration CholQR breakdown was flagged (info[0] >= RS_INFO_POWER)
+constexpr rs_status_t RS_INFO_REPLAY = static_cast<rs_status_t>(1000);
+
 rs_status_t sync_and_check(rs_lowrank_t h) {
   RS_CUDA(h, cudaStreamSynchronize(h->st));
+  if (h->comm) {  // a failed peer or network error surfaces here rather than as a hang later
+    ncclResult_t ar = ncclSuccess;
+    RS_NCCL(h, ncclCommGetAsyncError(h->comm, &ar));
+    if (ar != ncclSuccess) return fail(h, RS_ERR_NCCL, "NCCL asynchronous error: %s", ncclGetErrorString(ar));
+  }
   int info[2] = {0, 0};
   RS_CUDA(h, cudaMemcpy(info, h->info, sizeof(info), cudaMemcpyDeviceToHost));
+  if (info[0] >= RS_INFO_POWER) return RS_INFO_REPLAY;
   if (info[0] == RS_ERR_NOT_SPD)
     return fail(h, RS_ERR_NOT_SPD, "CholQR breakdown: Gram matrix not positive definite at column %d", info[1]);
   if (info[0] == RS_ERR_RANK_DEFICIENT)
@@ -339,6 +396,332 @@ rs_status_t sync_and_check(rs_lowrank_t h) {
   return RS_OK;
 }
 
+// ---------------------------------------------------------------------------------------------
+// The four steps of Fig. 2, enqueue-only (no host synchronisation), shared by the phase calls
+// and by the graph-captured rs_lowrank_run.
+// ---------------------------------------------------------------------------------------------
+
+// Step 1: B := Omega A summed over ranks (Fig. 2(b) lines 2-3)
+rs_status_t enqueue_sample(rs_lowrank_t h, const double* A, long long lda) {
+  const Layout& L = h->L;
+  RS_CUDA(h, cudaMemsetAsync(h->info, 0, 16, h->st));
+  const long long lxn = static_cast<long long>(L.lp) * h->n;
+  if (h->m_local > 0) {
+    const int splits = gemm_choose_splits(L.lp, static_cast<int>(h->n), h->m_local, max_splits_for(h, lxn), h->sms);
+    const int ns = gemm_nsplit(h->m_local, splits);
+    {
+      Scope sc(h, "gemm_sample", 2.0 * h->ell * static_cast<double>(h->m_local) * h->n);
+      View2D Av{A, h->m_local, h->n, lda};
+      GemmOutDesc out{h->part, 1, L.lp, lxn, L.lp, static_cast<int>(h->n)};
+      PhiloxDesc phx{true, h->seed, 0u, h->row_offset, h->ell};
+      RS_CUDA(h, gemm_kc(h->st, L.lp, static_cast<int>(h->n), h->m_local, Av, Av, phx, out, splits));
+    }
+    {
+      Scope sc(h, "reduce", 0.0);
+      RS_CUDA(h, splitk_reduce(h->st, h->B, h->part, ns, lxn, lxn));
+    }
+  } else {
+    RS_CUDA(h, cudaMemsetAsync(h->B, 0, lxn * 8, h->st));
+  }
+  return allreduce(h, h->B, lxn);
+}
+
+// line 12: dst := Csrc A summed over ranks
+rs_status_t gemm_b(rs_lowrank_t h, const double* A, long long lda, const double* Csrc, double* dst) {
+  const Layout& L = h->L;
+  const long long ml = h->m_local, n = h->n;
+  const long long lxn = static_cast<long long>(L.lp) * n;
+  if (ml > 0) {
+    const int splits = gemm_choose_splits(L.lp, static_cast<int>(n), ml, max_splits_for(h, lxn), h->sms);
+    const int ns = gemm_nsplit(ml, splits);
+    {
+      Scope sc(h, "gemm_power_b", 2.0 * h->ell * static_cast<double>(ml) * n);
+      View2D Cv{Csrc, ml, L.lp, L.ldc};
+      View2D Av{A, ml, n, lda};
+      GemmOutDesc out{h->part, 1, L.lp, lxn, L.lp, static_cast<int>(n)};
+      PhiloxDesc nophx{false, 0, 0, 0, 0};
+      RS_CUDA(h, gemm_kc(h->st, L.lp, static_cast<int>(n), ml, Cv, Av, nophx, out, splits));
+    }
+    Scope sc(h, "reduce", 0.0);
+    RS_CUDA(h, splitk_reduce(h->st, dst, h->part, ns, lxn, lxn));
+  } else {
+    RS_CUDA(h, cudaMemsetAsync(dst, 0, lxn * 8, h->st));
+  }
+  return allreduce(h, dst, lxn);
+}
+
+// line 7: C := Bt A^T   (C row-major lp x ldc: C[i, j] at i*ldc + j)
+rs_status_t gemm_c(rs_lowrank_t h, const double* A, long long lda) {
+  const Layout& L = h->L;
+  const long long ml = h->m_local, n = h->n;
+  if (ml > 0) {
+    Scope sc(h, "gemm_power_c", 2.0 * h->ell * static_cast<double>(ml) * n);
+    View2D Bv{h->Bt, L.lp, n, L.lp};
+    View2D Av{A, ml, n, lda};
+    GemmOutDesc out{h->C, L.ldc, 1, 0, L.lp, static_cast<int>(ml)};
+    RS_CUDA(h, gemm_mc(h->st, L.lp, static_cast<int>(ml), n, Bv, Av, out, 1));
+  }
+  return RS_OK;
+}
+
+// One plain pass of Fig. 2(a) lines 5-12 up to B1 = C1 A (allreduced): B := QR(B) (replicated
+// CholQR2), C := B A^T, C := QR(C) (distributed CholQR2 whose second R^{-T} is applied to the
+// l x n product instead of C -- exact re-association, R2 = I + O(kappa^2 u)).  The caller finishes
+// with B := R2^{-T} B1 (power_apply).  Cholesky breakdowns are flagged with h->chol_code.
+rs_status_t power_to_b1(rs_lowrank_t h, const double* A, long long lda) {
+  const Layout& L = h->L;
+  const long long ml = h->m_local;
+  rs_status_t s = cholqr2_rows_small(h, h->B, h->Bt);  // line 5
+  if (s != RS_OK) return s;
+  if ((s = gemm_c(h, A, lda)) != RS_OK) return s;     // line 7
+  // line 10
+  if ((s = gram_rows_kc(h, h->C, L.ldc, ml, L.lp, L.lp)) != RS_OK) return s;
+  if ((s = allreduce(h, h->G, static_cast<long long>(L.lp) * L.lp)) != RS_OK) return s;
+  {
+    Scope sc(h, "chol", L.ell * static_cast<double>(L.ell) * L.ell / 3.0);
+    RS_CUDA(h, chol_inv(h->st, h->G, L.lp, L.ell, L.lp, h->Rf, L.lp, h->Linv, L.lp, h->cholw, h->info, h->chol_code));
+  }
+  if (ml > 0) {
+    Scope sc(h, "apply", 2.0 * L.ell * static_cast<double>(L.ell) * ml);
+    View2D Lv{h->Linv, L.lp, L.lp, L.lp};
+    View2D Cv{h->C, ml, L.lp, L.ldc};
+    GemmOutDesc out{h->C1, L.ldc, 1, 0, L.lp, static_cast<int>(ml)};
+    RS_CUDA(h, gemm_mc(h->st, L.lp, static_cast<int>(ml), L.lp, Lv, Cv, out, 1, 1));  // Linv lower
+  }
+  if ((s = gram_rows_kc(h, h->C1, L.ldc, ml, L.lp, L.lp)) != RS_OK) return s;
+  if ((s = allreduce(h, h->G, static_cast<long long>(L.lp) * L.lp)) != RS_OK) return s;
+  {
+    Scope sc(h, "chol", L.ell * static_cast<double>(L.ell) * L.ell / 3.0);
+    RS_CUDA(h, chol_inv(h->st, h->G, L.lp, L.ell, L.lp, h->Rf, L.lp, h->Linv, L.lp, h->cholw, h->info, h->chol_code));
+  }
+  return gemm_b(h, A, lda, h->C1, h->B1);  // line 12 (B1 = C1 A)
+}
+
+rs_status_t power_apply(rs_lowrank_t h) {
+  const Layout& L = h->L;
+  Scope sc(h, "apply", 2.0 * L.ell * static_cast<double>(L.ell) * h->n);
+  RS_CUDA(h, small_gemm(h->st, L.lp, static_cast<int>(h->n), L.lp, h->Linv, 1, L.lp, h->B1, 1, L.lp, h->B, 1, L.lp,
+                        false));
+  return RS_OK;
+}
+
+// The R20 fallback of one pass, from its input B: 2 shifted + 2 plain CholQR passes on B and on C.
+rs_status_t power_robust(rs_lowrank_t h, const double* A, long long lda) {
+  const Layout& L = h->L;
+  rs_status_t s;
+  const double* src = h->B;
+  for (int pass = 0; pass < 4; ++pass) {  // B -> B1 -> Bt -> B1 -> Bt
+    double* dst = pass % 2 == 0 ? h->B1 : h->Bt;
+    if ((s = cholqr_small_pass(h, src, L.ell, L.lp, dst, pass < 2)) != RS_OK) return s;
+    src = dst;
+  }
+  if ((s = gemm_c(h, A, lda)) != RS_OK) return s;
+  if ((s = cholqr_dist(h, h->C, L.ell, L.lp, 4, 2)) != RS_OK) return s;
+  return gemm_b(h, A, lda, h->C, h->B);
+}
+
+// q passes, enqueue only.  The sample is kept in B0; a breakdown in pass it sets info to
+// RS_INFO_POWER + it, which pivot (or rs_lowrank_run) turns into replay_power_and_pivot.
+rs_status_t enqueue_power(rs_lowrank_t h, const double* A, long long lda, int q) {
+  const Layout& L = h->L;
+  RS_CUDA(h, cudaMemcpyAsync(h->B0, h->B, static_cast<size_t>(L.lp) * h->n * 8, cudaMemcpyDeviceToDevice, h->st));
+  h->pow_A = A;
+  h->pow_lda = lda;
+  h->pow_q = q;
+  rs_status_t s = RS_OK;
+  for (int it = 0; it < q && s == RS_OK; ++it) {
+    h->chol_code = RS_INFO_POWER + it;
+    s = power_to_b1(h, A, lda);
+    if (s == RS_OK) s = power_apply(h);
+  }
+  h->chol_code = RS_ERR_NOT_SPD;
+  if (s == RS_OK) h->powers = q;
+  return s;
+}
+
+// The breakdown path: q passes from the stored sample with a host check after each pass; a pass
+// whose CholQR broke down is redone from its input B with shifted CholQR (R20).
+rs_status_t power_sync(rs_lowrank_t h, const double* A, long long lda, int q) {
+  rs_status_t s;
+  h->chol_code = RS_ERR_NOT_SPD;
+  for (int it = 0; it < q; ++it) {
+    if ((s = power_to_b1(h, A, lda)) != RS_OK) return s;
+    int info[2] = {0, 0};
+    RS_CUDA(h, cudaMemcpyAsync(info, h->info, sizeof(info), cudaMemcpyDeviceToHost, h->st));
+    RS_CUDA(h, cudaStreamSynchronize(h->st));
+    if (info[0] == RS_ERR_NOT_SPD) {
+      RS_CUDA(h, cudaMemsetAsync(h->info, 0, 16, h->st));
+      if ((s = power_robust(h, A, lda)) != RS_OK) return s;
+      h->robust_iters++;
+    } else if ((s = power_apply(h)) != RS_OK) {
+      return s;
+    }
+  }
+  h->powers = q;
+  return RS_OK;
+}
+
+// Step 2: truncated QRCP of B (Fig. 2(b) line 6) and T = R^_11^{-1} R^_12 (line 9)
+rs_status_t enqueue_pivot(rs_lowrank_t h, int64_t* perm) {
+  const Layout& L = h->L;
+  {
+    Scope sc(h, "qrcp", 0.0);
+    RS_CUDA(h, qrcp_truncated(h->st, h->B, L.lp, h->ell, h->n, h->k, h->qr, h->perm, h->Rho, L.kp, h->gaps, h->info,
+                              h->sms));
+  }
+  {
+    Scope sc(h, "other", static_cast<double>(h->k) * h->k * (h->n - h->k));
+    RS_CUDA(h, permute_cols(h->st, h->Rho, L.kp, h->k, h->n, h->perm, h->Rhat, L.kp));
+    RS_CUDA(h, trsm_upper_cols(h->st, h->Rhat, L.kp, h->k, h->Rhat + static_cast<long long>(h->k) * L.kp, L.kp,
+                               h->n - h->k, h->T, L.kp));
+  }
+  if (perm) RS_CUDA(h, cudaMemcpyAsync(perm, h->perm, h->n * 8, cudaMemcpyDeviceToDevice, h->st));
+  return RS_OK;
+}
+
+rs_status_t replay_power_and_pivot(rs_lowrank_t h, int64_t* perm) {
+  const Layout& L = h->L;
+  RS_CUDA(h, cudaMemsetAsync(h->info, 0, 16, h->st));
+  RS_CUDA(h, cudaMemcpyAsync(h->B, h->B0, static_cast<size_t>(L.lp) * h->n * 8, cudaMemcpyDeviceToDevice, h->st));
+  h->robust_iters = 0;
+  rs_status_t s = power_sync(h, h->pow_A, h->pow_lda, h->pow_q);
+  if (s != RS_OK) return s;
+  if ((s = enqueue_pivot(h, perm)) != RS_OK) return s;
+  s = sync_and_check(h);
+  return s == RS_INFO_REPLAY ? fail(h, RS_ERR_NOT_SPD, "CholQR breakdown in the power iteration") : s;
+}
+
+rs_status_t check_factor_args(rs_lowrank_t h, const double* A, long long lda, const double* Q, long long ldq,
+                              const double* R, long long ldr) {
+  rs_status_t s;
+  if (h->m_local > 0) {
+    if ((s = check_matrix(h, A, lda, h->m_local, "A")) != RS_OK) return s;
+    if ((s = check_matrix(h, Q, ldq, h->m_local, "Q")) != RS_OK) return s;
+  }
+  return check_matrix(h, R, ldr, h->k, "R");
+}
+
+// Step 3: [Q, Rbar] := QR(A P_{1:k}) by CholQR with npass passes (even, so the last lands in Q),
+// the first nshift with the Gram shifted by 11 (m k + k(k+1)) u ||X||_F^2 (R20); R := Rbar [I_k T]
+// (Fig. 2(b) lines 8 and 10).
+rs_status_t enqueue_factor(rs_lowrank_t h, const double* A, long long lda, double* Q, long long ldq, double* R,
+                           long long ldr, int npass, int nshift) {
+  const Layout& L = h->L;
+  const long long ml = h->m_local, n = h->n;
+  const int k = h->k;
+  // Q := A(:, P_{1:k})
+  if (ml > 0) {
+    Scope sc(h, "factor", 0.0);
+    RS_CUDA(h, gather_cols(h->st, A, lda, ml, h->perm, k, Q, ldq));
+  }
+  const double* src = Q;
+  long long ld_src = ldq;
+  double* bufs[2] = {h->Rbar, h->R2};
+  int which = -1;  // index of the running product Rbar = R_p ... R_1 (-1: identity)
+  for (int pass = 0; pass < npass; ++pass) {
+    double* dst = pass % 2 == 0 ? h->Q1 : Q;
+    const long long ld_dst = pass % 2 == 0 ? L.ldq1 : ldq;
+    // Gram G = X^T X (k x k) of the tall X = src (m_local x k column-major)
+    rs_status_t st2 = gram_rows_kc(h, src, ld_src, ml, k, L.kp);
+    if (st2 != RS_OK) return st2;
+    st2 = allreduce(h, h->G, static_cast<long long>(L.kp) * L.kp);
+    if (st2 != RS_OK) return st2;
+    {
+      Scope sc(h, "chol", k * static_cast<double>(k) * k / 3.0);
+      if (pass < nshift)
+        RS_CUDA(h, shift_diag(h->st, h->G, L.kp, k,
+                              11.0 * (static_cast<double>(h->m_global) * k + k * (k + 1.0)) * 0x1p-53));
+      RS_CUDA(h, chol_inv(h->st, h->G, L.kp, k, L.kp, h->R1, L.kp, h->Linv, L.kp, h->cholw, h->info,
+                          RS_ERR_NOT_SPD));
+    }
+    // dst = src * R_p^{-1}  (R_p^{-1}[kk, c] = Linv[c + kk*kp]: N-contiguous operand)
+    if (ml > 0) {
+      Scope sc(h, "factor", 2.0 * k * static_cast<double>(k) * ml);
+      View2D Xv{src, ml, k, ld_src};
+      View2D Wv{h->Linv, k, k, L.kp};
+      GemmOutDesc out{dst, 1, ld_dst, 0, static_cast<int>(ml), k};
+      RS_CUDA(h, gemm_mc(h->st, static_cast<int>(ml), k, k, Xv, Wv, out, 1, 2));  // R^-1 upper
+    }
+    {
+      Scope sc(h, "other", 2.0 * k * static_cast<double>(k) * k);
+      if (which < 0) {
+        which = 0;
+        RS_CUDA(h, copy_2d(h->st, h->R1, L.kp, bufs[0], L.kp, L.kp, L.kp));
+      } else {  // Rbar := R_p Rbar
+        RS_CUDA(h, small_gemm(h->st, k, k, k, h->R1, 1, L.kp, bufs[which], 1, L.kp, bufs[1 - which], 1, L.kp,
+                              false));
+        which = 1 - which;
+      }
+    }
+    src = dst;
+    ld_src = ld_dst;
+  }
+  Scope sc(h, "other", 2.0 * k * static_cast<double>(k) * n);
+  // R = Rbar [I_k T]
+  RS_CUDA(h, copy_2d(h->st, bufs[which], L.kp, R, ldr, k, k));
+  if (n > k)
+    RS_CUDA(h, small_gemm(h->st, k, static_cast<int>(n - k), k, bufs[which], 1, L.kp, h->T, 1, L.kp,
+                          R + static_cast<long long>(k) * ldr, 1, ldr, false));
+  return RS_OK;
+}
+
+// CholQR2 broke down (kappa(A P_1)^2 u > 1, e.g. an adaptive l past the numerical rank): shifted
+// CholQR with 2, then 4 shifted passes ahead of the two plain ones (R20)
+rs_status_t factor_fallback(rs_lowrank_t h, const double* A, long long lda, double* Q, long long ldq, double* R,
+                            long long ldr) {
+  rs_status_t s = RS_ERR_NOT_SPD;
+  for (int nshift = 2; s == RS_ERR_NOT_SPD && nshift <= 4; nshift += 2) {
+    RS_CUDA(h, cudaMemsetAsync(h->info, 0, 16, h->st));
+    s = enqueue_factor(h, A, lda, Q, ldq, R, ldr, nshift + 2, nshift);
+    if (s == RS_OK) s = sync_and_check(h);
+    h->factor_shifts = nshift;
+  }
+  return s;
+}
+
+void release_graph(rs_lowrank_t h) {
+  if (h->gexec) cudaGraphExecDestroy(h->gexec);
+  h->gexec = nullptr;
+  h->gkey.clear();
+  for (auto& p : h->gscopes) {
+    h->event_pool.push_back(p.e0);
+    h->event_pool.push_back(p.e1);
+  }
+  h->gscopes.clear();
+}
+
+// Capture sample -> power (q) -> pivot -> factor (CholQR2) on the handle's stream as one CUDA
+// graph: replays launch the ~70 kernels and NCCL collectives of a step with one call
+// and no host round trip.  Anything the capture cannot hold disables the graph for this handle
+// (the phases then run directly).
+rs_status_t capture_step(rs_lowrank_t h, const double* A, long long lda, int q, int64_t* perm, double* Q,
+                         long long ldq, double* R, long long ldr) {
+  release_graph(h);
+  cudaGraph_t g = nullptr;
+  if (cudaStreamBeginCapture(h->st, cudaStreamCaptureModeThreadLocal) != cudaSuccess) {
+    cudaGetLastError();
+    h->graph_disabled = true;
+    return RS_OK;
+  }
+  h->capturing = true;
+  rs_status_t s = enqueue_sample(h, A, lda);
+  if (s == RS_OK && q > 0) s = enqueue_power(h, A, lda, q);
+  if (s == RS_OK) s = enqueue_pivot(h, perm);
+  if (s == RS_OK) s = enqueue_factor(h, A, lda, Q, ldq, R, ldr, 2, 0);
+  h->capturing = false;
+  const cudaError_t ec = cudaStreamEndCapture(h->st, &g);
+  cudaError_t ei = cudaErrorUnknown;
+  if (s == RS_OK && ec == cudaSuccess && g) ei = cudaGraphInstantiate(&h->gexec, g, 0);
+  if (g) cudaGraphDestroy(g);
+  if (ei != cudaSuccess) {
+    cudaGetLastError();
+    h->gexec = nullptr;
+    h->graph_disabled = true;
+    release_graph(h);
+    h->err.clear();
+  }
+  return RS_OK;
+}
 }  // namespace
 
 extern "C" {
@@ -391,6 +774,7 @@ rs_status_t rs_lowrank_create(rs_lowrank_t* out, int64_t m_global, int64_t m_loc
   h->ws = base;
   auto D = [&](size_t off) { return reinterpret_cast<double*>(base + off); };
   h->B = D(L.off_B);
+  h->B0 = D(L.off_B0);
   h->Bt = D(L.off_Bt);
   h->B1 = D(L.off_B1);
   h->C = D(L.off_C);
@@ -424,36 +808,17 @@ rs_status_t rs_lowrank_create(rs_lowrank_t* out, int64_t m_global, int64_t m_loc
 
 rs_status_t rs_lowrank_sample(rs_lowrank_t h, const double* A, int64_t lda) {
   if (!h) return RS_ERR_INVALID_ARG;
-  const Layout& L = h->L;
   if (h->m_local > 0) {
     rs_status_t s = check_matrix(h, A, lda, h->m_local, "A");
     if (s != RS_OK) return s;
   }
-  RS_CUDA(h, cudaMemsetAsync(h->info, 0, 16, h->st));
-  const long long lxn = static_cast<long long>(L.lp) * h->n;
-  if (h->m_local > 0) {
-    const int splits = gemm_choose_splits(L.lp, static_cast<int>(h->n), h->m_local, max_splits_for(h, lxn), h->sms);
-    const int ns = gemm_nsplit(h->m_local, splits);
-    {
-      Scope sc(h, "gemm_sample", 2.0 * h->ell * static_cast<double>(h->m_local) * h->n);
-      View2D Av{A, h->m_local, h->n, lda};
-      GemmOutDesc out{h->part, 1, L.lp, lxn, L.lp, static_cast<int>(h->n)};
-      PhiloxDesc phx{true, h->seed, 0u, h->row_offset, h->ell};
-      RS_CUDA(h, gemm_kc(h->st, L.lp, static_cast<int>(h->n), h->m_local, Av, Av, phx, out, splits));
-    }
-    {
-      Scope sc(h, "reduce", 0.0);
-      RS_CUDA(h, splitk_reduce(h->st, h->B, h->part, ns, lxn, lxn));
-    }
-  } else {
-    RS_CUDA(h, cudaMemsetAsync(h->B, 0, lxn * 8, h->st));
-  }
-  rs_status_t s = allreduce(h, h->B, lxn);
+  rs_status_t s = enqueue_sample(h, A, lda);
   if (s != RS_OK) return s;
   h->state = ST_SAMPLED;
   h->powers = 0;
   h->robust_iters = 0;
-  h->ell = L.ell;
+  h->pow_q = 0;
+  h->ell = h->L.ell;
   h->k = h->k0;
   h->adaptive = false;
   return RS_OK;
@@ -463,124 +828,25 @@ rs_status_t rs_lowrank_power_iterate(rs_lowrank_t h, const double* A, int64_t ld
   if (!h) return RS_ERR_INVALID_ARG;
   if (h->state != ST_SAMPLED) return fail(h, RS_ERR_BAD_STATE, "power_iterate needs a fresh sample");
   if (h->adaptive) return fail(h, RS_ERR_BAD_STATE, "the adaptive sample already includes its power iterations");
+  if (h->pow_q > 0) return fail(h, RS_ERR_BAD_STATE, "power_iterate already ran on this sample");
   if (q < 0) return fail(h, RS_ERR_INVALID_ARG, "q < 0");
   if (q == 0) return RS_OK;
-  const Layout& L = h->L;
   if (h->m_local > 0) {
     rs_status_t s = check_matrix(h, A, lda, h->m_local, "A");
     if (s != RS_OK) return s;
   }
-  const long long ml = h->m_local, n = h->n;
-  const long long lxn = static_cast<long long>(L.lp) * n;
-  // line 12: dst := Csrc A summed over ranks
-  auto gemm_b = [&](const double* Csrc, double* dst) -> rs_status_t {
-    if (ml > 0) {
-      const int splits = gemm_choose_splits(L.lp, static_cast<int>(n), ml, max_splits_for(h, lxn), h->sms);
-      const int ns = gemm_nsplit(ml, splits);
-      {
-        Scope sc(h, "gemm_power_b", 2.0 * h->ell * static_cast<double>(ml) * n);
-        View2D Cv{Csrc, ml, L.lp, L.ldc};
-        View2D Av{A, ml, n, lda};
-        GemmOutDesc out{h->part, 1, L.lp, lxn, L.lp, static_cast<int>(n)};
-        PhiloxDesc nophx{false, 0, 0, 0, 0};
-        RS_CUDA(h, gemm_kc(h->st, L.lp, static_cast<int>(n), ml, Cv, Av, nophx, out, splits));
-      }
-      Scope sc(h, "reduce", 0.0);
-      RS_CUDA(h, splitk_reduce(h->st, dst, h->part, ns, lxn, lxn));
-    } else {
-      RS_CUDA(h, cudaMemsetAsync(dst, 0, lxn * 8, h->st));
-    }
-    return allreduce(h, dst, lxn);
-  };
-  // line 7: C := Bt A^T   (C row-major lp x ldc: C[i, j] at i*ldc + j)
-  auto gemm_c = [&]() -> rs_status_t {
-    if (ml > 0) {
-      Scope sc(h, "gemm_power_c", 2.0 * h->ell * static_cast<double>(ml) * n);
-      View2D Bv{h->Bt, L.lp, n, L.lp};
-      View2D Av{A, ml, n, lda};
-      GemmOutDesc out{h->C, L.ldc, 1, 0, L.lp, static_cast<int>(ml)};
-      RS_CUDA(h, gemm_mc(h->st, L.lp, static_cast<int>(ml), n, Bv, Av, out, 1));
-    }
-    return RS_OK;
-  };
-  for (int it = 0; it < q; ++it) {
-    // line 5: B := QR(B)  (replicated CholQR2)
-    rs_status_t s = cholqr2_rows_small(h, h->B, h->Bt);
-    if (s != RS_OK) return s;
-    if ((s = gemm_c()) != RS_OK) return s;
-    // line 10: C := QR(C)  (distributed CholQR2; the second R^{-T} is applied to B below)
-    s = gram_rows_kc(h, h->C, L.ldc, ml, L.lp, L.lp);
-    if (s != RS_OK) return s;
-    s = allreduce(h, h->G, static_cast<long long>(L.lp) * L.lp);
-    if (s != RS_OK) return s;
-    {
-      Scope sc(h, "chol", L.ell * static_cast<double>(L.ell) * L.ell / 3.0);
-      RS_CUDA(h, chol_inv(h->st, h->G, L.lp, L.ell, L.lp, h->Rf, L.lp, h->Linv, L.lp, h->cholw, h->info, RS_ERR_NOT_SPD));
-    }
-    if (ml > 0) {
-      Scope sc(h, "apply", 2.0 * L.ell * static_cast<double>(L.ell) * ml);
-      View2D Lv{h->Linv, L.lp, L.lp, L.lp};
-      View2D Cv{h->C, ml, L.lp, L.ldc};
-      GemmOutDesc out{h->C1, L.ldc, 1, 0, L.lp, static_cast<int>(ml)};
-      RS_CUDA(h, gemm_mc(h->st, L.lp, static_cast<int>(ml), L.lp, Lv, Cv, out, 1, 1));  // Linv lower
-    }
-    s = gram_rows_kc(h, h->C1, L.ldc, ml, L.lp, L.lp);
-    if (s != RS_OK) return s;
-    s = allreduce(h, h->G, static_cast<long long>(L.lp) * L.lp);
-    if (s != RS_OK) return s;
-    {
-      Scope sc(h, "chol", L.ell * static_cast<double>(L.ell) * L.ell / 3.0);
-      RS_CUDA(h, chol_inv(h->st, h->G, L.lp, L.ell, L.lp, h->Rf, L.lp, h->Linv, L.lp, h->cholw, h->info, RS_ERR_NOT_SPD));
-    }
-    // line 12: B := C A   (B1 = C1 A summed over ranks; then B = R2^{-T} B1, exact re-association)
-    if ((s = gemm_b(h->C1, h->B1)) != RS_OK) return s;
-    // B is still this iteration's input: on a CholQR breakdown (kappa^2 u > 1) redo the
-    // iteration with shifted CholQR (2 shifted + 2 plain passes on B and on C, R20).  The Gram
-    // matrices are replicated, so every rank takes the same branch.
-    int info[2] = {0, 0};
-    RS_CUDA(h, cudaMemcpyAsync(info, h->info, sizeof(info), cudaMemcpyDeviceToHost, h->st));
-    RS_CUDA(h, cudaStreamSynchronize(h->st));
-    if (info[0] == RS_ERR_NOT_SPD) {
-      RS_CUDA(h, cudaMemsetAsync(h->info, 0, 16, h->st));
-      const double* src = h->B;
-      for (int pass = 0; pass < 4; ++pass) {  // B -> B1 -> Bt -> B1 -> Bt
-        double* dst = pass % 2 == 0 ? h->B1 : h->Bt;
-        if ((s = cholqr_small_pass(h, src, L.ell, L.lp, dst, pass < 2)) != RS_OK) return s;
-        src = dst;
-      }
-      if ((s = gemm_c()) != RS_OK) return s;
-      if ((s = cholqr_dist(h, h->C, L.ell, L.lp, 4, 2)) != RS_OK) return s;
-      if ((s = gemm_b(h->C, h->B)) != RS_OK) return s;
-      h->robust_iters++;
-    } else {
-      Scope sc(h, "apply", 2.0 * L.ell * static_cast<double>(L.ell) * n);
-      RS_CUDA(h, small_gemm(h->st, L.lp, static_cast<int>(n), L.lp, h->Linv, 1, L.lp, h->B1, 1, L.lp, h->B, 1, L.lp, false));
-    }
-    h->powers++;
-  }
-  return RS_OK;
+  return enqueue_power(h, A, lda, q);
 }
 
 rs_status_t rs_lowrank_pivot(rs_lowrank_t h, int64_t* perm) {
   if (!h) return RS_ERR_INVALID_ARG;
   if (h->state != ST_SAMPLED) return fail(h, RS_ERR_BAD_STATE, "pivot needs a sample");
-  const Layout& L = h->L;
-  {
-    Scope sc(h, "qrcp", 0.0);
-    RS_CUDA(h, qrcp_truncated(h->st, h->B, L.lp, h->ell, h->n, h->k, h->qr, h->perm, h->Rho, L.kp, h->gaps, h->info,
-                              h->sms));
-  }
-  {
-    Scope sc(h, "other", static_cast<double>(h->k) * h->k * (h->n - h->k));
-    RS_CUDA(h, permute_cols(h->st, h->Rho, L.kp, h->k, h->n, h->perm, h->Rhat, L.kp));
-    RS_CUDA(h, trsm_upper_cols(h->st, h->Rhat, L.kp, h->k, h->Rhat + static_cast<long long>(h->k) * L.kp, L.kp,
-                               h->n - h->k, h->T, L.kp));
-  }
-  if (perm) RS_CUDA(h, cudaMemcpyAsync(perm, h->perm, h->n * 8, cudaMemcpyDeviceToDevice, h->st));
-  rs_status_t s = sync_and_check(h);
+  rs_status_t s = enqueue_pivot(h, perm);
   if (s != RS_OK) return s;
-  h->gaps_host.assign(h->k, 0.0);
-  RS_CUDA(h, cudaMemcpy(h->gaps_host.data(), h->gaps, h->k * 8, cudaMemcpyDeviceToHost));
+  s = sync_and_check(h);
+  if (s == RS_INFO_REPLAY) s = replay_power_and_pivot(h, perm);
+  if (s != RS_OK) return s;
+  h->gaps_valid = false;
   h->state = ST_PIVOTED;
   return RS_OK;
 }
@@ -589,88 +855,60 @@ rs_status_t rs_lowrank_factor(rs_lowrank_t h, const double* A, int64_t lda, doub
                               int64_t ldr) {
   if (!h) return RS_ERR_INVALID_ARG;
   if (h->state != ST_PIVOTED && h->state != ST_FACTORED) return fail(h, RS_ERR_BAD_STATE, "factor needs pivot");
-  const Layout& L = h->L;
-  const long long ml = h->m_local, n = h->n;
-  const int k = h->k;
-  rs_status_t s;
-  if (ml > 0) {
-    if ((s = check_matrix(h, A, lda, ml, "A")) != RS_OK) return s;
-    if ((s = check_matrix(h, Q, ldq, ml, "Q")) != RS_OK) return s;
-  }
-  if ((s = check_matrix(h, R, ldr, k, "R")) != RS_OK) return s;
-  // CholQR with npass passes (even, so the last pass lands in Q); the first nshift Grams get
-  // + 11 (m k + k(k+1)) u ||X||_F^2 I (shifted CholeskyQR: each shifted pass is breakdown-free and
-  // cuts kappa by ~ 1/sqrt(11 m k u), so the plain passes that follow see kappa^2 u < 1)
-  auto run = [&](int npass, int nshift) -> rs_status_t {
-    // Q := A(:, P_{1:k})
-    if (ml > 0) {
-      Scope sc(h, "factor", 0.0);
-      RS_CUDA(h, gather_cols(h->st, A, lda, ml, h->perm, k, Q, ldq));
-    }
-    const double* src = Q;
-    long long ld_src = ldq;
-    double* bufs[2] = {h->Rbar, h->R2};
-    int which = -1;  // index of the running product Rbar = R_p ... R_1 (-1: identity)
-    for (int pass = 0; pass < npass; ++pass) {
-      double* dst = pass % 2 == 0 ? h->Q1 : Q;
-      const long long ld_dst = pass % 2 == 0 ? L.ldq1 : ldq;
-      // Gram G = X^T X (k x k) of the tall X = src (m_local x k column-major)
-      rs_status_t st2 = gram_rows_kc(h, src, ld_src, ml, k, L.kp);
-      if (st2 != RS_OK) return st2;
-      st2 = allreduce(h, h->G, static_cast<long long>(L.kp) * L.kp);
-      if (st2 != RS_OK) return st2;
-      {
-        Scope sc(h, "chol", k * static_cast<double>(k) * k / 3.0);
-        if (pass < nshift)
-          RS_CUDA(h, shift_diag(h->st, h->G, L.kp, k,
-                                11.0 * (static_cast<double>(h->m_global) * k + k * (k + 1.0)) * 0x1p-53));
-        RS_CUDA(h, chol_inv(h->st, h->G, L.kp, k, L.kp, h->R1, L.kp, h->Linv, L.kp, h->cholw, h->info,
-                            RS_ERR_NOT_SPD));
-      }
-      // dst = src * R_p^{-1}  (R_p^{-1}[kk, c] = Linv[c + kk*kp]: N-contiguous operand)
-      if (ml > 0) {
-        Scope sc(h, "factor", 2.0 * k * static_cast<double>(k) * ml);
-        View2D Xv{src, ml, k, ld_src};
-        View2D Wv{h->Linv, k, k, L.kp};
-        GemmOutDesc out{dst, 1, ld_dst, 0, static_cast<int>(ml), k};
-        RS_CUDA(h, gemm_mc(h->st, static_cast<int>(ml), k, k, Xv, Wv, out, 1, 2));  // R^-1 upper
-      }
-      {
-        Scope sc(h, "other", 2.0 * k * static_cast<double>(k) * k);
-        if (which < 0) {
-          which = 0;
-          RS_CUDA(h, copy_2d(h->st, h->R1, L.kp, bufs[0], L.kp, L.kp, L.kp));
-        } else {  // Rbar := R_p Rbar
-          RS_CUDA(h, small_gemm(h->st, k, k, k, h->R1, 1, L.kp, bufs[which], 1, L.kp, bufs[1 - which], 1, L.kp,
-                                false));
-          which = 1 - which;
-        }
-      }
-      src = dst;
-      ld_src = ld_dst;
-    }
-    {
-      Scope sc(h, "other", 2.0 * k * static_cast<double>(k) * n);
-      // R = Rbar [I_k T]
-      RS_CUDA(h, copy_2d(h->st, bufs[which], L.kp, R, ldr, k, k));
-      if (n > k)
-        RS_CUDA(h, small_gemm(h->st, k, static_cast<int>(n - k), k, bufs[which], 1, L.kp, h->T, 1, L.kp,
-                              R + static_cast<long long>(k) * ldr, 1, ldr, false));
-    }
-    return sync_and_check(h);
-  };
-  // CholQR2; on breakdown (kappa(A P_1)^2 u > 1, e.g. an adaptive l past the numerical rank)
-  // shifted CholQR with 2, then 4 shifted passes ahead of the two plain ones (R20)
-  s = run(2, 0);
+  rs_status_t s = check_factor_args(h, A, lda, Q, ldq, R, ldr);
+  if (s != RS_OK) return s;
+  s = enqueue_factor(h, A, lda, Q, ldq, R, ldr, 2, 0);
+  if (s == RS_OK) s = sync_and_check(h);
   h->factor_shifts = 0;
-  for (int nshift = 2; s == RS_ERR_NOT_SPD && nshift <= 4; nshift += 2) {
-    RS_CUDA(h, cudaMemsetAsync(h->info, 0, 16, h->st));
-    s = run(nshift + 2, nshift);
-    h->factor_shifts = nshift;
-  }
+  if (s == RS_ERR_NOT_SPD) s = factor_fallback(h, A, lda, Q, ldq, R, ldr);
   if (s != RS_OK) return s;
   h->state = ST_FACTORED;
   return RS_OK;
+}
+
+rs_status_t rs_lowrank_run(rs_lowrank_t h, const double* A, int64_t lda, int32_t q, int64_t* perm, double* Q,
+                           int64_t ldq, double* R, int64_t ldr) {
+  if (!h) return RS_ERR_INVALID_ARG;
+  if (q < 0) return fail(h, RS_ERR_INVALID_ARG, "q < 0");
+  rs_status_t s;
+  if (h->m_local > 0 && (s = check_matrix(h, A, lda, h->m_local, "A")) != RS_OK) return s;
+  if ((s = check_factor_args(h, A, lda, Q, ldq, R, ldr)) != RS_OK) return s;
+  h->k = h->k0;  // a fixed-rank run (an earlier adaptive sample set k = l)
+  h->ell = h->L.ell;
+  h->adaptive = false;
+  if (!h->ar_fn && !h->graph_disabled) {
+    const std::vector<long long> key = {reinterpret_cast<long long>(A), lda, q, reinterpret_cast<long long>(perm),
+                                        reinterpret_cast<long long>(Q), ldq, reinterpret_cast<long long>(R), ldr,
+                                        h->prof ? 1 : 0};
+    if (!h->gexec || key != h->gkey) {
+      if ((s = capture_step(h, A, lda, q, perm, Q, ldq, R, ldr)) != RS_OK) return s;
+      if (h->gexec) h->gkey = key;
+    }
+    if (h->gexec) {
+      RS_CUDA(h, cudaGraphLaunch(h->gexec, h->st));
+      s = sync_and_check(h);
+      if (h->prof) drain_graph_scopes(h);
+      if (s == RS_OK) {
+        h->state = ST_FACTORED;
+        h->powers = q;
+        h->robust_iters = 0;
+        h->factor_shifts = 0;
+        h->pow_A = A;
+        h->pow_lda = lda;
+        h->pow_q = q;
+        h->gaps_valid = false;
+        return RS_OK;
+      }
+      if (s != RS_INFO_REPLAY && s != RS_ERR_NOT_SPD) return s;
+      // a CholQR breakdown somewhere in the step: redo it through the phases, which apply the
+      // shifted-CholQR fallbacks (R20) where the breakdown happened
+      RS_CUDA(h, cudaMemsetAsync(h->info, 0, 16, h->st));
+    }
+  }
+  if ((s = rs_lowrank_sample(h, A, lda)) != RS_OK) return s;
+  if ((s = rs_lowrank_power_iterate(h, A, lda, q)) != RS_OK) return s;
+  if ((s = rs_lowrank_pivot(h, perm)) != RS_OK) return s;
+  return rs_lowrank_factor(h, A, lda, Q, ldq, R, ldr);
 }
 
 // ---------------------------------------------------------------------------------------------
@@ -929,6 +1167,7 @@ rs_status_t rs_lowrank_sample_adaptive(rs_lowrank_t h, const double* A, int64_t 
   h->ell = l;
   h->k = l;
   h->adaptive = true;
+  h->pow_q = 0;
   h->state = ST_SAMPLED;
   h->powers = q;
   if (ell_out) *ell_out = l;
@@ -943,11 +1182,8 @@ rs_status_t rs_lowrank_run_host(rs_lowrank_t h, const double* A_host, int64_t ld
   const long long ml = h->m_local, n = h->n;
   if (ml > 0)
     RS_CUDA(h, cudaMemcpy2DAsync(A_dev, ld_dev * 8, A_host, lda * 8, ml * 8, n, cudaMemcpyHostToDevice, h->st));
-  rs_status_t s = rs_lowrank_sample(h, A_dev, ld_dev);
+  rs_status_t s = rs_lowrank_run(h, A_dev, ld_dev, q, nullptr, Q_dev, ld_qdev, R_dev, ld_rdev);
   if (s != RS_OK) return s;
-  if ((s = rs_lowrank_power_iterate(h, A_dev, ld_dev, q)) != RS_OK) return s;
-  if ((s = rs_lowrank_pivot(h, nullptr)) != RS_OK) return s;
-  if ((s = rs_lowrank_factor(h, A_dev, ld_dev, Q_dev, ld_qdev, R_dev, ld_rdev)) != RS_OK) return s;
   if (perm_host) RS_CUDA(h, cudaMemcpyAsync(perm_host, h->perm, n * 8, cudaMemcpyDeviceToHost, h->st));
   if (Q_host && ml > 0)
     RS_CUDA(h, cudaMemcpy2DAsync(Q_host, ldq * 8, Q_dev, ld_qdev * 8, ml * 8, h->k, cudaMemcpyDeviceToHost, h->st));
@@ -964,6 +1200,7 @@ rs_status_t rs_lowrank_destroy(rs_lowrank_t h) {
     cudaEventDestroy(p.e0);
     cudaEventDestroy(p.e1);
   }
+  release_graph(h);
   for (auto e : h->event_pool) cudaEventDestroy(e);
   delete h;
   return RS_OK;
@@ -978,6 +1215,12 @@ rs_status_t rs_lowrank_get_sample(rs_lowrank_t h, double* B, int64_t ldb) {
 
 rs_status_t rs_lowrank_set_sample(rs_lowrank_t h, const double* B, int64_t ldb) {
   if (!h || !B || ldb < h->ell) return RS_ERR_INVALID_ARG;
+  // a fixed-rank sample of l = k0 + p rows: undo what an earlier adaptive run set
+  h->ell = h->L.ell;
+  h->k = h->k0;
+  h->adaptive = false;
+  h->robust_iters = 0;
+  h->pow_q = 0;
   RS_CUDA(h, cudaMemcpy2DAsync(h->B, h->L.lp * 8, B, ldb * 8, h->ell * 8, h->n, cudaMemcpyDeviceToDevice, h->st));
   RS_CUDA(h, cudaMemsetAsync(h->info, 0, 16, h->st));
   h->state = ST_SAMPLED;
@@ -995,6 +1238,11 @@ rs_status_t rs_lowrank_get_pivot_data(rs_lowrank_t h, double* T, int64_t ldt, do
   if (Rhat)
     RS_CUDA(h, cudaMemcpy2DAsync(Rhat, ldrh * 8, h->Rhat, h->L.kp * 8, k * 8, h->n, cudaMemcpyDeviceToDevice, h->st));
   RS_CUDA(h, cudaStreamSynchronize(h->st));
+  if (!h->gaps_valid) {  // read lazily: pivot and rs_lowrank_run keep no host copy
+    h->gaps_host.assign(k, 0.0);
+    RS_CUDA(h, cudaMemcpy(h->gaps_host.data(), h->gaps, static_cast<size_t>(k) * 8, cudaMemcpyDeviceToHost));
+    h->gaps_valid = true;
+  }
   if (gaps_host) std::copy(h->gaps_host.begin(), h->gaps_host.end(), gaps_host);
   return RS_OK;
 }
@@ -1125,6 +1373,17 @@ rs_status_t rs_comm_init(void** comm, int32_t nranks, const char id[128], int32_
   ncclComm_t c;
   if (ncclCommInitRank(&c, nranks, uid, rank) != ncclSuccess) return RS_ERR_NCCL;
   *comm = c;
+  return RS_OK;
+}
+
+rs_status_t rs_comm_info(void* comm, int32_t* nranks, int32_t* rank) {
+  if (!comm || !nranks || !rank) return RS_ERR_INVALID_ARG;
+  int n = 0, r = 0;
+  if (ncclCommCount(static_cast<ncclComm_t>(comm), &n) != ncclSuccess ||
+      ncclCommUserRank(static_cast<ncclComm_t>(comm), &r) != ncclSuccess)
+    return RS_ERR_NCCL;
+  *nranks = n;
+  *rank = r;
   return RS_OK;
 }
 

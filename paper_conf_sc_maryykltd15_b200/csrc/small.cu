@@ -221,12 +221,9 @@ cudaError_t trsm_upper_cols(cudaStream_t st, const double* U, int ldu, int k, co
   if (ncols <= 0) return cudaSuccess;
   if (k <= 128) {
     const size_t smem2 = (static_cast<size_t>(k) * k + k + static_cast<size_t>(TRSM2_WARPS) * k) * 8;
-    static bool attr2 = false;
-    if (!attr2) {
-      cudaError_t e = cudaFuncSetAttribute(trsm_upper_cols_smem_kernel, cudaFuncAttributeMaxDynamicSharedMemorySize,
-                                           static_cast<int>((128 * 128 + 128 + TRSM2_WARPS * 128) * 8));
+    {
+      cudaError_t e = ensure_smem(trsm_upper_cols_smem_kernel, static_cast<int>((128 * 128 + 128 + TRSM2_WARPS * 128) * 8));
       if (e != cudaSuccess) return e;
-      attr2 = true;
     }
     const int blocks = static_cast<int>(std::min<long long>((ncols + TRSM2_WARPS - 1) / TRSM2_WARPS, 148LL));
     trsm_upper_cols_smem_kernel<<<blocks, TRSM2_WARPS * 32, smem2, st>>>(U, ldu, k, Y, ldy, ncols, X, ldx);
@@ -235,12 +232,9 @@ cudaError_t trsm_upper_cols(cudaStream_t st, const double* U, int ldu, int k, co
   }
   const size_t smem = static_cast<size_t>(TRSM_WARPS) * k * 8;
   if (smem > 220 * 1024) return cudaErrorInvalidValue;
-  static bool attr = false;
-  if (!attr) {
-    cudaError_t e =
-        cudaFuncSetAttribute(trsm_upper_cols_kernel, cudaFuncAttributeMaxDynamicSharedMemorySize, 220 * 1024);
+  {
+    cudaError_t e = ensure_smem(trsm_upper_cols_kernel, 220 * 1024);
     if (e != cudaSuccess) return e;
-    attr = true;
   }
   const int blocks = static_cast<int>(std::min<long long>((ncols + TRSM_WARPS - 1) / TRSM_WARPS, 148LL * 16));
   trsm_upper_cols_kernel<<<blocks, TRSM_WARPS * 32, smem, st>>>(U, ldu, k, Y, ldy, ncols, X, ldx);

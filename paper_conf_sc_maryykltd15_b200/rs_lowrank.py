@@ -26,12 +26,13 @@ STATUS = {0: "RS_OK", 1: "RS_ERR_INVALID_ARG", 2: "RS_ERR_BAD_STATE", 3: "RS_ERR
 
 ABI_FUNCTIONS = (
     "rs_lowrank_workspace_bytes", "rs_lowrank_create", "rs_lowrank_sample", "rs_lowrank_power_iterate",
-    "rs_lowrank_pivot", "rs_lowrank_factor", "rs_lowrank_run_host", "rs_lowrank_sample_adaptive",
+    "rs_lowrank_pivot", "rs_lowrank_factor", "rs_lowrank_run", "rs_lowrank_run_host", "rs_lowrank_sample_adaptive",
     "rs_lowrank_destroy",
     "rs_lowrank_get_sample", "rs_lowrank_set_sample", "rs_lowrank_get_pivot_data", "rs_lowrank_omega",
     "rs_lowrank_get_info", "rs_lowrank_get_fallbacks", "rs_lowrank_set_profiling", "rs_lowrank_get_profile", "rs_lowrank_reset_profile",
     "rs_lowrank_kernel_launches", "rs_qp3_workspace_bytes", "rs_qp3_truncated", "rs_lowrank_sample_columns",
     "rs_lowrank_last_error", "rs_lowrank_set_allreduce_hook", "rs_comm_get_unique_id", "rs_comm_init", "rs_comm_destroy",
+    "rs_comm_info",
 )
 
 
@@ -67,6 +68,7 @@ def load_library(path: str = LIB_PATH):
         "rs_lowrank_power_iterate": (ctypes.c_int, [P, P, I64, I32]),
         "rs_lowrank_pivot": (ctypes.c_int, [P, P]),
         "rs_lowrank_factor": (ctypes.c_int, [P, P, I64, P, I64, P, I64]),
+        "rs_lowrank_run": (ctypes.c_int, [P, P, I64, I32, P, P, I64, P, I64]),
         "rs_lowrank_run_host": (ctypes.c_int, [P, P, I64, P, I64, I32, P, P, I64, P, I64, P, I64, P, I64]),
         "rs_lowrank_sample_adaptive": (ctypes.c_int, [P, P, I64, ctypes.c_double, I32, I32, I32, ctypes.POINTER(I32),
                                                       D, D, I32]),
@@ -89,6 +91,7 @@ def load_library(path: str = LIB_PATH):
         "rs_comm_get_unique_id": (ctypes.c_int, [ctypes.c_char_p]),
         "rs_comm_init": (ctypes.c_int, [ctypes.POINTER(P), I32, ctypes.c_char_p, I32]),
         "rs_comm_destroy": (ctypes.c_int, [P]),
+        "rs_comm_info": (ctypes.c_int, [P, ctypes.POINTER(I32), ctypes.POINTER(I32)]),
     }
     for name, (res, args) in sig.items():
         fn = getattr(lib, name)
@@ -202,6 +205,17 @@ def factor(h: Handle, A: torch.Tensor, Q: torch.Tensor, R: torch.Tensor):
                                             colmajor_ld(Q, "Q"), R.data_ptr(), colmajor_ld(R, "R")), h.ptr)
 
 
+def run(h: Handle, A: torch.Tensor, q: int, perm: torch.Tensor | None, Q: torch.Tensor, R: torch.Tensor):
+    """The whole step (rs_lowrank_run): sample -> power_iterate(q) -> pivot -> factor, replayed as one
+    CUDA graph after the first call with the same buffers."""
+    if perm is not None and (perm.dtype != torch.int64 or not perm.is_cuda):
+        raise ValueError("perm must be a CUDA int64 tensor")
+    _check(load_library().rs_lowrank_run(h.ptr, A.data_ptr(), colmajor_ld(A, "A"), q,
+                                         perm.data_ptr() if perm is not None else None, Q.data_ptr(),
+                                         colmajor_ld(Q, "Q"), R.data_ptr(), colmajor_ld(R, "R")), h.ptr)
+    h.adaptive_ell = 0
+
+
 def run_host(h: Handle, A_host: torch.Tensor, A_dev: torch.Tensor, q: int, perm_host: torch.Tensor,
              Q_host: torch.Tensor, R_host: torch.Tensor, Q_dev: torch.Tensor, R_dev: torch.Tensor):
     _check(load_library().rs_lowrank_run_host(
@@ -260,6 +274,7 @@ def get_sample(h: Handle) -> torch.Tensor:
 
 def set_sample(h: Handle, B: torch.Tensor):
     _check(load_library().rs_lowrank_set_sample(h.ptr, B.data_ptr(), colmajor_ld(B, "B")), h.ptr)
+    h.adaptive_ell = 0
 
 
 def get_pivot_data(h: Handle):
@@ -386,6 +401,13 @@ def comm_init(nranks: int, uid: bytes, rank: int) -> int:
     c = ctypes.c_void_p()
     _check(load_library().rs_comm_init(ctypes.byref(c), nranks, uid, rank))
     return c.value
+
+
+def comm_info(comm: int) -> tuple[int, int]:
+    """(nranks, rank) of an NCCL communicator made by comm_init."""
+    n, r = ctypes.c_int32(), ctypes.c_int32()
+    _check(load_library().rs_comm_info(comm, ctypes.byref(n), ctypes.byref(r)))
+    return int(n.value), int(r.value)
 
 
 def comm_destroy(comm: int):

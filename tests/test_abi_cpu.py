@@ -76,3 +76,14 @@ def test_create_rejects_bad_arguments_without_touching_a_device(lib):
     assert lib.rs_lowrank_create(ctypes.byref(h), 100, 50, 60, 30, 4, 4, 1, ws, 0, None, None) == 1
     assert lib.rs_lowrank_create(None, 100, 100, 0, 30, 4, 4, 1, ws, 0, None, None) == 1
     assert lib.rs_lowrank_destroy(None) == 1
+
+
+def test_no_runtime_development_switches(lib):
+    """A/B switches are compile-time only (-DRS_DEV_*): the shipped library reads no RS_* variable."""
+    from paper_conf_sc_maryykltd15_b200.rs_lowrank import LIB_PATH
+
+    strs = subprocess.run(["strings", LIB_PATH], capture_output=True, text=True).stdout
+    for name in ("RS_PHILOX_GENMODE", "RS_PHILOX_CLUSTER", "RS_KC_NO_PWG", "RS_MC_NO_PWG", "RS_MC_WM",
+                 "RS_MC_NO_TMA3D", "RS_MC_NO_PERSIST", "RS_QRCP_SMEM", "RS_QRCP_TIMING", "RS_QRCP_BARRIER",
+                 "RS_CHOL_BLOCKED", "RS_CHOL_TPT", "RS_CHOL_SMEM_MAX_N"):
+        assert name not in strs, name

@@ -25,7 +25,7 @@ from paper_conf_sc_maryykltd15_b200.partition import row_split  # noqa: E402
 from synth.matrices import make_matrix  # noqa: E402
 
 SEED = 0x5C15
-_OVERLAP = os.environ.get("RS_MR_OVERLAP") == "1"  # debugging: let the ranks' kernels overlap
+_SERIAL = os.environ.get("RS_MR_SERIAL") == "1"  # debugging: serialise the ranks' library calls
 
 
 @pytest.fixture(scope="module", autouse=True)
@@ -47,11 +47,10 @@ class _DevBuf:
 class InProcessAllreduce:
     """Sum over N handles in one process.  Every rank syncs its stream and parks its buffer; rank 0
     copies the N buffers to the host, sums them in rank order (deterministic, plain numpy) and writes
-    the sum back to every buffer before any rank continues.  A token serialises the ranks' library
-    calls between reductions, so the N ranks' kernels never overlap on the one GPU -- as with one
-    process per GPU.  (With the ranks' kernels overlapping, the first call of a fresh process gave
-    a ~1e-5 B mismatch in about one process in five under CUDA's lazy module loading, never with
-    CUDA_MODULE_LOADING=EAGER, scripts/debug_multirank*.py.)"""
+    the sum back to every buffer before any rank continues.  Between reductions the N ranks' kernels
+    run concurrently on the one GPU (their streams overlap); RS_MR_SERIAL=1 serialises the ranks'
+    library calls with a token instead (debugging aid; DESIGN.md §7 has the history of the r01
+    overlap finding and the r02 evidence that it does not occur with the current library)."""
 
     def __init__(self, nranks):
         self.n = nranks
@@ -65,7 +64,7 @@ class InProcessAllreduce:
             stream.synchronize()
             self.bufs[rank] = (buf, count)
             self.calls[rank] += 1
-            if not _OVERLAP:
+            if _SERIAL:
                 self.token.release()
             self.barrier.wait()
             if rank == 0:
@@ -82,7 +81,7 @@ class InProcessAllreduce:
                     v.copy_(src)
                 torch.cuda.synchronize()
             self.barrier.wait()
-            if not _OVERLAP:
+            if _SERIAL:
                 self.token.acquire()
 
         return fn
@@ -96,7 +95,7 @@ def _run_ranks(A, nranks, k, p, q):
     dev = torch.device("cuda", 0)
 
     def work(r):
-        if not _OVERLAP:
+        if _SERIAL:
             comm.token.acquire()
         try:
             torch.cuda.set_device(dev)
@@ -125,7 +124,7 @@ def _run_ranks(A, nranks, k, p, q):
             errs[r] = e
             comm.barrier.abort()
         finally:
-            if not _OVERLAP:
+            if _SERIAL:
                 comm.token.release()
 
     ts = [threading.Thread(target=work, args=(r,)) for r in range(nranks)]
@@ -161,8 +160,7 @@ def test_multirank_pipeline_matches_oracle(m, n, k, p, q, nranks):
     assert list(r0["perm"][:kc]) == list(o.perm[:kc])
     if kc == k:
         assert list(r0["perm"]) == list(o.perm)
-        kap11 = np.linalg.cond(o.Rhat[:, :k])
-        assert rel(r0["R"], o.R) <= max(1e-11, 50 * kap11 * 2.0 ** -53)
+        assert rel(r0["R"], o.R) <= 1e-11
         assert rel(Q, o.Q) <= q_tolerance(o.Rbar)
         e = OPL.approx_error(A, r0["perm"], Q, r0["R"])
         assert abs(e - o.err) <= 1e-12, (e, o.err)

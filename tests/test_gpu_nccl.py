@@ -1,6 +1,7 @@
 """The library's NCCL code path (allreduce of B and of every Gram matrix) at world size 1 on the
-GPU: results must be bitwise identical to the communicator-free run (a 1-rank allreduce is a copy),
-and the multi-rank row partition must reproduce the 1-rank sample (global-index Omega)."""
+GPU: ncclAllReduce is called whenever a communicator is attached (counted through the "comm"
+profiling scope), and results must be bitwise identical to the communicator-free run (a 1-rank
+allreduce is a copy) -- through the phases and through the CUDA-graph-captured rs_lowrank_run."""
 
 import os
 
@@ -29,11 +30,21 @@ def test_nccl_world_size_one_matches_no_comm():
         Ad = to_dev(A)
         outs = []
         for c in (None, comm):
-            perm, Q, R, h = rs.rs_lowrank.rs_lowrank(Ad, 40, 10, 1, 0x5C15, nccl_comm=c)
+            h = rs.create(6000, 6000, 0, 500, 40, 10, 0x5C15, nccl_comm=c)
+            rs.set_profiling(h, True)
+            perm, Q, R, _ = rs.rs_lowrank.rs_lowrank(Ad, 40, 10, 1, 0x5C15, h=h)
+            prof = rs.get_profile(h)
+            ncomm = prof.get("comm", {}).get("launches", 0)
+            # B after the sample and after the power pass, 2 Grams of C, 2 k x k Grams of the factor
+            assert ncomm == (6 if c is not None else 0), prof.get("comm")
+            outs.append((to_np(rs.get_sample(h)), perm.cpu().numpy(), to_np(Q), to_np(R)))
+            for _ in range(2):   # capture, then replay
+                rs.run(h, Ad, 1, perm, Q, R)
             outs.append((to_np(rs.get_sample(h)), perm.cpu().numpy(), to_np(Q), to_np(R)))
             rs.destroy(h)
-        for x, y in zip(outs[0], outs[1]):
-            np.testing.assert_array_equal(x, y)
+        for o in outs[1:]:
+            for x, y in zip(outs[0], o):
+                np.testing.assert_array_equal(x, y)
     finally:
         rs.rs_lowrank.comm_destroy(comm)
 

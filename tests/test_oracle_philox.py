@@ -114,3 +114,11 @@ def test_omega_golden_regression(golden_dir):
     want = np.loadtxt(path)
     got = P.omega(4, 0, 16, 0x5C15)
     np.testing.assert_array_equal(got, want)
+
+
+def test_omega_row_subset_equals_full_rows():
+    """omega(..., rows=R) generates only the rows R of the same Omega (per-entry counters)."""
+    from oracle.philox import omega
+
+    full = omega(40, 3, 700, 0x5C15)
+    np.testing.assert_array_equal(omega(40, 3, 700, 0x5C15, rows=[39, 0, 17]), full[[39, 0, 17]])
