@@ -131,6 +131,22 @@ RS_DEVINL void tma_load_3d(void* smem_dst, const CUtensorMap* m, uint64_t* bar, 
 // ---- FP64 tensor core: mma.sync m8n8k4 (lowers to DMMA.8x8x4 on sm_100a) ---------------
 // A fragment: a = A[lane/4][lane%4]; B fragment: b = B[lane%4][lane/4];
 // C/D: d0 = C[lane/4][2*(lane%4)], d1 = C[lane/4][2*(lane%4)+1].
+// Consumer-side release of a TMA / generator ring slot, DEFERRED BY ONE STAGE: called right after
+// the full-barrier wait of stage `it`, it releases the slot of stage it - 1.  A slot may only be
+// refilled once every shared-memory load from it has completed.  Releasing at the end of the
+// stage itself is not enough: ptxas schedules the (lane-0) arrive above the stage's DMMAs, right
+// behind LDS.128s whose data is still in flight, and the producer's next TMA into the slot can
+// then overwrite it before those loads read it -- rare wrong results that showed up with the
+// ranks' kernels overlapping on one GPU.  Here the arrive sits in the basic block
+// after the next stage's wait, so all of stage it - 1's DMMAs -- which consume every one of its
+// loads -- have issued before it.
+RS_DEVINL void ring_release_prev(uint64_t* empty, int it, int ns, int lane) {
+  if (it > 0) {
+    __syncwarp();
+    if (lane == 0) mbar_arrive(&empty[(it - 1) % ns]);
+  }
+}
+
 RS_DEVINL void dmma_8x8x4(double& d0, double& d1, double a, double b) {
   asm volatile("mma.sync.aligned.m8n8k4.row.col.f64.f64.f64.f64 {%0,%1}, {%2}, {%3}, {%0,%1};"
                : "+d"(d0), "+d"(d1)

@@ -418,6 +418,46 @@ cudaError_t gemm_mc(cudaStream_t st, int M, int N, long long K, const View2D& Lv
 #undef RS_MC
 }
 
+template <int NB>
+cudaError_t launch_tsa_t(cudaStream_t st, int grid, const CUtensorMap& tX, const CUtensorMap& tU, const TsaArgs& a) {
+  constexpr int smem = TsaSmem<NB>::TOTAL;
+  cudaError_t e = ensure_smem(tsa_kernel<NB>, smem);
+  if (e != cudaSuccess) return e;
+  tsa_kernel<NB><<<grid, TSA_THREADS, smem, st>>>(tX, tU, a);
+  count_launch();
+  return cudaGetLastError();
+}
+
+cudaError_t gemm_tsa(cudaStream_t st, long long m, int k, const View2D& Xv, const double* W, long long ldw, double* Y,
+                     long long ldy, int n_store) {
+  if (k < 1 || k > 128 || m < 0) return cudaErrorNotSupported;
+  if (m == 0) return cudaSuccess;
+  const int NB = (k + 15) / 16;
+  TsaArgs a{};
+  a.y = Y;
+  a.ldy = ldy;
+  a.m = static_cast<int>(m);
+  a.n_store = std::min(n_store, 16 * NB);
+  a.ntiles = static_cast<int>((m + 127) / 128);
+  CUtensorMap tX, tU;
+  const View2D Uv{W, k, k, ldw};
+  a.x3d = make_tmap3(&tX, Xv, 8);
+  a.u3d = make_tmap3(&tU, Uv, static_cast<uint32_t>(NB));
+  if (!a.x3d && !make_tmap(&tX, Xv, 16, 16)) return cudaErrorInvalidValue;
+  if (!a.u3d && !make_tmap(&tU, Uv, 16, 16)) return cudaErrorInvalidValue;
+  const int grid = std::min(a.ntiles, num_sms_cached());
+  switch (NB) {
+    case 1: return launch_tsa_t<1>(st, grid, tX, tU, a);
+    case 2: return launch_tsa_t<2>(st, grid, tX, tU, a);
+    case 3: return launch_tsa_t<3>(st, grid, tX, tU, a);
+    case 4: return launch_tsa_t<4>(st, grid, tX, tU, a);
+    case 5: return launch_tsa_t<5>(st, grid, tX, tU, a);
+    case 6: return launch_tsa_t<6>(st, grid, tX, tU, a);
+    case 7: return launch_tsa_t<7>(st, grid, tX, tU, a);
+    default: return launch_tsa_t<8>(st, grid, tX, tU, a);
+  }
+}
+
 cudaError_t gemm_syrk(cudaStream_t st, int rows, long long K, const View2D& Xv, const GemmOutDesc& out, int splits) {
   if (rows < 1 || rows > 128) return cudaErrorInvalidValue;
   const int R = (rows + 15) / 16;

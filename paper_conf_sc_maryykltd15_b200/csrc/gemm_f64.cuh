@@ -205,15 +205,15 @@ __global__ void __launch_bounds__(GEMM_THREADS, 1)
 
   for (int it = 0; it < nk; ++it) {
     const int s = it % SM::NS;
-    if (threadIdx.x == 0 && it + SM::NS - 1 < nk) issue(it + SM::NS - 1);
     mbar_wait(&full[s], (it / SM::NS) & 1);
+    ring_release_prev(empty, it, SM::NS, lane);
+    // refill the slot of stage it - 1 (waits until every warp has released it)
+    if (threadIdx.x == 0 && it + SM::NS - 1 < nk) issue(it + SM::NS - 1);
     const unsigned char* Ls = sL + s * SM::L_BYTES;
     const unsigned char* Rs = sR + s * SM::R_BYTES;
     kc_stage_mma<MFW>(
         acc, [&](int mf, int p) { return *reinterpret_cast<const double2*>(Ls + kc_pair_off(rowL(mf), p, kk)); },
         [&](int nf, int p) { return *reinterpret_cast<const double2*>(Rs + kc_pair_off(rowR(nf), p, kk)); });
-    __syncwarp();
-    if (lane == 0) mbar_arrive(&empty[s]);
   }
   kc_store<MFW>(acc, a.out, m0, n0, wn, kk, rowL);
 }
@@ -287,13 +287,12 @@ __global__ void __launch_bounds__(KCP_THREADS, 1)
   for (int it = 0; it < nk; ++it) {
     const int s = it % SM::NS;
     mbar_wait(&full[s], (it / SM::NS) & 1);
+    ring_release_prev(empty, it, SM::NS, lane);
     const unsigned char* Ls = sL + s * SM::L_BYTES;
     const unsigned char* Rs = sR + s * SM::R_BYTES;
     kc_stage_mma<MFW>(
         acc, [&](int mf, int p) { return *reinterpret_cast<const double2*>(Ls + kc_pair_off(rowL(mf), p, kk)); },
         [&](int nf, int p) { return *reinterpret_cast<const double2*>(Rs + kc_pair_off(rowR(nf), p, kk)); });
-    __syncwarp();
-    if (lane == 0) mbar_arrive(&empty[s]);
   }
   kc_store<MFW>(acc, a.out, m0, n0, wn, kk, rowL);
 }
@@ -344,7 +343,11 @@ __global__ void __launch_bounds__(PHX_THREADS, 1)
   if (threadIdx.x == 0) {
 #pragma unroll
     for (int s = 0; s < SM::NS; ++s) {
+#ifdef RS_PHX_THREAD_ARRIVE
+      mbar_init(&full[s], 1 + GRP_WARPS * 32);  // TMA producer + every generator thread (+ peers' tx bytes)
+#else
       mbar_init(&full[s], 1 + GRP_WARPS);  // TMA producer + the stage's generator warps (+ peers' tx bytes)
+#endif
       mbar_init(&empty[s], NCONS * CS);
     }
     fence_mbar_init();
@@ -410,8 +413,12 @@ __global__ void __launch_bounds__(PHX_THREADS, 1)
           }
         }
       }
+#ifdef RS_PHX_THREAD_ARRIVE
+      mbar_arrive(&full[s]);  // each thread releases its own stores
+#else
       __syncwarp();
       if (lane == 0) mbar_arrive(&full[s]);
+#endif
     }
   } else {
     // ------------------------- MMA warpgroups -------------------------
@@ -434,18 +441,22 @@ __global__ void __launch_bounds__(PHX_THREADS, 1)
       // CTA-scope wait: the slot's data is in this CTA's shared memory (no L1 to invalidate);
       // the remote generators' stores are ordered before their release.cluster arrive
       mbar_wait(&full[s], (it / SM::NS) & 1);
+      if (it > 0) {  // deferred release of stage it - 1 (ring_release_prev), here and in the peers
+        const int sp = (it - 1) % SM::NS;
+        __syncwarp();
+        if (lane == 0) {
+          mbar_arrive(&empty[sp]);
+#pragma unroll
+          for (int pc = 1; pc < CS; ++pc)
+            mbar_arrive_remote_cta(mapa_shared(smem_u32(&empty[sp]), (crank + pc) % CS));
+        }
+      }
       const double* Ls = reinterpret_cast<const double*>(sL + s * SM::L_BYTES);
       const unsigned char* Rs = sR + s * SM::R_BYTES;
       kc_stage_mma<MFW>(
           acc,
           [&](int mf, int p) { return *reinterpret_cast<const double2*>(Ls + rowL(mf) * PHX_LD + 8 * p + 2 * kk); },
           [&](int nf, int p) { return *reinterpret_cast<const double2*>(Rs + kc_pair_off(rowR(nf), p, kk)); });
-      __syncwarp();
-      if (lane == 0) {
-        mbar_arrive(&empty[s]);
-#pragma unroll
-        for (int pc = 1; pc < CS; ++pc) mbar_arrive_remote_cta(mapa_shared(smem_u32(&empty[s]), (crank + pc) % CS));
-      }
     }
     kc_store<MFW>(acc, a.out, m0, n0, wn, kk, rowL);
   }
@@ -606,8 +617,9 @@ __global__ void __launch_bounds__(GEMM_THREADS, 1)
 
   for (int it = 0; it < nk; ++it) {
     const int s = it % MC_NS;
-    if (threadIdx.x == 0 && it + MC_NS - 1 < nk) issue(it + MC_NS - 1);
     mbar_wait(&full[s], (it / MC_NS) & 1);
+    ring_release_prev(empty, it, MC_NS, lane);
+    if (threadIdx.x == 0 && it + MC_NS - 1 < nk) issue(it + MC_NS - 1);
     const long long kc = kb + static_cast<long long>(it) * KT;  // first K of the stage
     const unsigned char* Ls = sL + s * SM::L_BYTES;
     const unsigned char* Rs = sR + s * SM::R_BYTES;
@@ -616,8 +628,6 @@ __global__ void __launch_bounds__(GEMM_THREADS, 1)
       mc_stage<NFR, 0, NB, TRI>(acc, Ls, Rs, nbox0, r, kk, kc, m0, n0);
     else
       mc_stage<NFR, NFR, NB, TRI>(acc, Ls, Rs, nbox0, r, kk, kc, m0, n0);
-    __syncwarp();
-    if (lane == 0) mbar_arrive(&empty[s]);
   }
 
   // ---- epilogue: stage the MT x NT tile in shared memory, then coalesced 16-byte stores ----
@@ -757,6 +767,7 @@ __global__ void __launch_bounds__(KCP_THREADS, 1)
   for (int it = 0; it < nk; ++it) {
     const int s = it % MC_NS;
     mbar_wait(&full[s], (it / MC_NS) & 1);
+    ring_release_prev(empty, it, MC_NS, lane);
     const long long kc = kb + static_cast<long long>(it) * KT;  // first K of the stage
     const unsigned char* Ls = sL + s * SM::L_BYTES;
     const unsigned char* Rs = sR + s * SM::R_BYTES;
@@ -765,8 +776,6 @@ __global__ void __launch_bounds__(KCP_THREADS, 1)
       mc_stage<NFR, 0, NB, TRI>(acc, Ls, Rs, nbox0, r, kk, kc, m0, n0);
     else
       mc_stage<NFR, NFR, NB, TRI>(acc, Ls, Rs, nbox0, r, kk, kc, m0, n0);
-    __syncwarp();
-    if (lane == 0) mbar_arrive(&empty[s]);
   }
 
   // ---- epilogue: stage the MT x NT tile in shared memory, then coalesced 16-byte stores ----
@@ -1081,8 +1090,9 @@ __global__ void __launch_bounds__(GEMM_THREADS, 1)
     for (int it = 0; it < nk; ++it) {
       const int g = i * nk + it;
       const int s = g % MCP_NS;
-      if (threadIdx.x == 0 && g + MCP_NS - 1 < total) issue(g + MCP_NS - 1);
       mbar_wait(&full[s], (g / MCP_NS) & 1);
+      ring_release_prev(empty, g, MCP_NS, lane);  // the ring runs on across tiles
+      if (threadIdx.x == 0 && g + MCP_NS - 1 < total) issue(g + MCP_NS - 1);
       const long long kc = static_cast<long long>(it) * KT;
       bool nl[2];
 #pragma unroll
@@ -1096,8 +1106,6 @@ __global__ void __launch_bounds__(GEMM_THREADS, 1)
         else
           mcp_stage<MFW, TRI, FM1, NFR>(acc, Ls, Rs, nbx, nl, r, kk, kc, m0);
       }
-      __syncwarp();
-      if (lane == 0) mbar_arrive(&empty[s]);
     }
     if (wm == 0)
       mcp_store<MFW, TRI, FM0, NFR>(acc, o, nbx, r, kk, m0, n0);
@@ -1162,10 +1170,9 @@ RS_DEVINL void syrk_warp(const unsigned char* sX, uint64_t* full, uint64_t* empt
     // no blocks: still release every slot so the producer can refill it
     for (int it = 0; it < nk; ++it) {
       const int s = it % SYRK_NS;
-      if (threadIdx.x == 0 && it + SYRK_NS - 1 < nk) issue(it + SYRK_NS - 1);
       mbar_wait(&full[s], (it / SYRK_NS) & 1);
-      __syncwarp();
-      if (lane == 0) mbar_arrive(&empty[s]);
+      ring_release_prev(empty, it, SYRK_NS, lane);
+      if (threadIdx.x == 0 && it + SYRK_NS - 1 < nk) issue(it + SYRK_NS - 1);
     }
     return;
   } else {
@@ -1179,8 +1186,9 @@ RS_DEVINL void syrk_warp(const unsigned char* sX, uint64_t* full, uint64_t* empt
         for (int f2 = 0; f2 < 2; ++f2) acc[b][f][f2][0] = acc[b][f][f2][1] = 0.0;
     for (int it = 0; it < nk; ++it) {
       const int s = it % SYRK_NS;
-      if (threadIdx.x == 0 && it + SYRK_NS - 1 < nk) issue(it + SYRK_NS - 1);
       mbar_wait(&full[s], (it / SYRK_NS) & 1);
+      ring_release_prev(empty, it, SYRK_NS, lane);
+      if (threadIdx.x == 0 && it + SYRK_NS - 1 < nk) issue(it + SYRK_NS - 1);
       const unsigned char* Xs = sX + s * SyrkSmem<R>::X_BYTES;
 #pragma unroll
       for (int p = 0; p < 2; ++p) {
@@ -1205,8 +1213,6 @@ RS_DEVINL void syrk_warp(const unsigned char* sX, uint64_t* full, uint64_t* empt
             }
         }
       }
-      __syncwarp();
-      if (lane == 0) mbar_arrive(&empty[s]);
     }
     // G[kc_row(I, f, r)][kc_row(J, f2, 2kk + e)] and its mirror
 #pragma unroll
@@ -1274,6 +1280,128 @@ __global__ void __launch_bounds__(GEMM_THREADS, 1)
     case 5: syrk_warp<R, 5>(sX, full, empty, nk, lane, issue, out, ld, ns); break;
     case 6: syrk_warp<R, 6>(sX, full, empty, nk, lane, issue, out, ld, ns); break;
     default: syrk_warp<R, 7>(sX, full, empty, nk, lane, issue, out, ld, ns); break;
+  }
+}
+
+// ------------------------------------------------------------------------------------------
+// TSA: Y = X U for a tall column-major X (m x k, k <= 128) and an upper-triangular U (k x k):
+// the CholQR applies of Fig. 2 -- C1 = L^{-1} C of the power iteration, seen as
+// C1^T = C^T L^{-T}, and Q1 = (A P1) R^{-1} of step 3.  Persistent CTAs
+// walk 128-row tiles of X through a TMA ring (one dedicated producer warp) while U stays resident
+// in shared memory.  MMA warp w owns rows 16w .. 16w + 15 of the tile and ALL NB column boxes,
+// so every warp runs the same fully unrolled schedule with no runtime branches: column box nb is
+// live in K stages 0..nb only (U[t][j] = 0 for t > j; the skipped terms are exact zeros).
+// Operand layouts are the MC family's (X: M-contiguous boxes, U: N-contiguous boxes, 128B
+// swizzle, fragment pairs by LDS.128).  The epilogue stores row pairs (2r, 2r+1) as 16-byte runs.
+// ------------------------------------------------------------------------------------------
+constexpr int TSA_NS = 6;
+constexpr int TSA_THREADS = (NCONS + 1) * 32;  // 8 MMA warps + 1 producer warp
+
+template <int NB>
+struct TsaSmem {
+  static constexpr int STAGE = 128 * KT * 8;  // one K stage of a 128-row X tile (8 boxes)
+  static constexpr int UST = NB * 2048;       // one K stage of U (NB boxes)
+  static constexpr int RES = NB * UST;
+  static constexpr int TOTAL = 1024 + RES + TSA_NS * STAGE + (2 * TSA_NS + 1) * 8;
+};
+
+struct TsaArgs {
+  double* y;
+  long long ldy;
+  int m, n_store, ntiles;
+  int x3d, u3d;
+};
+
+template <int NB>
+__global__ void __launch_bounds__(TSA_THREADS, 1)
+    tsa_kernel(const __grid_constant__ CUtensorMap tmX, const __grid_constant__ CUtensorMap tmU, const TsaArgs a) {
+  using SM = TsaSmem<NB>;
+  extern __shared__ unsigned char smem_raw[];
+  unsigned char* smem = align1024(smem_raw);
+  unsigned char* sU = smem;
+  unsigned char* sX = smem + SM::RES;
+  uint64_t* full = reinterpret_cast<uint64_t*>(sX + TSA_NS * SM::STAGE);
+  uint64_t* empty = full + TSA_NS;
+  uint64_t* resb = empty + TSA_NS;
+  const int warp = threadIdx.x >> 5, lane = threadIdx.x & 31;
+  const int mytiles = blockIdx.x < a.ntiles ? (a.ntiles - blockIdx.x + gridDim.x - 1) / gridDim.x : 0;
+  const int total = mytiles * NB;
+  if (threadIdx.x == 0) {
+#pragma unroll
+    for (int s = 0; s < TSA_NS; ++s) {
+      mbar_init(&full[s], 1);
+      mbar_init(&empty[s], NCONS);
+    }
+    mbar_init(resb, 1);
+    fence_mbar_init();
+  }
+  __syncthreads();
+  if (warp == NCONS) {  // producer
+    if (lane == 0) {
+      tma_prefetch_desc(&tmX);
+      tma_prefetch_desc(&tmU);
+      mbar_arrive_expect_tx(resb, static_cast<uint32_t>(SM::RES));
+#pragma unroll 1
+      for (int s = 0; s < NB; ++s) mc_load(sU + s * SM::UST, &tmU, resb, a.u3d, 0, NB, s * KT);
+#pragma unroll 1
+      for (int g = 0; g < total; ++g) {
+        const int s = g % TSA_NS;
+        if (g >= TSA_NS) mbar_wait_sleep(&empty[s], ((g / TSA_NS) - 1) & 1);
+        const int m0 = (blockIdx.x + (g / NB) * gridDim.x) * 128;
+        mbar_arrive_expect_tx(&full[s], SM::STAGE);
+        mc_load(sX + s * SM::STAGE, &tmX, &full[s], a.x3d, m0, 8, (g % NB) * KT);
+      }
+    }
+    return;
+  }
+  mbar_wait(resb, 0);
+  const int r = lane >> 2, kk = lane & 3;
+  int g = 0;
+  for (int i = 0; i < mytiles; ++i) {
+    const int m0 = (blockIdx.x + i * gridDim.x) * 128;
+    double acc[2][NB][2][2];
+#pragma unroll
+    for (int f = 0; f < 2; ++f)
+#pragma unroll
+      for (int nb = 0; nb < NB; ++nb)
+#pragma unroll
+        for (int f2 = 0; f2 < 2; ++f2) acc[f][nb][f2][0] = acc[f][nb][f2][1] = 0.0;
+#pragma unroll
+    for (int s = 0; s < NB; ++s, ++g) {
+      const int slot = g % TSA_NS;
+      mbar_wait(&full[slot], (g / TSA_NS) & 1);
+      ring_release_prev(empty, g, TSA_NS, lane);
+      const unsigned char* Xs = sX + slot * SM::STAGE + warp * 2048;
+      const unsigned char* Us = sU + s * SM::UST;
+#pragma unroll
+      for (int ks = 0; ks < KT / 4; ++ks) {
+        const uint32_t krow = 8 * (ks >> 1) + 2 * kk + (ks & 1);
+        const uint32_t off = krow * 128u + (((static_cast<uint32_t>(r) ^ krow) & 7u) << 4);
+        const double2 a2 = *reinterpret_cast<const double2*>(Xs + off);
+#pragma unroll
+        for (int nb = s; nb < NB; ++nb) {
+          const double2 b2 = *reinterpret_cast<const double2*>(Us + nb * 2048 + off);
+          dmma_8x8x4(acc[0][nb][0][0], acc[0][nb][0][1], a2.x, b2.x);
+          dmma_8x8x4(acc[0][nb][1][0], acc[0][nb][1][1], a2.x, b2.y);
+          dmma_8x8x4(acc[1][nb][0][0], acc[1][nb][0][1], a2.y, b2.x);
+          dmma_8x8x4(acc[1][nb][1][0], acc[1][nb][1][1], a2.y, b2.y);
+        }
+      }
+    }
+    // Y[row, col]: rows 2r (f = 0) and 2r + 1 (f = 1) of the warp's 16, col 16 nb + 2 (2 kk + e) + f2
+    const long long row = static_cast<long long>(m0) + 16 * warp + 2 * r;
+    if (row < a.m) {
+      const bool ok1 = row + 1 < a.m;
+#pragma unroll
+      for (int nb = 0; nb < NB; ++nb)
+#pragma unroll
+        for (int e = 0; e < 2; ++e)
+#pragma unroll
+          for (int f2 = 0; f2 < 2; ++f2) {
+            const int col = 16 * nb + 2 * (2 * kk + e) + f2;
+            if (col < a.n_store) put2(a.y + row + col * a.ldy, acc[0][nb][f2][e], acc[1][nb][f2][e], ok1, 0);
+          }
+    }
   }
 }
 

@@ -42,6 +42,12 @@ cudaError_t gemm_mc(cudaStream_t st, int M, int N, long long K, const View2D& Lv
                     const GemmOutDesc& out, int splits, int tri = 0);
 // G (+split partials) = X X^T for the rows <= 128 rows of a K-contiguous X (Xv: dim0 = K, dim1 =
 // rows); lower-triangle blocks only, stored to both triangles (out.ld_m must be 1).
+// Y = X U for a tall X (Xv: dim0 = m rows, contiguous; dim1 = k <= 128 columns) and an upper-
+// triangular k x k U with U[t][j] = W[j + t * ldw] (the transposed storage of a lower-triangular
+// L^{-1}, or the row-major R^{-1}); Y column-major (ldy), columns < n_store written (n_store <=
+// 16 ceil(k / 16); columns >= k are zero).  Returns cudaErrorNotSupported when k > 128.
+cudaError_t gemm_tsa(cudaStream_t st, long long m, int k, const View2D& Xv, const double* W, long long ldw, double* Y,
+                     long long ldy, int n_store);
 cudaError_t gemm_syrk(cudaStream_t st, int rows, long long K, const View2D& Xv, const GemmOutDesc& out, int splits);
 int gemm_choose_splits(int M, int N, long long K, int max_splits, int num_sms);
 int gemm_nsplit(long long K, int splits);   // splits actually launched for a requested count

@@ -288,6 +288,20 @@ rs_status_t gram_rows_kc(rs_lowrank_t h, const double* X, long long ldx, long lo
   return RS_OK;
 }
 
+// dst := L^{-1} src for the rows [0, rp) of the row-major distributed C blocks (ld ldc; rows >= rr
+// zero): C1^T = C^T L^{-T} on the tall-skinny triangular kernel (L^{-T}[t][j] = Linv[j + t rp], one
+// pass over C); the MC family when rr > 128.
+cudaError_t apply_rows_tri(rs_lowrank_t h, const double* src, int rr, int rp, double* dst) {
+  const long long ml = h->m_local;
+  View2D Xv{src, ml, rr, h->L.ldc};
+  cudaError_t e = gemm_tsa(h->st, ml, rr, Xv, h->Linv, rp, dst, h->L.ldc, rp);
+  if (e != cudaErrorNotSupported) return e;
+  View2D Lv{h->Linv, rp, rp, rp};
+  View2D Cv{src, ml, rp, h->L.ldc};
+  GemmOutDesc out{dst, h->L.ldc, 1, 0, rp, static_cast<int>(ml)};
+  return gemm_mc(h->st, rp, static_cast<int>(ml), rp, Lv, Cv, out, 1, 1);  // Linv lower
+}
+
 // One CholQR pass on a replicated short-wide block X (rp x n, column-major, ld rp; rows >= rr are
 // zero): G = X X^T (+ s I when shift), R^T R = G, Y = R^{-T} X.  The shift
 // s = 11 (n rr + rr (rr+1)) u ||X||_F^2 is shifted CholeskyQR's: breakdown-free for kappa(X) < ~1/u,
@@ -356,10 +370,7 @@ rs_status_t cholqr_dist(rs_lowrank_t h, double* Cn, int rr, int rp, int npass, i
     }
     if (ml > 0) {
       Scope sc(h, "apply", 2.0 * rr * static_cast<double>(rr) * ml);
-      View2D Lv{h->Linv, rp, rp, rp};
-      View2D Cv{src, ml, rp, L.ldc};
-      GemmOutDesc out{dst, L.ldc, 1, 0, rp, static_cast<int>(ml)};
-      RS_CUDA(h, gemm_mc(h->st, rp, static_cast<int>(ml), rp, Lv, Cv, out, 1, 1));  // Linv lower
+      RS_CUDA(h, apply_rows_tri(h, src, rr, rp, dst));
     }
   }
   return RS_OK;
@@ -483,10 +494,7 @@ rs_status_t power_to_b1(rs_lowrank_t h, const double* A, long long lda) {
   }
   if (ml > 0) {
     Scope sc(h, "apply", 2.0 * L.ell * static_cast<double>(L.ell) * ml);
-    View2D Lv{h->Linv, L.lp, L.lp, L.lp};
-    View2D Cv{h->C, ml, L.lp, L.ldc};
-    GemmOutDesc out{h->C1, L.ldc, 1, 0, L.lp, static_cast<int>(ml)};
-    RS_CUDA(h, gemm_mc(h->st, L.lp, static_cast<int>(ml), L.lp, Lv, Cv, out, 1, 1));  // Linv lower
+    RS_CUDA(h, apply_rows_tri(h, h->C, L.ell, L.lp, h->C1));
   }
   if ((s = gram_rows_kc(h, h->C1, L.ldc, ml, L.lp, L.lp)) != RS_OK) return s;
   if ((s = allreduce(h, h->G, static_cast<long long>(L.lp) * L.lp)) != RS_OK) return s;
@@ -638,9 +646,13 @@ rs_status_t enqueue_factor(rs_lowrank_t h, const double* A, long long lda, doubl
     if (ml > 0) {
       Scope sc(h, "factor", 2.0 * k * static_cast<double>(k) * ml);
       View2D Xv{src, ml, k, ld_src};
-      View2D Wv{h->Linv, k, k, L.kp};
-      GemmOutDesc out{dst, 1, ld_dst, 0, static_cast<int>(ml), k};
-      RS_CUDA(h, gemm_mc(h->st, static_cast<int>(ml), k, k, Xv, Wv, out, 1, 2));  // R^-1 upper
+      cudaError_t e = gemm_tsa(h->st, ml, k, Xv, h->Linv, L.kp, dst, ld_dst, k);  // R^-1 upper, resident
+      if (e == cudaErrorNotSupported) {  // k > 128
+        View2D Wv{h->Linv, k, k, L.kp};
+        GemmOutDesc out{dst, 1, ld_dst, 0, static_cast<int>(ml), k};
+        e = gemm_mc(h->st, static_cast<int>(ml), k, k, Xv, Wv, out, 1, 2);
+      }
+      RS_CUDA(h, e);
     }
     {
       Scope sc(h, "other", 2.0 * k * static_cast<double>(k) * k);

@@ -23,7 +23,9 @@ rs.load_library()
 A, _ = make_matrix(a.m, a.n, "exp-k", a.k, seed=7)
 Ad = rs.empty_colmajor(a.m, a.n)
 Ad.copy_(torch.from_numpy(A))
-perm, Q, R, h = rs.rs_lowrank.rs_lowrank(Ad, a.k, a.p, a.q, seed=0x5C15)
+perm, Q, R, h = rs.rs_lowrank.rs_lowrank(Ad, a.k, a.p, a.q, seed=0x5C15)   # the phases
+rs.run(h, Ad, a.q, perm, Q, R)   # the whole step captured as a CUDA graph, then replayed
+rs.run(h, Ad, a.q, perm, Q, R)
 torch.cuda.synchronize()
 rs.destroy(h)
 print("ok", float(np.abs(Q.cpu().numpy().T @ Q.cpu().numpy() - np.eye(a.k)).max()))
