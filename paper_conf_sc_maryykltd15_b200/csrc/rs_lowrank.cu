@@ -137,6 +137,10 @@ struct rs_lowrank_s {
   bool capturing = false;
   bool graph_disabled = false;
   cudaGraphExec_t gexec = nullptr;
+  // the graph is captured on and launched into an internal stream (the caller's stream may be the
+  // legacy default stream, which cannot be captured), fenced with events on both sides
+  cudaStream_t gstream = nullptr;
+  cudaEvent_t gev_in = nullptr, gev_out = nullptr;
   std::vector<long long> gkey;
   std::vector<Pending> gscopes;  // profiling scopes baked into the graph (external event records)
 };
@@ -709,19 +713,31 @@ void release_graph(rs_lowrank_t h) {
 rs_status_t capture_step(rs_lowrank_t h, const double* A, long long lda, int q, int64_t* perm, double* Q,
                          long long ldq, double* R, long long ldr) {
   release_graph(h);
+  if (!h->gstream) {
+    if (cudaStreamCreateWithFlags(&h->gstream, cudaStreamNonBlocking) != cudaSuccess ||
+        cudaEventCreateWithFlags(&h->gev_in, cudaEventDisableTiming) != cudaSuccess ||
+        cudaEventCreateWithFlags(&h->gev_out, cudaEventDisableTiming) != cudaSuccess) {
+      cudaGetLastError();
+      h->graph_disabled = true;
+      return RS_OK;
+    }
+  }
   cudaGraph_t g = nullptr;
-  if (cudaStreamBeginCapture(h->st, cudaStreamCaptureModeThreadLocal) != cudaSuccess) {
+  if (cudaStreamBeginCapture(h->gstream, cudaStreamCaptureModeThreadLocal) != cudaSuccess) {
     cudaGetLastError();
     h->graph_disabled = true;
     return RS_OK;
   }
+  cudaStream_t user = h->st;
+  h->st = h->gstream;  // every enqueue below goes to the capturing stream
   h->capturing = true;
   rs_status_t s = enqueue_sample(h, A, lda);
   if (s == RS_OK && q > 0) s = enqueue_power(h, A, lda, q);
   if (s == RS_OK) s = enqueue_pivot(h, perm);
   if (s == RS_OK) s = enqueue_factor(h, A, lda, Q, ldq, R, ldr, 2, 0);
   h->capturing = false;
-  const cudaError_t ec = cudaStreamEndCapture(h->st, &g);
+  h->st = user;
+  const cudaError_t ec = cudaStreamEndCapture(h->gstream, &g);
   cudaError_t ei = cudaErrorUnknown;
   if (s == RS_OK && ec == cudaSuccess && g) ei = cudaGraphInstantiate(&h->gexec, g, 0);
   if (g) cudaGraphDestroy(g);
@@ -733,6 +749,16 @@ rs_status_t capture_step(rs_lowrank_t h, const double* A, long long lda, int q, 
     h->err.clear();
   }
   return RS_OK;
+}
+
+// one replay, ordered after the work already on the handle's stream and before what follows it
+cudaError_t launch_step(rs_lowrank_t h) {
+  cudaError_t e = cudaEventRecord(h->gev_in, h->st);
+  if (e == cudaSuccess) e = cudaStreamWaitEvent(h->gstream, h->gev_in, 0);
+  if (e == cudaSuccess) e = cudaGraphLaunch(h->gexec, h->gstream);
+  if (e == cudaSuccess) e = cudaEventRecord(h->gev_out, h->gstream);
+  if (e == cudaSuccess) e = cudaStreamWaitEvent(h->st, h->gev_out, 0);
+  return e;
 }
 }  // namespace
 
@@ -897,7 +923,7 @@ rs_status_t rs_lowrank_run(rs_lowrank_t h, const double* A, int64_t lda, int32_t
       if (h->gexec) h->gkey = key;
     }
     if (h->gexec) {
-      RS_CUDA(h, cudaGraphLaunch(h->gexec, h->st));
+      RS_CUDA(h, launch_step(h));
       s = sync_and_check(h);
       if (h->prof) drain_graph_scopes(h);
       if (s == RS_OK) {
@@ -1213,6 +1239,12 @@ rs_status_t rs_lowrank_destroy(rs_lowrank_t h) {
     cudaEventDestroy(p.e1);
   }
   release_graph(h);
+  if (h->gstream) {
+    cudaStreamSynchronize(h->gstream);
+    cudaStreamDestroy(h->gstream);
+    cudaEventDestroy(h->gev_in);
+    cudaEventDestroy(h->gev_out);
+  }
   for (auto e : h->event_pool) cudaEventDestroy(e);
   delete h;
   return RS_OK;

@@ -268,6 +268,34 @@ def test_graph_run_equals_phases_bitwise():
         np.testing.assert_array_equal(g1[key], g2[key])
 
 
+@pytest.mark.parametrize("own_stream", [False, True])
+def test_graph_run_is_captured_once_and_replayed(own_stream):
+    """The first rs_lowrank_run captures (the library's launchers run during the capture), later
+    calls replay the graph (no launcher runs: the launch counter stands still) -- on the legacy
+    default stream as well as on a caller's stream -- and reproduce the first result bitwise."""
+    m, n, k, p, q = 20000, 600, 40, 10, 1
+    A, _ = make_matrix(m, n, "exp-k", k, seed=21)
+    st = torch.cuda.Stream() if own_stream else torch.cuda.default_stream()
+    with torch.cuda.stream(st):
+        Ad = to_dev(A)
+        h = rs.create(m, m, 0, n, k, p, SEED, stream=st)
+        try:
+            perm = torch.empty(n, dtype=torch.int64, device="cuda")
+            Q, R = rs.empty_colmajor(m, k), rs.empty_colmajor(k, n)
+            n0 = rs.kernel_launches()
+            rs.run(h, Ad, q, perm, Q, R)
+            n1 = rs.kernel_launches()
+            Q1, R1 = to_np(Q), to_np(R)
+            for _ in range(3):
+                rs.run(h, Ad, q, perm, Q, R)
+            n2 = rs.kernel_launches()
+            assert n1 > n0 and n2 == n1, (n0, n1, n2)
+            np.testing.assert_array_equal(to_np(Q), Q1)
+            np.testing.assert_array_equal(to_np(R), R1)
+        finally:
+            rs.destroy(h)
+
+
 def test_cfg4_full_size_sampled():
     """BASELINE configs[3] at full size (m = 1e6, n = 5 000, k = 100, p = 10, q = 1) in the launch
     configuration bench.py times (rs_lowrank_run).  The sample B = Omega A is compared entry by
