@@ -343,10 +343,10 @@ __global__ void __launch_bounds__(PHX_THREADS, 1)
   if (threadIdx.x == 0) {
 #pragma unroll
     for (int s = 0; s < SM::NS; ++s) {
-#ifdef RS_PHX_THREAD_ARRIVE
-      mbar_init(&full[s], 1 + GRP_WARPS * 32);  // TMA producer + every generator thread (+ peers' tx bytes)
-#else
+#ifdef RS_PHX_LOCAL_STS
       mbar_init(&full[s], 1 + GRP_WARPS);  // TMA producer + the stage's generator warps (+ peers' tx bytes)
+#else
+      mbar_init(&full[s], 1);  // the TMA producer's arrive; every Omega byte completes as tx (st.async)
 #endif
       mbar_init(&empty[s], NCONS * CS);
     }
@@ -374,7 +374,11 @@ __global__ void __launch_bounds__(PHX_THREADS, 1)
         __syncwarp();
       }
       if (g == 0) {
+#ifdef RS_PHX_LOCAL_STS
         mbar_arrive_expect_tx(&full[s], SM::R_BYTES + (MT - ROWS) * KT * 8);  // A tile + peers' Omega rows
+#else
+        mbar_arrive_expect_tx(&full[s], SM::R_BYTES + MT * KT * 8);  // A tile + all Omega rows
+#endif
         tma_load_2d(sR + s * SM::R_BYTES, &tmR, &full[s], static_cast<int>(kb + static_cast<long long>(it) * KT), n0);
       }
       const long long j0 = a.row_offset + kb + static_cast<long long>(it) * KT;  // global row of A
@@ -398,8 +402,15 @@ __global__ void __launch_bounds__(PHX_THREADS, 1)
             v3 = f4_get(z2, o - 1);
           }
         }
+#ifdef RS_PHX_LOCAL_STS
         reinterpret_cast<double2*>(dst)[0] = make_double2(v0, v1);
         reinterpret_cast<double2*>(dst)[1] = make_double2(v2, v3);
+#else
+        // own ring too by st.async completing tx bytes on full[s]: every Omega byte is counted by
+        // the barrier the MMA warps wait on (no generator arrive to order the stores behind)
+        st_async_v2(mapa_shared(smem_u32(dst), crank), v0, v1, mapa_shared(smem_u32(&full[s]), crank));
+        st_async_v2(mapa_shared(smem_u32(dst), crank) + 16, v2, v3, mapa_shared(smem_u32(&full[s]), crank));
+#endif
         if (CS > 1) {  // the same 32 bytes into every peer's ring; completes tx on its full[s]
           const uint32_t sa = smem_u32(dst);
           const uint32_t fb = smem_u32(&full[s]);
@@ -413,9 +424,7 @@ __global__ void __launch_bounds__(PHX_THREADS, 1)
           }
         }
       }
-#ifdef RS_PHX_THREAD_ARRIVE
-      mbar_arrive(&full[s]);  // each thread releases its own stores
-#else
+#ifdef RS_PHX_LOCAL_STS
       __syncwarp();
       if (lane == 0) mbar_arrive(&full[s]);
 #endif
