@@ -133,13 +133,27 @@ def oracle_sample_run(c: dict, m_s: int) -> dict:
     return {"seconds_sample": sum(t.values()), "seconds_extrapolated": full, "phases": t, "m_sample": m_s}
 
 
-def cpu_threads() -> int:
+def full_oracle_reference(c: dict):
+    """The oracle timed once on the FULL workload (scripts/oracle_full.py, stored under profiles/):
+    context for the bounded in-run sample above, not re-measured here."""
+    path = os.path.join(ROOT, "profiles", f"r02_oracle_full_{c['name']}.json")
+    if not os.path.exists(path):
+        return None
     try:
-        from threadpoolctl import threadpool_info
+        j = json.loads(open(path).read().strip().splitlines()[-1])
+    except (OSError, ValueError, IndexError):
+        return None
+    if (j.get("m"), j.get("n"), j.get("k"), j.get("p"), j.get("q")) != (c["m"], c["n"], c["k"], c["p"], c["q"]):
+        return None
+    return {"value": j["seconds_total"], "unit": "s", "threads": j.get("threads"), "phases_s": j.get("phases_s"),
+            "source": os.path.relpath(path, ROOT)}
 
-        return max([int(i.get("num_threads", 1)) for i in threadpool_info()] + [1])
-    except Exception:  # noqa: BLE001
-        return os.cpu_count() or 1
+
+def cpu_threads() -> int:
+    """Threads the oracle's C GEMM (OpenMP over output tiles) runs with."""
+    from oracle.gemm import default_threads
+
+    return default_threads()
 
 
 def oracle_m_sample(c: dict) -> int:
@@ -166,7 +180,7 @@ def run_reference(args, c):
         "warmup": args.warmup, "ms_per_step": 1e3 * sum(samp) / len(samp), "higher_is_better": False,
         "scaling": "strong", "vs_baseline": None, "dtype": "f64", "data": "synthetic",
         "config": {"workload": describe(c), "m": c["m"], "n": c["n"], "k": c["k"], "p": c["p"], "q": c["q"],
-                   "law": c["law"], "parallelism": "cpu oracle (numpy, BLAS threads)"},
+                   "law": c["law"], "parallelism": "cpu oracle (fixed-order C GEMM, OpenMP over output tiles; numpy Householder)"},
         "cpu_baseline": {"value": v, "unit": "s", "cores": cores, "kind": "oracle",
                          "sample": f"oracle pipeline on the first {m_s} of {c['m']} rows per step; sample/power/"
                                    f"factor time scaled by m/{m_s}, QRCP time unscaled"},
@@ -391,6 +405,9 @@ def run_ours(args, c):
                "sample": f"oracle pipeline on the first {m_s} of {m} rows ({r['seconds_sample']:.1f} s of CPU work); "
                          f"sample/power/factor scaled by m/{m_s}, QRCP unscaled",
                "phases_s": r["phases"]}
+        full = full_oracle_reference(c)
+        if full:
+            cpu["full_size_measured"] = full
 
     phases = {nm: round(v["ms"] / args.steps, 4) for nm, v in prof.items() if v["launches"]}
     line = {

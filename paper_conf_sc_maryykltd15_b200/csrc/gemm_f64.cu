@@ -8,6 +8,8 @@
 
 #include "gemm_f64.cuh"
 #include "internal.h"
+#include "philox.cuh"
+#include "sample_ring.cuh"
 
 namespace rs {
 
@@ -455,6 +457,94 @@ cudaError_t gemm_tsa(cudaStream_t st, long long m, int k, const View2D& Xv, cons
     case 6: return launch_tsa_t<6>(st, grid, tX, tU, a);
     case 7: return launch_tsa_t<7>(st, grid, tX, tU, a);
     default: return launch_tsa_t<8>(st, grid, tX, tU, a);
+  }
+}
+
+// ---- sample GEMM with an L2 ring of Omega chunks (sample_ring.cuh) ----
+SampleRingPlan sample_ring_plan(int N, long long K, int max_splits, int G) {
+  SampleRingPlan p{};
+  p.ntn = (N + NT - 1) / NT;
+  double best = -1.0;
+  for (int s = 1; s <= max_splits; ++s) {
+    const long long kspl = ((K + s - 1) / s + RG_CH - 1) / RG_CH * RG_CH;
+    if (kspl < 4 * RG_CH && s > 1) break;  // keep >= 4 chunks (128 stages) per unit
+    const int sr = static_cast<int>((K + kspl - 1) / kspl);
+    const long long units = static_cast<long long>(p.ntn) * sr;
+    const long long rounds = (units + G - 1) / G;
+    const double eff = static_cast<double>(units) / static_cast<double>(rounds * G) - 1e-4 * sr;
+    if (eff > best + 1e-12) {
+      best = eff;
+      p.S = sr;
+      p.kspl = kspl;
+      p.rounds = static_cast<int>(rounds);
+    }
+  }
+  p.ngroups = p.S + p.rounds;  // gid = split + round < S + rounds
+  return p;
+}
+
+size_t sample_ring_bytes(int M, int N, long long K, int max_splits, int G) {
+  if (M < 1 || M > 128 || K < 8 * RG_CH) return 0;
+  const SampleRingPlan p = sample_ring_plan(N, K, max_splits, G);
+  const int MT = gemm_mtile(M);
+  return static_cast<size_t>(p.ngroups) * RG_R * MT * RG_CH * 8 + 2 * static_cast<size_t>(p.ngroups) * RG_R * 4 + 256;
+}
+
+template <int MFW>
+cudaError_t launch_ring_t(cudaStream_t st, int grid, const CUtensorMap& tA, const CUtensorMap& tW, const GemmArgs& a,
+                          const RingArgs& rg) {
+  constexpr int smem = KCSmem<MFW, false>::TOTAL;
+  cudaError_t e = ensure_smem(kc_sample_ring_kernel<MFW>, smem);
+  if (e != cudaSuccess) return e;
+  void* args[] = {const_cast<CUtensorMap*>(&tA), const_cast<CUtensorMap*>(&tW), const_cast<GemmArgs*>(&a),
+                  const_cast<RingArgs*>(&rg)};
+  e = cudaLaunchCooperativeKernel(reinterpret_cast<void*>(kc_sample_ring_kernel<MFW>), dim3(grid), dim3(RG_THREADS),
+                                  args, smem, st);
+  count_launch();
+  return e != cudaSuccess ? e : cudaGetLastError();
+}
+
+cudaError_t gemm_sample_ring(cudaStream_t st, int M, int N, long long K, const View2D& Av, const PhiloxDesc& phx,
+                             const GemmOutDesc& out, int max_splits, void* ring_ws, size_t ring_bytes,
+                             int* nsplit_out) {
+  const int G = num_sms_cached();
+  if (M < 1 || M > 128 || K < 8 * RG_CH || !phx.enabled) return cudaErrorNotSupported;
+  if (sample_ring_bytes(M, N, K, max_splits, G) > ring_bytes) return cudaErrorNotSupported;
+  const SampleRingPlan p = sample_ring_plan(N, K, max_splits, G);
+  const int MT = gemm_mtile(M);
+  const int mfw = MT / 16;
+  GemmArgs a = make_args(M, N, K, p.S, out);
+  a.key.k0 = static_cast<uint32_t>(phx.seed);
+  a.key.k1 = static_cast<uint32_t>(phx.seed >> 32);
+  a.tag = phx.tag;
+  a.row_offset = phx.row_offset;
+  a.ell = phx.ell;
+  a.omega_row0 = phx.omega_row0;
+  RingArgs rg{};
+  rg.ntn = p.ntn;
+  rg.S = p.S;
+  rg.kspl = p.kspl;
+  rg.nunits = p.ntn * p.S;
+  rg.ring = static_cast<double*>(ring_ws);
+  const size_t ring_elems = static_cast<size_t>(p.ngroups) * RG_R * MT * RG_CH;
+  rg.ready = reinterpret_cast<unsigned int*>(rg.ring + ring_elems);
+  rg.consumed = rg.ready + p.ngroups * RG_R;
+  cudaError_t e = cudaMemsetAsync(rg.ready, 0, 2 * static_cast<size_t>(p.ngroups) * RG_R * 4, st);
+  if (e != cudaSuccess) return e;
+  CUtensorMap tA, tW;
+  if (!make_tmap(&tA, Av, 16, NT)) return cudaErrorInvalidValue;
+  const View2D Wv{rg.ring, RG_CH, static_cast<long long>(p.ngroups) * RG_R * MT, RG_CH};
+  if (!make_tmap(&tW, Wv, 16, static_cast<uint32_t>(MT))) return cudaErrorInvalidValue;
+  if (nsplit_out) *nsplit_out = p.S;
+  switch (mfw) {
+    case 1: return launch_ring_t<1>(st, G, tA, tW, a, rg);
+    case 2: return launch_ring_t<2>(st, G, tA, tW, a, rg);
+    case 3: return launch_ring_t<3>(st, G, tA, tW, a, rg);
+    case 4: return launch_ring_t<4>(st, G, tA, tW, a, rg);
+    case 5: return launch_ring_t<5>(st, G, tA, tW, a, rg);
+    case 6: return launch_ring_t<6>(st, G, tA, tW, a, rg);
+    case 7: return launch_ring_t<7>(st, G, tA, tW, a, rg);
+    default: return launch_ring_t<8>(st, G, tA, tW, a, rg);
   }
 }
 

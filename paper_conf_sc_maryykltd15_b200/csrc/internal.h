@@ -48,6 +48,19 @@ cudaError_t gemm_mc(cudaStream_t st, int M, int N, long long K, const View2D& Lv
 // 16 ceil(k / 16); columns >= k are zero).  Returns cudaErrorNotSupported when k > 128.
 cudaError_t gemm_tsa(cudaStream_t st, long long m, int k, const View2D& Xv, const double* W, long long ldw, double* Y,
                      long long ldy, int n_store);
+// Sample GEMM B = Omega A with Omega generated once per K split into an L2 ring of chunks shared by
+// all N tiles (sample_ring.cuh): split partials into `out` (split_stride), *nsplit_out splits.
+// Returns cudaErrorNotSupported when the shape or the ring workspace does not fit (use gemm_kc).
+struct SampleRingPlan {
+  int ntn, S, rounds, ngroups;
+  long long kspl;
+};
+SampleRingPlan sample_ring_plan(int N, long long K, int max_splits, int G);
+size_t sample_ring_bytes(int M, int N, long long K, int max_splits, int G);
+cudaError_t gemm_sample_ring(cudaStream_t st, int M, int N, long long K, const View2D& Av, const PhiloxDesc& phx,
+                             const GemmOutDesc& out, int max_splits, void* ring_ws, size_t ring_bytes,
+                             int* nsplit_out);
+int num_sms_cached();
 cudaError_t gemm_syrk(cudaStream_t st, int rows, long long K, const View2D& Xv, const GemmOutDesc& out, int splits);
 int gemm_choose_splits(int M, int N, long long K, int max_splits, int num_sms);
 int gemm_nsplit(long long K, int splits);   // splits actually launched for a requested count

@@ -46,7 +46,8 @@ struct Layout {
   int smax;          // max split-K partial tiles of an l x n product
   long long part_elems;
   size_t off_B, off_B0, off_Bt, off_B1, off_C, off_C1, off_part, off_G, off_Rf, off_Linv, off_cholw, off_Rho, off_Rhat,
-      off_T, off_Q1, off_R1, off_R2, off_Rbar, off_perm, off_info, off_qr, off_gaps;
+      off_T, off_Q1, off_R1, off_R2, off_Rbar, off_perm, off_info, off_qr, off_gaps, off_ring;
+  size_t ring_bytes;  // Omega chunk ring of the sample GEMM (0: the cluster kernel generates in smem)
   size_t total;
 };
 
@@ -93,6 +94,10 @@ Layout plan(long long m_local, long long n, int k, int p) {
   L.off_info = take(64);
   L.off_qr = take(qrcp_workspace_bytes(L.ell, n));
   L.off_gaps = take(static_cast<size_t>(std::max(k, 1)) * 8);
+  // sized for a 148-SM B200; a device with other SM counts re-plans at launch (and falls back to the
+  // cluster kernel if the ring does not fit)
+  L.ring_bytes = sample_ring_bytes(L.lp, static_cast<int>(n), m_local, L.smax, 148);
+  L.off_ring = take(L.ring_bytes);
   L.total = off + 1024;
   return L;
 }
@@ -114,6 +119,7 @@ struct rs_lowrank_s {
   void* ar_ctx = nullptr;
   Layout L;
   char* ws;
+  void* ring;
   double *B, *B0, *Bt, *B1, *C, *C1, *part, *G, *Rf, *Linv, *cholw, *Rho, *Rhat, *T, *Q1, *R1, *R2, *Rbar, *gaps;
   int64_t* perm;
   int* info;
@@ -422,14 +428,22 @@ rs_status_t enqueue_sample(rs_lowrank_t h, const double* A, long long lda) {
   RS_CUDA(h, cudaMemsetAsync(h->info, 0, 16, h->st));
   const long long lxn = static_cast<long long>(L.lp) * h->n;
   if (h->m_local > 0) {
-    const int splits = gemm_choose_splits(L.lp, static_cast<int>(h->n), h->m_local, max_splits_for(h, lxn), h->sms);
-    const int ns = gemm_nsplit(h->m_local, splits);
+    int ns = 0;
     {
       Scope sc(h, "gemm_sample", 2.0 * h->ell * static_cast<double>(h->m_local) * h->n);
       View2D Av{A, h->m_local, h->n, lda};
       GemmOutDesc out{h->part, 1, L.lp, lxn, L.lp, static_cast<int>(h->n)};
       PhiloxDesc phx{true, h->seed, 0u, h->row_offset, h->ell};
-      RS_CUDA(h, gemm_kc(h->st, L.lp, static_cast<int>(h->n), h->m_local, Av, Av, phx, out, splits));
+      // Omega generated once per K split into an L2 ring shared by all N tiles; the cluster kernel
+      // (Omega generated in shared memory per pair of N tiles) when the ring does not apply
+      cudaError_t e = gemm_sample_ring(h->st, L.lp, static_cast<int>(h->n), h->m_local, Av, phx, out,
+                                       max_splits_for(h, lxn), h->ring, L.ring_bytes, &ns);
+      if (e == cudaErrorNotSupported) {
+        const int splits = gemm_choose_splits(L.lp, static_cast<int>(h->n), h->m_local, max_splits_for(h, lxn), h->sms);
+        ns = gemm_nsplit(h->m_local, splits);
+        e = gemm_kc(h->st, L.lp, static_cast<int>(h->n), h->m_local, Av, Av, phx, out, splits);
+      }
+      RS_CUDA(h, e);
     }
     {
       Scope sc(h, "reduce", 0.0);
@@ -813,6 +827,7 @@ rs_status_t rs_lowrank_create(rs_lowrank_t* out, int64_t m_global, int64_t m_loc
   auto D = [&](size_t off) { return reinterpret_cast<double*>(base + off); };
   h->B = D(L.off_B);
   h->B0 = D(L.off_B0);
+  h->ring = base + L.off_ring;
   h->Bt = D(L.off_Bt);
   h->B1 = D(L.off_B1);
   h->C = D(L.off_C);
