@@ -23,7 +23,7 @@
 namespace rs {
 
 #ifndef RS_RG_CH
-#define RS_RG_CH 512
+#define RS_RG_CH 256
 #endif
 #ifndef RS_RG_R
 #define RS_RG_R 4
@@ -79,6 +79,7 @@ RS_DEVINL void rg_red_release_add(unsigned int* p, unsigned int v) {
   asm volatile("red.release.gpu.global.add.u32 [%0], %1;" ::"l"(p), "r"(v) : "memory");
 }
 RS_DEVINL void rg_wait_geq(const unsigned int* p, unsigned int target) {
+  // (measured: relaxed polling with exponential back-off made cfg4 0.5 ms slower than this)
   while (rg_ld_acquire(p) < target) __nanosleep(64);
 }
 
