@@ -16,8 +16,6 @@
 #include <cstdio>
 #include <cstdlib>
 
-#include <cooperative_groups.h>
-
 #include "common.cuh"
 #include "internal.h"
 
@@ -53,12 +51,7 @@ RS_DEVINL unsigned int ld_acquire_u32(const unsigned int* p) {
 }
 
 // all NB CTAs: arrive once, wait until `target` arrivals have been counted
-// (-DRS_DEV_QRCP_CGSYNC: cooperative_groups grid sync instead, A/B experiment)
 RS_DEVINL void grid_sync_count(unsigned int* count, unsigned int target) {
-#ifdef RS_DEV_QRCP_CGSYNC
-  (void)count, (void)target;
-  cooperative_groups::this_grid().sync();
-#else
   __syncthreads();
   if (threadIdx.x == 0) {
     asm volatile("red.release.gpu.global.add.u32 [%0], 1;" ::"l"(count) : "memory");
@@ -66,7 +59,6 @@ RS_DEVINL void grid_sync_count(unsigned int* count, unsigned int target) {
     }
   }
   __syncthreads();
-#endif
 }
 
 // (value, index, owner) argmax with ties to the lowest index

@@ -114,8 +114,6 @@ __global__ void __launch_bounds__(RG_THREADS, 1)
       if (lane != 0) return;
       tma_prefetch_desc(&tmA);
       tma_prefetch_desc(&tmW);
-      const uint64_t pol_first = l2_policy_evict_first(), pol_last = l2_policy_evict_last();
-      (void)pol_first, (void)pol_last;
       // per smem slot: the ring chunk its stage came from, to count the chunk consumed once the
       // slot is handed back (the stage's TMA reads of the chunk completed long before)
       int hist_gid[8], hist_slot[8];
@@ -143,14 +141,8 @@ __global__ void __launch_bounds__(RG_THREADS, 1)
           hist_slot[s] = slot;
           hist_last[s] = kin + KT >= RG_CH || it + 1 == x.nk;
           mbar_arrive_expect_tx(&full[s], SM::R_BYTES + SM::L_BYTES_TMA);
-#ifdef RS_DEV_RING_NO_HINTS
           tma_load_2d(sR + s * SM::R_BYTES, &tmA, &full[s], static_cast<int>(k), x.nt * NT);
           tma_load_2d(sL + s * SM::L_BYTES, &tmW, &full[s], kin, (x.gid * RG_R + slot) * MT);
-#else
-          // A streams through L2 once (evict first); the ring chunks are re-read by every member
-          tma_load_2d_hint(sR + s * SM::R_BYTES, &tmA, &full[s], static_cast<int>(k), x.nt * NT, pol_first);
-          tma_load_2d_hint(sL + s * SM::L_BYTES, &tmW, &full[s], kin, (x.gid * RG_R + slot) * MT, pol_last);
-#endif
         }
       }
       // the last stages: their chunks are counted once their data has landed
@@ -165,8 +157,6 @@ __global__ void __launch_bounds__(RG_THREADS, 1)
     const int gt = threadIdx.x - (NCONS + 1) * 32;  // 0 .. 95
     constexpr int GT = RG_GEN_WARPS * 32;
     const int o = static_cast<int>(a.row_offset & 3);
-    const uint64_t pol_keep = l2_policy_evict_last();
-    (void)pol_keep;
     for (int u = blockIdx.x; u < rg.nunits; u += G) {
       const RgUnit x = rg_unit(rg, a.K, u, G);
       for (int c = x.mem; c < x.nch; c += x.gsz) {
@@ -199,13 +189,8 @@ __global__ void __launch_bounds__(RG_THREADS, 1)
             if (kk + 3 >= x.ke) v3 = 0.0;
           }
           double* p = dst + static_cast<size_t>(row) * RG_CH + 4 * q;
-#ifdef RS_DEV_RING_NO_HINTS
           reinterpret_cast<double2*>(p)[0] = make_double2(v0, v1);
           reinterpret_cast<double2*>(p)[1] = make_double2(v2, v3);
-#else
-          st_global_v2_hint(p, v0, v1, pol_keep);  // keep the chunk in L2 until it is re-read
-          st_global_v2_hint(p + 2, v2, v3, pol_keep);
-#endif
         }
         named_bar_sync(1, GT);  // every generator thread's stores precede the release below
         if (gt == 0) {
