@@ -497,19 +497,24 @@ __host__ __device__ constexpr int ct_smem_doubles(int np) {
 // one pivot step k with (k + 1) % 4 == A1 (the tile row that holds row k + 1)
 template <int A1, int TPT, int NTHR>
 RS_DEVINL void chol_tile_step(CholTile<TPT, NTHR>& T, int k, int n, int np, double* Gs, double* Xs, double* s_ri,
-                              int* info, int code) {
+                              int* info, int code, int col0) {
   const int tid = threadIdx.x;
   const int k4 = 4 * (k >> 2);
   const double* Gk = Gs + ct_gofs(k, np) - k4;  // Gk[c] = G(k, c), c >= 4 (k / 4)
   const double* Xk = Xs + ct_xofs(k);           // Xk[c] = acc(k, c), c < 4 (k / 4) + 4
+#ifdef RS_DEV_CHOL_RSQRT_ALL
   double d = Gk[k];
   if (!(d > 0.0)) {
-    if (tid == 0 && info && k < n) atomicCAS(info, 0, code), atomicCAS(info + 1, 0, k + 1);
+    if (tid == 0 && info && k < n) atomicCAS(info, 0, code), atomicCAS(info + 1, 0, col0 + k + 1);
     d = 1.0;
   }
   const double ri = rsqrt(d);
-  const double dinv = ri * ri;
   if (tid == 0) s_ri[k] = ri;
+#else
+  // 1 / sqrt(d_k) was formed once by the thread that published row k (below / at the start)
+  const double ri = s_ri[k];
+#endif
+  const double dinv = ri * ri;
   const int ipub = (k + 1) >> 2;  // tile row block holding row k + 1
   double* Gn = Gs + ct_gofs(k + 1, np) - 4 * ipub;
   double* Xn = Xs + ct_xofs(k + 1);
@@ -534,6 +539,16 @@ RS_DEVINL void chol_tile_step(CholTile<TPT, NTHR>& T, int k, int n, int np, doub
       if (T.kind[s2] == 0) {
         reinterpret_cast<double2*>(&Gn[c])[0] = make_double2(T.v[s2][A1][0], T.v[s2][A1][1]);
         reinterpret_cast<double2*>(&Gn[c])[1] = make_double2(T.v[s2][A1][2], T.v[s2][A1][3]);
+#ifndef RS_DEV_CHOL_RSQRT_ALL
+        if (T.TJ[s2] == ipub) {  // the diagonal tile: d_{k+1} = G(k+1, k+1), checked and inverted once
+          double dn = T.v[s2][A1][A1];
+          if (!(dn > 0.0)) {
+            if (info && k + 1 < n) atomicCAS(info, 0, code), atomicCAS(info + 1, 0, col0 + k + 2);
+            dn = 1.0;
+          }
+          s_ri[k + 1] = rsqrt(dn);
+        }
+#endif
       } else {
         const int lim = k + 1 - c;  // X(k + 1, c + bb) = 0 for c + bb > k + 1
         reinterpret_cast<double2*>(&Xn[c])[0] =
@@ -549,7 +564,7 @@ RS_DEVINL void chol_tile_step(CholTile<TPT, NTHR>& T, int k, int n, int np, doub
 template <int TPT, int NTHR>
 __global__ void __launch_bounds__(NTHR, 1)
     chol_tile_kernel(const double* __restrict__ G, int ldg, int n, double* __restrict__ R, int ldr,
-                     double* __restrict__ Linv, int ldl, int* info, int code, int npad) {
+                     double* __restrict__ Linv, int ldl, int* info, int code, int npad, int col0) {
   extern __shared__ __align__(16) double ct_smem[];
   const int tid = threadIdx.x;
   const int np = (n + 3) / 4 * 4;
@@ -595,12 +610,22 @@ __global__ void __launch_bounds__(NTHR, 1)
   // row 0 of G (identity-padded past n) and of X's accumulators (e_0)
   for (int j = tid; j < np; j += NTHR) Gs[j] = (j < n) ? G[static_cast<long long>(j) * ldg] : (j == 0 ? 1.0 : 0.0);
   if (tid < 4) Xs[tid] = tid == 0 ? 1.0 : 0.0;
+#ifndef RS_DEV_CHOL_RSQRT_ALL
+  if (tid == 0) {
+    double d0 = n > 0 ? G[0] : 1.0;
+    if (!(d0 > 0.0)) {
+      if (info) atomicCAS(info, 0, code), atomicCAS(info + 1, 0, col0 + 1);
+      d0 = 1.0;
+    }
+    s_ri[0] = rsqrt(d0);
+  }
+#endif
   __syncthreads();
   for (int k = 0; k < np; k += 4) {  // np is a multiple of 4
-    chol_tile_step<1>(T, k, n, np, Gs, Xs, s_ri, info, code);
-    chol_tile_step<2>(T, k + 1, n, np, Gs, Xs, s_ri, info, code);
-    chol_tile_step<3>(T, k + 2, n, np, Gs, Xs, s_ri, info, code);
-    chol_tile_step<0>(T, k + 3, n, np, Gs, Xs, s_ri, info, code);
+    chol_tile_step<1>(T, k, n, np, Gs, Xs, s_ri, info, code, col0);
+    chol_tile_step<2>(T, k + 1, n, np, Gs, Xs, s_ri, info, code, col0);
+    chol_tile_step<3>(T, k + 2, n, np, Gs, Xs, s_ri, info, code, col0);
+    chol_tile_step<0>(T, k + 3, n, np, Gs, Xs, s_ri, info, code, col0);
   }
   // R(k, t) = G(k, t) / sqrt(d_k) (t >= k), Linv(k, t) = acc(k, t) / sqrt(d_k) (t <= k), zero
   // elsewhere and in the padding; consecutive threads take consecutive rows (column-major)
@@ -617,10 +642,51 @@ __global__ void __launch_bounds__(NTHR, 1)
   }
 }
 
+cudaError_t chol_inv_at(cudaStream_t st, const double* G, int ldg, int n, int npad, double* R, int ldr, double* Linv,
+                        int ldl, double* gwork, int* info, int info_code, int col0);
+
+// 128 < n <= 256: 2 x 2 blocks on the register-tile kernel.  G = R^T R with R = [R11 R12; 0 R22]:
+// R11 = chol(G11), R12 = R11^{-T} G12 = L11^{-1} G12, R22 = chol(G22 - R12^T R12), and
+// L^{-1} = R^{-T} = [L11^{-1} 0; -L22^{-1} R12^T L11^{-1}  L22^{-1}] -- two one-CTA factorisations and
+// four small GEMMs instead of the 8-CTA cluster kernel's one barrier per pivot (cfg3's l = 220).
+static cudaError_t chol_inv_2x2(cudaStream_t st, const double* G, int ldg, int n, int npad, double* R, int ldr,
+                                double* Linv, int ldl, double* gwork, int* info, int info_code, int col0) {
+  const int n1 = 16 * ((n + 31) / 32), n2 = n - n1;
+  double* S = gwork;                                   // n2 x n2: G22 - R12^T R12
+  double* Tm = gwork + static_cast<size_t>(n2) * n2;   // n2 x n1: R12^T L11^{-1}
+  cudaError_t e = cudaMemset2DAsync(R, static_cast<size_t>(ldr) * 8, 0, static_cast<size_t>(npad) * 8, npad, st);
+  if (e == cudaSuccess)
+    e = cudaMemset2DAsync(Linv, static_cast<size_t>(ldl) * 8, 0, static_cast<size_t>(npad) * 8, npad, st);
+  if (e == cudaSuccess) e = chol_inv_at(st, G, ldg, n1, n1, R, ldr, Linv, ldl, nullptr, info, info_code, col0);
+  double* R12 = R + static_cast<long long>(n1) * ldr;
+  if (e == cudaSuccess)  // R12 = L11^{-1} G12
+    e = small_gemm(st, n1, n2, n1, Linv, 1, ldl, G + static_cast<long long>(n1) * ldg, 1, ldg, R12, 1, ldr, false);
+  if (e == cudaSuccess) e = copy_2d(st, G + n1 + static_cast<long long>(n1) * ldg, ldg, S, n2, n2, n2);
+  if (e == cudaSuccess)  // S = G22 - R12^T R12 (full, both triangles)
+    e = small_gemm(st, n2, n2, n1, R12, ldr, 1, R12, 1, ldr, S, 1, n2, true, -1.0);
+  double* R22 = R + n1 + static_cast<long long>(n1) * ldr;
+  double* L22 = Linv + n1 + static_cast<long long>(n1) * ldl;
+  if (e == cudaSuccess) e = chol_inv_at(st, S, n2, n2, n2, R22, ldr, L22, ldl, nullptr, info, info_code, col0 + n1);
+  if (e == cudaSuccess)  // T = R12^T L11^{-1}
+    e = small_gemm(st, n2, n1, n1, R12, ldr, 1, Linv, 1, ldl, Tm, 1, n2, false);
+  if (e == cudaSuccess)  // L21^{-1} block = -L22^{-1} T
+    e = small_gemm(st, n2, n1, n2, L22, 1, ldl, Tm, 1, n2, Linv + n1, 1, ldl, false, -1.0);
+  return e;
+}
+
 cudaError_t chol_inv(cudaStream_t st, const double* G, int ldg, int n, int npad, double* R, int ldr, double* Linv,
                      int ldl, double* gwork, int* info, int info_code) {
+  return chol_inv_at(st, G, ldg, n, npad, R, ldr, Linv, ldl, gwork, info, info_code, 0);
+}
+
+cudaError_t chol_inv_at(cudaStream_t st, const double* G, int ldg, int n, int npad, double* R, int ldr, double* Linv,
+                        int ldl, double* gwork, int* info, int info_code, int col0) {
   if (n <= 0) return cudaSuccess;
   if (n > 512) return cudaErrorInvalidValue;
+#ifndef RS_DEV_CHOL_CLUSTER_256
+  if (n > CT_MAXN && n <= 2 * CT_MAXN && gwork)
+    return chol_inv_2x2(st, G, ldg, n, npad, R, ldr, Linv, ldl, gwork, info, info_code, col0);
+#endif
   // compile-time development switches: -DRS_DEV_CHOL_SMEM_MAX_N=<n> (crossover experiments),
   // -DRS_DEV_CHOL_BLOCKED (the blocked kernel for n <= 128), -DRS_DEV_CHOL_TPT=2 (two tiles per thread)
 #ifdef RS_DEV_CHOL_SMEM_MAX_N
@@ -651,15 +717,15 @@ cudaError_t chol_inv(cudaStream_t st, const double* G, int ldg, int n, int npad,
     // still take part in every pivot's barrier
     const int tiles = nt * (nt + 1);
     if (tpt == 1 && tiles <= 256)  // n <= 60 (adaptive blocks, Fig. 7's k = 54)
-      chol_tile_kernel<1, 256><<<1, 256, ct_smem, st>>>(G, ldg, n, R, ldr, Linv, ldl, info, info_code, npad);
+      chol_tile_kernel<1, 256><<<1, 256, ct_smem, st>>>(G, ldg, n, R, ldr, Linv, ldl, info, info_code, npad, col0);
     else if (tpt == 1 && tiles <= 512)  // n <= 88 (l = 64)
-      chol_tile_kernel<1, 512><<<1, 512, ct_smem, st>>>(G, ldg, n, R, ldr, Linv, ldl, info, info_code, npad);
+      chol_tile_kernel<1, 512><<<1, 512, ct_smem, st>>>(G, ldg, n, R, ldr, Linv, ldl, info, info_code, npad, col0);
     else if (tpt == 1 && tiles <= 832)  // n <= 112 (l = 110: 72 registers per thread instead of 64)
-      chol_tile_kernel<1, 832><<<1, 832, ct_smem, st>>>(G, ldg, n, R, ldr, Linv, ldl, info, info_code, npad);
+      chol_tile_kernel<1, 832><<<1, 832, ct_smem, st>>>(G, ldg, n, R, ldr, Linv, ldl, info, info_code, npad, col0);
     else if (tpt == 1 && tiles <= 1024)  // n <= 124
-      chol_tile_kernel<1, 1024><<<1, 1024, ct_smem, st>>>(G, ldg, n, R, ldr, Linv, ldl, info, info_code, npad);
+      chol_tile_kernel<1, 1024><<<1, 1024, ct_smem, st>>>(G, ldg, n, R, ldr, Linv, ldl, info, info_code, npad, col0);
     else
-      chol_tile_kernel<2, 576><<<1, 576, ct_smem, st>>>(G, ldg, n, R, ldr, Linv, ldl, info, info_code, npad);
+      chol_tile_kernel<2, 576><<<1, 576, ct_smem, st>>>(G, ldg, n, R, ldr, Linv, ldl, info, info_code, npad, col0);
   } else if (n <= smem_max_n && n <= CH_SMEM_MAX_N) {
     const int np = (n + CB - 1) / CB * CB;
     const size_t smem = static_cast<size_t>(np) * (np + 1) * 8;
