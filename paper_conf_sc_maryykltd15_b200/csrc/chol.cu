@@ -502,18 +502,8 @@ RS_DEVINL void chol_tile_step(CholTile<TPT, NTHR>& T, int k, int n, int np, doub
   const int k4 = 4 * (k >> 2);
   const double* Gk = Gs + ct_gofs(k, np) - k4;  // Gk[c] = G(k, c), c >= 4 (k / 4)
   const double* Xk = Xs + ct_xofs(k);           // Xk[c] = acc(k, c), c < 4 (k / 4) + 4
-#ifdef RS_DEV_CHOL_RSQRT_ALL
-  double d = Gk[k];
-  if (!(d > 0.0)) {
-    if (tid == 0 && info && k < n) atomicCAS(info, 0, code), atomicCAS(info + 1, 0, col0 + k + 1);
-    d = 1.0;
-  }
-  const double ri = rsqrt(d);
-  if (tid == 0) s_ri[k] = ri;
-#else
   // 1 / sqrt(d_k) was formed once by the thread that published row k (below / at the start)
   const double ri = s_ri[k];
-#endif
   const double dinv = ri * ri;
   const int ipub = (k + 1) >> 2;  // tile row block holding row k + 1
   double* Gn = Gs + ct_gofs(k + 1, np) - 4 * ipub;
@@ -539,7 +529,6 @@ RS_DEVINL void chol_tile_step(CholTile<TPT, NTHR>& T, int k, int n, int np, doub
       if (T.kind[s2] == 0) {
         reinterpret_cast<double2*>(&Gn[c])[0] = make_double2(T.v[s2][A1][0], T.v[s2][A1][1]);
         reinterpret_cast<double2*>(&Gn[c])[1] = make_double2(T.v[s2][A1][2], T.v[s2][A1][3]);
-#ifndef RS_DEV_CHOL_RSQRT_ALL
         if (T.TJ[s2] == ipub) {  // the diagonal tile: d_{k+1} = G(k+1, k+1), checked and inverted once
           double dn = T.v[s2][A1][A1];
           if (!(dn > 0.0)) {
@@ -548,7 +537,6 @@ RS_DEVINL void chol_tile_step(CholTile<TPT, NTHR>& T, int k, int n, int np, doub
           }
           s_ri[k + 1] = rsqrt(dn);
         }
-#endif
       } else {
         const int lim = k + 1 - c;  // X(k + 1, c + bb) = 0 for c + bb > k + 1
         reinterpret_cast<double2*>(&Xn[c])[0] =
@@ -610,7 +598,6 @@ __global__ void __launch_bounds__(NTHR, 1)
   // row 0 of G (identity-padded past n) and of X's accumulators (e_0)
   for (int j = tid; j < np; j += NTHR) Gs[j] = (j < n) ? G[static_cast<long long>(j) * ldg] : (j == 0 ? 1.0 : 0.0);
   if (tid < 4) Xs[tid] = tid == 0 ? 1.0 : 0.0;
-#ifndef RS_DEV_CHOL_RSQRT_ALL
   if (tid == 0) {
     double d0 = n > 0 ? G[0] : 1.0;
     if (!(d0 > 0.0)) {
@@ -619,7 +606,6 @@ __global__ void __launch_bounds__(NTHR, 1)
     }
     s_ri[0] = rsqrt(d0);
   }
-#endif
   __syncthreads();
   for (int k = 0; k < np; k += 4) {  // np is a multiple of 4
     chol_tile_step<1>(T, k, n, np, Gs, Xs, s_ri, info, code, col0);

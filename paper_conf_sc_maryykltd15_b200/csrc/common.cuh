@@ -140,6 +140,13 @@ RS_DEVINL void tma_load_3d(void* smem_dst, const CUtensorMap* m, uint64_t* bar, 
 // ranks' kernels overlapping on one GPU.  Here the arrive sits in the basic block
 // after the next stage's wait, so all of stage it - 1's DMMAs -- which consume every one of its
 // loads -- have issued before it.
+// Alternative (-DRS_RELEASE_FENCE, A/B experiment): release the slot at the end of its own stage,
+// after a CTA-scope fence that makes the warp wait for its outstanding shared-memory loads.
+RS_DEVINL void ring_release_fenced(uint64_t* empty, int s, int lane) {
+  asm volatile("fence.acq_rel.cta;" ::: "memory");
+  __syncwarp();
+  if (lane == 0) mbar_arrive(&empty[s]);
+}
 RS_DEVINL void ring_release_prev(uint64_t* empty, int it, int ns, int lane) {
   if (it > 0) {
     __syncwarp();

@@ -206,7 +206,9 @@ __global__ void __launch_bounds__(GEMM_THREADS, 1)
   for (int it = 0; it < nk; ++it) {
     const int s = it % SM::NS;
     mbar_wait(&full[s], (it / SM::NS) & 1);
+#ifndef RS_RELEASE_FENCE
     ring_release_prev(empty, it, SM::NS, lane);
+#endif
     // refill the slot of stage it - 1 (waits until every warp has released it)
     if (threadIdx.x == 0 && it + SM::NS - 1 < nk) issue(it + SM::NS - 1);
     const unsigned char* Ls = sL + s * SM::L_BYTES;
@@ -214,6 +216,9 @@ __global__ void __launch_bounds__(GEMM_THREADS, 1)
     kc_stage_mma<MFW>(
         acc, [&](int mf, int p) { return *reinterpret_cast<const double2*>(Ls + kc_pair_off(rowL(mf), p, kk)); },
         [&](int nf, int p) { return *reinterpret_cast<const double2*>(Rs + kc_pair_off(rowR(nf), p, kk)); });
+#ifdef RS_RELEASE_FENCE
+    ring_release_fenced(empty, s, lane);
+#endif
   }
   kc_store<MFW>(acc, a.out, m0, n0, wn, kk, rowL);
 }
@@ -287,12 +292,17 @@ __global__ void __launch_bounds__(KCP_THREADS, 1)
   for (int it = 0; it < nk; ++it) {
     const int s = it % SM::NS;
     mbar_wait(&full[s], (it / SM::NS) & 1);
+#ifndef RS_RELEASE_FENCE
     ring_release_prev(empty, it, SM::NS, lane);
+#endif
     const unsigned char* Ls = sL + s * SM::L_BYTES;
     const unsigned char* Rs = sR + s * SM::R_BYTES;
     kc_stage_mma<MFW>(
         acc, [&](int mf, int p) { return *reinterpret_cast<const double2*>(Ls + kc_pair_off(rowL(mf), p, kk)); },
         [&](int nf, int p) { return *reinterpret_cast<const double2*>(Rs + kc_pair_off(rowR(nf), p, kk)); });
+#ifdef RS_RELEASE_FENCE
+    ring_release_fenced(empty, s, lane);
+#endif
   }
   kc_store<MFW>(acc, a.out, m0, n0, wn, kk, rowL);
 }
@@ -776,7 +786,9 @@ __global__ void __launch_bounds__(KCP_THREADS, 1)
   for (int it = 0; it < nk; ++it) {
     const int s = it % MC_NS;
     mbar_wait(&full[s], (it / MC_NS) & 1);
+#ifndef RS_RELEASE_FENCE
     ring_release_prev(empty, it, MC_NS, lane);
+#endif
     const long long kc = kb + static_cast<long long>(it) * KT;  // first K of the stage
     const unsigned char* Ls = sL + s * SM::L_BYTES;
     const unsigned char* Rs = sR + s * SM::R_BYTES;
@@ -785,6 +797,9 @@ __global__ void __launch_bounds__(KCP_THREADS, 1)
       mc_stage<NFR, 0, NB, TRI>(acc, Ls, Rs, nbox0, r, kk, kc, m0, n0);
     else
       mc_stage<NFR, NFR, NB, TRI>(acc, Ls, Rs, nbox0, r, kk, kc, m0, n0);
+#ifdef RS_RELEASE_FENCE
+    ring_release_fenced(empty, s, lane);
+#endif
   }
 
   // ---- epilogue: stage the MT x NT tile in shared memory, then coalesced 16-byte stores ----
