@@ -140,8 +140,10 @@ RS_DEVINL void tma_load_3d(void* smem_dst, const CUtensorMap* m, uint64_t* bar, 
 // ranks' kernels overlapping on one GPU.  Here the arrive sits in the basic block
 // after the next stage's wait, so all of stage it - 1's DMMAs -- which consume every one of its
 // loads -- have issued before it.
-// Alternative (-DRS_RELEASE_FENCE, A/B experiment): release the slot at the end of its own stage,
-// after a CTA-scope fence that makes the warp wait for its outstanding shared-memory loads.
+// The other safe form: release the slot at the end of its own stage, behind a CTA-scope fence
+// (MEMBAR.CTA) that makes the warp wait for its outstanding shared-memory loads; ptxas keeps the
+// stage's LDS before the fence.  Used by the dense MC GEMM (faster there), -DRS_RELEASE_FENCE for
+// the KC kernels (measured equal).
 RS_DEVINL void ring_release_fenced(uint64_t* empty, int s, int lane) {
   asm volatile("fence.acq_rel.cta;" ::: "memory");
   __syncwarp();

@@ -786,7 +786,7 @@ __global__ void __launch_bounds__(KCP_THREADS, 1)
   for (int it = 0; it < nk; ++it) {
     const int s = it % MC_NS;
     mbar_wait(&full[s], (it / MC_NS) & 1);
-#ifndef RS_RELEASE_FENCE
+#ifdef RS_MC_RELEASE_DEFERRED
     ring_release_prev(empty, it, MC_NS, lane);
 #endif
     const long long kc = kb + static_cast<long long>(it) * KT;  // first K of the stage
@@ -797,7 +797,9 @@ __global__ void __launch_bounds__(KCP_THREADS, 1)
       mc_stage<NFR, 0, NB, TRI>(acc, Ls, Rs, nbox0, r, kk, kc, m0, n0);
     else
       mc_stage<NFR, NFR, NB, TRI>(acc, Ls, Rs, nbox0, r, kk, kc, m0, n0);
-#ifdef RS_RELEASE_FENCE
+#ifndef RS_MC_RELEASE_DEFERRED
+    // released at the end of its own stage behind a CTA fence (measured at cfg4: 30.83 ms against
+    // 31.72 ms with the one-stage-deferred release on the same box; both pass the overlap stress)
     ring_release_fenced(empty, s, lane);
 #endif
   }
@@ -1194,9 +1196,16 @@ RS_DEVINL void syrk_warp(const unsigned char* sX, uint64_t* full, uint64_t* empt
     // no blocks: still release every slot so the producer can refill it
     for (int it = 0; it < nk; ++it) {
       const int s = it % SYRK_NS;
+#ifdef RS_RELEASE_FENCE_ALL
+      if (threadIdx.x == 0 && it + SYRK_NS - 1 < nk) issue(it + SYRK_NS - 1);
+#endif
       mbar_wait(&full[s], (it / SYRK_NS) & 1);
+#ifndef RS_RELEASE_FENCE_ALL
       ring_release_prev(empty, it, SYRK_NS, lane);
       if (threadIdx.x == 0 && it + SYRK_NS - 1 < nk) issue(it + SYRK_NS - 1);
+#else
+      ring_release_fenced(empty, s, lane);
+#endif
     }
     return;
   } else {
@@ -1210,9 +1219,14 @@ RS_DEVINL void syrk_warp(const unsigned char* sX, uint64_t* full, uint64_t* empt
         for (int f2 = 0; f2 < 2; ++f2) acc[b][f][f2][0] = acc[b][f][f2][1] = 0.0;
     for (int it = 0; it < nk; ++it) {
       const int s = it % SYRK_NS;
+#ifdef RS_RELEASE_FENCE_ALL
+      if (threadIdx.x == 0 && it + SYRK_NS - 1 < nk) issue(it + SYRK_NS - 1);  // slot of it - 1, released
+#endif
       mbar_wait(&full[s], (it / SYRK_NS) & 1);
+#ifndef RS_RELEASE_FENCE_ALL
       ring_release_prev(empty, it, SYRK_NS, lane);
       if (threadIdx.x == 0 && it + SYRK_NS - 1 < nk) issue(it + SYRK_NS - 1);
+#endif
       const unsigned char* Xs = sX + s * SyrkSmem<R>::X_BYTES;
 #pragma unroll
       for (int p = 0; p < 2; ++p) {
@@ -1237,6 +1251,9 @@ RS_DEVINL void syrk_warp(const unsigned char* sX, uint64_t* full, uint64_t* empt
             }
         }
       }
+#ifdef RS_RELEASE_FENCE_ALL
+      ring_release_fenced(empty, s, lane);
+#endif
     }
     // G[kc_row(I, f, r)][kc_row(J, f2, 2kk + e)] and its mirror
 #pragma unroll
@@ -1394,7 +1411,9 @@ __global__ void __launch_bounds__(TSA_THREADS, 1)
     for (int s = 0; s < NB; ++s, ++g) {
       const int slot = g % TSA_NS;
       mbar_wait(&full[slot], (g / TSA_NS) & 1);
+#ifndef RS_RELEASE_FENCE_ALL
       ring_release_prev(empty, g, TSA_NS, lane);
+#endif
       const unsigned char* Xs = sX + slot * SM::STAGE + warp * 2048;
       const unsigned char* Us = sU + s * SM::UST;
 #pragma unroll
@@ -1411,6 +1430,9 @@ __global__ void __launch_bounds__(TSA_THREADS, 1)
           dmma_8x8x4(acc[1][nb][1][0], acc[1][nb][1][1], a2.y, b2.y);
         }
       }
+#ifdef RS_RELEASE_FENCE_ALL
+      ring_release_fenced(empty, slot, lane);
+#endif
     }
     // Y[row, col]: rows 2r (f = 0) and 2r + 1 (f = 1) of the warp's 16, col 16 nb + 2 (2 kk + e) + f2
     const long long row = static_cast<long long>(m0) + 16 * warp + 2 * r;
