@@ -1196,11 +1196,11 @@ RS_DEVINL void syrk_warp(const unsigned char* sX, uint64_t* full, uint64_t* empt
     // no blocks: still release every slot so the producer can refill it
     for (int it = 0; it < nk; ++it) {
       const int s = it % SYRK_NS;
-#ifdef RS_RELEASE_FENCE_ALL
+#ifndef RS_SYRK_RELEASE_DEFERRED
       if (threadIdx.x == 0 && it + SYRK_NS - 1 < nk) issue(it + SYRK_NS - 1);
 #endif
       mbar_wait(&full[s], (it / SYRK_NS) & 1);
-#ifndef RS_RELEASE_FENCE_ALL
+#ifdef RS_SYRK_RELEASE_DEFERRED
       ring_release_prev(empty, it, SYRK_NS, lane);
       if (threadIdx.x == 0 && it + SYRK_NS - 1 < nk) issue(it + SYRK_NS - 1);
 #else
@@ -1219,11 +1219,11 @@ RS_DEVINL void syrk_warp(const unsigned char* sX, uint64_t* full, uint64_t* empt
         for (int f2 = 0; f2 < 2; ++f2) acc[b][f][f2][0] = acc[b][f][f2][1] = 0.0;
     for (int it = 0; it < nk; ++it) {
       const int s = it % SYRK_NS;
-#ifdef RS_RELEASE_FENCE_ALL
+#ifndef RS_SYRK_RELEASE_DEFERRED
       if (threadIdx.x == 0 && it + SYRK_NS - 1 < nk) issue(it + SYRK_NS - 1);  // slot of it - 1, released
 #endif
       mbar_wait(&full[s], (it / SYRK_NS) & 1);
-#ifndef RS_RELEASE_FENCE_ALL
+#ifdef RS_SYRK_RELEASE_DEFERRED
       ring_release_prev(empty, it, SYRK_NS, lane);
       if (threadIdx.x == 0 && it + SYRK_NS - 1 < nk) issue(it + SYRK_NS - 1);
 #endif
@@ -1251,7 +1251,7 @@ RS_DEVINL void syrk_warp(const unsigned char* sX, uint64_t* full, uint64_t* empt
             }
         }
       }
-#ifdef RS_RELEASE_FENCE_ALL
+#ifndef RS_SYRK_RELEASE_DEFERRED
       ring_release_fenced(empty, s, lane);
 #endif
     }

@@ -225,7 +225,7 @@ __global__ void __launch_bounds__(RG_THREADS, 1)
     for (int it = 0; it < x.nk; ++it, ++g) {
       const int s = g % SM::NS;
       mbar_wait(&full[s], (g / SM::NS) & 1);
-#ifndef RS_RELEASE_FENCE_ALL
+#ifdef RS_RING_RELEASE_DEFERRED
       ring_release_prev(empty, g, SM::NS, lane);
 #endif
       const unsigned char* Ls = sL + s * SM::L_BYTES;
@@ -233,8 +233,8 @@ __global__ void __launch_bounds__(RG_THREADS, 1)
       kc_stage_mma<MFW>(
           acc, [&](int mf, int p) { return *reinterpret_cast<const double2*>(Ls + kc_pair_off(rowL(mf), p, kk)); },
           [&](int nf, int p) { return *reinterpret_cast<const double2*>(Rs + kc_pair_off(rowR(nf), p, kk)); });
-#ifdef RS_RELEASE_FENCE_ALL
-      ring_release_fenced(empty, s, lane);
+#ifndef RS_RING_RELEASE_DEFERRED
+      ring_release_fenced(empty, s, lane);  // measured 32.53 vs 32.68 ms (deferred) at cfg4
 #endif
     }
     GemmOut o = a.out;
