@@ -82,11 +82,14 @@ def test_sample_parity(m, n, k, p):
     assert rel(B, Bo) <= 1e-13
 
 
-def test_sample_row_offset_partition_sums_to_whole():
-    """Two row blocks (offset not a multiple of 4) computed by two handles sum to the 1-rank B."""
-    m, n, k, p = 3001, 257, 16, 8
+@pytest.mark.parametrize("m,split", [(3001, 1499), (10001, 4999)])
+def test_sample_row_offset_partition_sums_to_whole(m, split):
+    """Two row blocks (offset not a multiple of 4) computed by two handles sum to the 1-rank B --
+    on the cluster sample kernel (m_local < 2048) and on the ring sample kernel (m_local >= 2048,
+    Philox blocks straddling the chunk and rank boundaries)."""
+    n, k, p = 257, 16, 8
     A, _ = make_matrix(m, n, "exp-k", k, seed=7)
-    parts = [(0, 1499), (1499, m)]
+    parts = [(0, split), (split, m)]
     Bs = []
     for r0, r1 in parts:
         h = rs.create(m, r1 - r0, r0, n, k, p, SEED)
@@ -97,7 +100,7 @@ def test_sample_row_offset_partition_sums_to_whole():
             rs.destroy(h)
     Bo = OPL.sample(A, k + p, SEED)
     assert rel(Bs[0] + Bs[1], Bo) <= 1e-13
-    assert rel(Bs[0], OPL.sample(np.asfortranarray(A[:1499]), k + p, SEED)) <= 1e-13
+    assert rel(Bs[0], OPL.sample(np.asfortranarray(A[:split]), k + p, SEED)) <= 1e-13
 
 
 @pytest.mark.parametrize("m,n,k,p", [(3001, 257, 16, 8), (20000, 1000, 100, 10), (500, 64, 5, 3)])
