@@ -1398,6 +1398,8 @@ __global__ void __launch_bounds__(TSA_THREADS, 1)
   mbar_wait(resb, 0);
   const int r = lane >> 2, kk = lane & 3;
   int g = 0;
+  int slot = 0;          // g % TSA_NS, kept incrementally (TSA_NS is not a power of two)
+  uint32_t par = 0;      // (g / TSA_NS) & 1
   for (int i = 0; i < mytiles; ++i) {
     const int m0 = (blockIdx.x + i * gridDim.x) * 128;
     double acc[2][NB][2][2];
@@ -1409,10 +1411,12 @@ __global__ void __launch_bounds__(TSA_THREADS, 1)
         for (int f2 = 0; f2 < 2; ++f2) acc[f][nb][f2][0] = acc[f][nb][f2][1] = 0.0;
 #pragma unroll
     for (int s = 0; s < NB; ++s, ++g) {
-      const int slot = g % TSA_NS;
-      mbar_wait(&full[slot], (g / TSA_NS) & 1);
+      mbar_wait(&full[slot], par);
 #ifndef RS_RELEASE_FENCE_ALL
-      ring_release_prev(empty, g, TSA_NS, lane);
+      if (g > 0) {  // ring_release_prev with the incrementally kept slot
+        __syncwarp();
+        if (lane == 0) mbar_arrive(&empty[slot == 0 ? TSA_NS - 1 : slot - 1]);
+      }
 #endif
       const unsigned char* Xs = sX + slot * SM::STAGE + warp * 2048;
       const unsigned char* Us = sU + s * SM::UST;
@@ -1420,19 +1424,26 @@ __global__ void __launch_bounds__(TSA_THREADS, 1)
       for (int ks = 0; ks < KT / 4; ++ks) {
         const uint32_t krow = 8 * (ks >> 1) + 2 * kk + (ks & 1);
         const uint32_t off = krow * 128u + (((static_cast<uint32_t>(r) ^ krow) & 7u) << 4);
+        // every load of the k-step first, then its DMMAs
+        double2 b2[NB];
+#pragma unroll
+        for (int nb = s; nb < NB; ++nb) b2[nb] = *reinterpret_cast<const double2*>(Us + nb * 2048 + off);
         const double2 a2 = *reinterpret_cast<const double2*>(Xs + off);
 #pragma unroll
         for (int nb = s; nb < NB; ++nb) {
-          const double2 b2 = *reinterpret_cast<const double2*>(Us + nb * 2048 + off);
-          dmma_8x8x4(acc[0][nb][0][0], acc[0][nb][0][1], a2.x, b2.x);
-          dmma_8x8x4(acc[0][nb][1][0], acc[0][nb][1][1], a2.x, b2.y);
-          dmma_8x8x4(acc[1][nb][0][0], acc[1][nb][0][1], a2.y, b2.x);
-          dmma_8x8x4(acc[1][nb][1][0], acc[1][nb][1][1], a2.y, b2.y);
+          dmma_8x8x4(acc[0][nb][0][0], acc[0][nb][0][1], a2.x, b2[nb].x);
+          dmma_8x8x4(acc[0][nb][1][0], acc[0][nb][1][1], a2.x, b2[nb].y);
+          dmma_8x8x4(acc[1][nb][0][0], acc[1][nb][0][1], a2.y, b2[nb].x);
+          dmma_8x8x4(acc[1][nb][1][0], acc[1][nb][1][1], a2.y, b2[nb].y);
         }
       }
 #ifdef RS_RELEASE_FENCE_ALL
       ring_release_fenced(empty, slot, lane);
 #endif
+      if (++slot == TSA_NS) {
+        slot = 0;
+        par ^= 1u;
+      }
     }
     // Y[row, col]: rows 2r (f = 0) and 2r + 1 (f = 1) of the warp's 16, col 16 nb + 2 (2 kk + e) + f2
     const long long row = static_cast<long long>(m0) + 16 * warp + 2 * r;
