@@ -82,17 +82,6 @@ RS_DEVINL void rg_wait_geq(const unsigned int* p, unsigned int target) {
   // (measured: relaxed polling with exponential back-off made cfg4 0.5 ms slower than this)
   while (rg_ld_acquire(p) < target) __nanosleep(64);
 }
-RS_DEVINL unsigned int rg_ld_relaxed(const unsigned int* p) {
-  unsigned int v;
-  asm volatile("ld.relaxed.gpu.global.u32 %0, [%1];" : "=r"(v) : "l"(p) : "memory");
-  return v;
-}
-// The generators' slot wait: relaxed polls (an acquire load also invalidates the SM's L1 --
-// CCTL.IVALL -- on every try, next to the MMA warps' shared-memory traffic), one acquire at the end.
-RS_DEVINL void rg_wait_geq_relaxed(const unsigned int* p, unsigned int target) {
-  while (rg_ld_relaxed(p) < target) __nanosleep(128);
-  (void)rg_ld_acquire(p);
-}
 
 template <int MFW>
 __global__ void __launch_bounds__(RG_THREADS, 1)
@@ -173,11 +162,7 @@ __global__ void __launch_bounds__(RG_THREADS, 1)
       for (int c = x.mem; c < x.nch; c += x.gsz) {
         const int slot = c % RG_R;
         unsigned int* cons = rg.consumed + x.gid * RG_R + slot;
-        #ifdef RS_DEV_RING_ACQ_POLL
         if (gt == 0 && c >= RG_R) rg_wait_geq(cons, static_cast<unsigned int>(x.gsz * (c / RG_R)));
-#else
-        if (gt == 0 && c >= RG_R) rg_wait_geq_relaxed(cons, static_cast<unsigned int>(x.gsz * (c / RG_R)));
-#endif
         named_bar_sync(1, GT);
         double* dst = rg.ring + static_cast<size_t>(x.gid * RG_R + slot) * MT * RG_CH;
         const long long kc0 = x.kb + static_cast<long long>(c) * RG_CH;  // first K row of the chunk

@@ -82,6 +82,32 @@ def test_sample_parity(m, n, k, p):
     assert rel(B, Bo) <= 1e-13
 
 
+@pytest.mark.parametrize("m,n,k,p", [
+    (40000, 130, 8, 4),      # l = 12 (one 16-row M tile), 2 N tiles: groups of 2 members
+    (30000, 300, 100, 28),   # l = 128 (MFW = 8), 3 N tiles
+    (2048, 700, 20, 10),     # m_local at the ring threshold (8 chunks of 256 rows)
+    (1000003, 129, 30, 2),   # m = 1e6 + 3 rows (A's tail inside the last chunk), 2 N tiles (129 = 128 + 1)
+])
+def test_sample_ring_shapes(m, n, k, p):
+    """The ring sample GEMM (m_local >= 2048, l <= 128) at its edges: tiny and full M tiles, a
+    ragged last N tile, the smallest K it takes, and a K tail inside a chunk -- B = Omega A
+    against the oracle's fixed-order product."""
+    rng = np.random.default_rng(m + n)
+    A = np.asfortranarray(rng.standard_normal((m, n)))
+    B = _sample_gpu(A, k, p)
+    assert rel(B, OPL.sample(A, k + p, SEED)) <= 1e-13
+
+
+def _sample_gpu(A, k, p):
+    m, n = A.shape
+    h = rs.create(m, m, 0, n, k, p, SEED)
+    try:
+        rs.sample(h, to_dev(A))
+        return to_np(rs.get_sample(h))
+    finally:
+        rs.destroy(h)
+
+
 @pytest.mark.parametrize("m,split", [(3001, 1499), (10001, 4999)])
 def test_sample_row_offset_partition_sums_to_whole(m, split):
     """Two row blocks (offset not a multiple of 4) computed by two handles sum to the 1-rank B --
