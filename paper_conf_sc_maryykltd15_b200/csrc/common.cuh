@@ -27,6 +27,9 @@ RS_DEVINL void mbar_arrive_expect_tx(uint64_t* bar, uint32_t bytes) {
 RS_DEVINL void mbar_arrive(uint64_t* bar) {
   asm volatile("mbarrier.arrive.shared::cta.b64 _, [%0];" ::"r"(smem_u32(bar)) : "memory");
 }
+RS_DEVINL void mbar_arrive_cnt(uint64_t* bar, uint32_t count) {
+  asm volatile("mbarrier.arrive.shared::cta.b64 _, [%0], %1;" ::"r"(smem_u32(bar)), "r"(count) : "memory");
+}
 RS_DEVINL void mbar_wait(uint64_t* bar, uint32_t parity) {
   asm volatile(
       "{\n"

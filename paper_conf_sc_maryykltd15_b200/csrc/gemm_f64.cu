@@ -78,6 +78,21 @@ bool make_tmap3(CUtensorMap* m, const View2D& v, uint32_t nbx) {
 }
 
 template <int MFW>
+cudaError_t launch_kc_tail_t(cudaStream_t st, dim3 grid, const CUtensorMap& tR, const CUtensorMap& tL,
+                             const CUtensorMap& tT, const GemmArgs& a) {
+  if constexpr (MFW >= 4) {
+    constexpr int smem = KCSmem<MFW, false, true>::TOTAL;
+    cudaError_t e = ensure_smem(kc_gemm_pwg_kernel<MFW, true>, smem);
+    if (e != cudaSuccess) return e;
+    kc_gemm_pwg_kernel<MFW, true><<<grid, KCP_THREADS, smem, st>>>(tR, tL, tT, a);
+    count_launch();
+    return cudaGetLastError();
+  } else {
+    return cudaErrorNotSupported;
+  }
+}
+
+template <int MFW>
 cudaError_t launch_kc_t(cudaStream_t st, dim3 grid, const CUtensorMap& tR, const CUtensorMap& tL, const GemmArgs& a) {
   constexpr int smem = KCSmem<MFW, false>::TOTAL;
   // producer warpgroup (default): with the producer sleeping in the slot wait (mbar_wait_sleep) the
@@ -87,7 +102,7 @@ cudaError_t launch_kc_t(cudaStream_t st, dim3 grid, const CUtensorMap& tR, const
   {
     cudaError_t e = ensure_smem(kc_gemm_pwg_kernel<MFW>, smem);
     if (e != cudaSuccess) return e;
-    kc_gemm_pwg_kernel<MFW><<<grid, KCP_THREADS, smem, st>>>(tR, tL, a);
+    kc_gemm_pwg_kernel<MFW><<<grid, KCP_THREADS, smem, st>>>(tR, tL, tR, a);
     count_launch();
     return cudaGetLastError();
   }
@@ -285,9 +300,12 @@ int gemm_mtile(int M) {
   return 16 * ((M + 16 * mt - 1) / (16 * mt));
 }
 
-int gemm_choose_splits(int M, int N, long long K, int max_splits, int num_sms) {
+int gemm_choose_splits(int M, int N, long long K, int max_splits, int num_sms, bool tail) {
   const long long mtiles = (M + gemm_mtile(M) - 1) / gemm_mtile(M);
-  const long long tiles = mtiles * ((N + NT - 1) / NT);
+  const long long tiles = mtiles * (tail && kc_tail_applies(M, N) ? N / NT : (N + NT - 1) / NT);
+#ifdef RS_DEV_KC_S
+  if (tail && kc_tail_applies(M, N)) return std::min(max_splits, RS_DEV_KC_S);  // A/B experiments only
+#endif
   if (tiles >= 2LL * num_sms || max_splits <= 1) return 1;
   int best = 1;
   double best_score = -1.0;
@@ -306,6 +324,54 @@ int gemm_choose_splits(int M, int N, long long K, int max_splits, int num_sms) {
   }
   return best;
 }
+
+bool kc_tail_applies(int M, int N) {
+#if defined(RS_DEV_KC_NO_PWG) || defined(RS_DEV_NO_TAIL)
+  return false;  // the fold lives in the producer-warpgroup kernels only (-DRS_DEV_NO_TAIL: A/B switch)
+#else
+  return M >= 1 && gemm_mtile(M) >= 64 && N > NT && N % NT != 0 && N % NT <= 16;
+#endif
+}
+
+long long kc_tail_elems(int M, int N, int splits) {
+  if (!kc_tail_applies(M, N)) return 0;
+  const int MT = gemm_mtile(M);
+  const long long mtiles = (M + MT - 1) / MT;
+  return static_cast<long long>(splits) * mtiles * (N / NT) * MT * 16;
+}
+
+namespace {
+// out(split s)[m, tail_n0 + c] (op)= sum over the N tiles nt = 0, 1, ... of the tail partials, in
+// that fixed order (bitwise reproducible); one thread per (s, m, c)
+__global__ void kc_tail_reduce_kernel(const GemmArgs a, int S, int mtiles, int MT, int w) {
+  const int ntn = a.tail_ntn;
+  const int mrows = min(a.out.m_store, mtiles * MT);
+  const long long total = static_cast<long long>(S) * mrows * w;
+  for (long long i = blockIdx.x * static_cast<long long>(blockDim.x) + threadIdx.x; i < total;
+       i += static_cast<long long>(gridDim.x) * blockDim.x) {
+    const int c = static_cast<int>(i % w);
+    const int m = static_cast<int>((i / w) % mrows);
+    const int s = static_cast<int>(i / (static_cast<long long>(w) * mrows));
+    const int n = a.tail_n0 + c;
+    if (n >= a.out.n_store) continue;
+    const int mt = m / MT, row = m % MT;
+    const double* tp = a.tail_p + ((static_cast<long long>(s) * mtiles + mt) * ntn * MT + row) * 16 + c;
+    double v = 0.0;
+    for (int nt = 0; nt < ntn; ++nt) v += tp[static_cast<long long>(nt) * MT * 16];
+    gemm_put(a.out.ptr + s * a.out.split_stride + m * a.out.ld_m + n * a.out.ld_n, v, a.out.mode);
+  }
+}
+
+cudaError_t kc_tail_reduce(cudaStream_t st, const GemmArgs& a, int S, int mtiles, int MT, int N) {
+  const int w = N - a.tail_n0;
+  const long long total = static_cast<long long>(S) * std::min(a.out.m_store, mtiles * MT) * w;
+  if (total <= 0) return cudaSuccess;
+  const int blocks = static_cast<int>(std::min<long long>((total + 255) / 256, 148LL * 4));
+  kc_tail_reduce_kernel<<<blocks, 256, 0, st>>>(a, S, mtiles, MT, w);
+  count_launch();
+  return cudaGetLastError();
+}
+}  // namespace
 
 int gemm_nsplit(long long K, int splits) {
   const int s = splits < 1 ? 1 : splits;
@@ -355,6 +421,27 @@ cudaError_t gemm_kc(cudaStream_t st, int M, int N, long long K, const View2D& Lv
     return cudaErrorInvalidValue;
   }
   dim3 grid((N + NT - 1) / NT, (M + MT - 1) / MT, static_cast<unsigned>(nsplit < 1 ? 1 : nsplit));
+  // tail fold: N / 128 full tiles share the last N % 128 columns along K
+  if (!phx.enabled && out.tail_ws && kc_tail_applies(M, N) &&
+      kc_tail_elems(M, N, static_cast<int>(grid.z)) <= out.tail_cap) {
+    CUtensorMap tT;
+    if (!make_tmap(&tT, Rv, 16, 16)) return cudaErrorInvalidValue;
+    grid.x = N / NT;
+    a.tail_p = out.tail_ws;
+    a.tail_n0 = static_cast<int>(grid.x) * NT;
+    a.tail_ntn = static_cast<int>(grid.x);
+    cudaError_t e;
+    switch (mfw) {
+      case 4: e = launch_kc_tail_t<4>(st, grid, tR, tL, tT, a); break;
+      case 5: e = launch_kc_tail_t<5>(st, grid, tR, tL, tT, a); break;
+      case 6: e = launch_kc_tail_t<6>(st, grid, tR, tL, tT, a); break;
+      case 7: e = launch_kc_tail_t<7>(st, grid, tR, tL, tT, a); break;
+      case 8: e = launch_kc_tail_t<8>(st, grid, tR, tL, tT, a); break;
+      default: return cudaErrorInvalidConfiguration;
+    }
+    if (e != cudaSuccess) return e;
+    return kc_tail_reduce(st, a, static_cast<int>(grid.z), static_cast<int>(grid.y), MT, N);
+  }
 #define RS_KC(W)                                                              \
   case W:                                                                     \
     return phx.enabled ? launch_phx_t<W>(st, grid, tR, a)                     \
@@ -466,6 +553,9 @@ SampleRingPlan sample_ring_plan(int N, long long K, int max_splits, int G) {
   p.ntn = (N + NT - 1) / NT;
   double best = -1.0;
   for (int s = 1; s <= max_splits; ++s) {
+#ifdef RS_DEV_RING_S
+    if (s != RS_DEV_RING_S) continue;  // A/B experiments only
+#endif
     const long long kspl = ((K + s - 1) / s + RG_CH - 1) / RG_CH * RG_CH;
     if (kspl < 4 * RG_CH && s > 1) break;  // keep >= 4 chunks (128 stages) per unit
     const int sr = static_cast<int>((K + kspl - 1) / kspl);
@@ -485,8 +575,8 @@ SampleRingPlan sample_ring_plan(int N, long long K, int max_splits, int G) {
 
 size_t sample_ring_bytes(int M, int N, long long K, int max_splits, int G) {
   if (M < 1 || M > 128 || K < 8 * RG_CH) return 0;
-  const SampleRingPlan p = sample_ring_plan(N, K, max_splits, G);
   const int MT = gemm_mtile(M);
+  const SampleRingPlan p = sample_ring_plan(N, K, max_splits, G);
   return static_cast<size_t>(p.ngroups) * RG_R * MT * RG_CH * 8 + 2 * static_cast<size_t>(p.ngroups) * RG_R * 4 + 256;
 }
 
@@ -510,8 +600,10 @@ cudaError_t gemm_sample_ring(cudaStream_t st, int M, int N, long long K, const V
   const int G = num_sms_cached();
   if (M < 1 || M > 128 || K < 8 * RG_CH || !phx.enabled) return cudaErrorNotSupported;
   if (sample_ring_bytes(M, N, K, max_splits, G) > ring_bytes) return cudaErrorNotSupported;
-  const SampleRingPlan p = sample_ring_plan(N, K, max_splits, G);
   const int MT = gemm_mtile(M);
+  // (no tail fold here: measured slower with it -- 34.29 vs 32.22 ms at cfg4, 33.84 with the tail
+  // DMMAs skipped -- the ring couples the members of a group)
+  const SampleRingPlan p = sample_ring_plan(N, K, max_splits, G);
   const int mfw = MT / 16;
   GemmArgs a = make_args(M, N, K, p.S, out);
   a.key.k0 = static_cast<uint32_t>(phx.seed);

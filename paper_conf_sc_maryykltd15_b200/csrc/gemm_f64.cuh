@@ -61,6 +61,12 @@ struct GemmArgs {
   long long omega_row0;  // first Omega row of this tile set (adaptive rounds draw rows [l, l + l_inc))
   int ell;               // number of Omega rows generated (rows >= ell of the tile are zero)
   int tri;       // MC: 0 dense, 1 L lower triangular, 2 R upper triangular (zero blocks skipped)
+  // KC tail fold (kc_tail_applies): the last N % 128 <= 16 columns [tail_n0, N) get no N tile of
+  // their own; the tail_ntn full N tiles of a split share them along K -- tile nt takes the K
+  // stages it = nt, nt + tail_ntn, ... -- and write per-CTA partials (MT x 16 each, index
+  // (split * mtiles + mtile) * tail_ntn + nt) that kc_tail_reduce sums in a fixed order
+  double* tail_p;
+  int tail_n0, tail_ntn;
   unsigned long long nmap;  // persistent MC: N box of warp column wn, slot nb = byte 2 wn + nb
   int l3d, r3d;  // MC: operand tensor map is the 3-D stacked-box form (one TMA per stage), see mc_load
 };
@@ -72,17 +78,19 @@ struct GemmArgs {
 #ifndef RS_KC_NS
 #define RS_KC_NS 4
 #endif
-template <int MFW, bool PHILOX>
+template <int MFW, bool PHILOX, bool TAIL = false>
 struct KCSmem {
   static constexpr int MT = 16 * MFW;
   static constexpr int R_BYTES = NT * KT * 8;
+  static constexpr int T_BYTES = TAIL ? 16 * KT * 8 : 0;  // tail-fold stage: 16 columns of A
+  static constexpr int ACC_BYTES = TAIL ? 4 * MFW * 32 * 16 : 0;  // tail accumulators (MT x 16 doubles)
   static constexpr int L_BYTES_TMA = MT * KT * 8;
   static constexpr int L_BYTES_RAW = PHILOX ? MT * PHX_LD * 8 : L_BYTES_TMA;
   static constexpr int L_BYTES = (L_BYTES_RAW + 1023) / 1024 * 1024;
   // small M (l <= 32): little MMA work per stage, so a deeper ring keeps more of A in flight and
   // lets several generator groups work on different stages at once
   static constexpr int NS = MFW <= 2 ? 8 : (PHILOX ? RS_PHX_NS : RS_KC_NS);
-  static constexpr int TOTAL = 1024 + NS * (R_BYTES + L_BYTES) + 2 * NS * 8;
+  static constexpr int TOTAL = 1024 + NS * (R_BYTES + L_BYTES + T_BYTES) + ACC_BYTES + (TAIL ? 3 : 2) * NS * 8;
 };
 
 // Align the dynamic shared-memory base to 1024 bytes (128B-swizzle atoms) by pointer arithmetic
@@ -137,6 +145,62 @@ RS_DEVINL void kc_store(const double (&acc)[MFW][4][2], const GemmOut& ou, int m
         if (gn < ou.n_store) gemm_put(base + gm * ou.ld_m + gn * ou.ld_n, acc[mf][nf][e], ou.mode);
       }
     }
+  }
+}
+
+// KC tail fold, run by the three otherwise idle warps of the producer warpgroup (warps 9-11;
+// warp 8 lane 0 issues TMA): on the tail stages it = nt, nt + tail_ntn, ... of this CTA (N tile
+// nt) they accumulate D[MT x 16] += L[MT x 16 K] T[16 K x 16], T = the stage's tail columns of A,
+// and release the stage slot themselves (the producer pre-arrives their 3 arrivals on every other
+// stage), so the MMA warps run the plain main loop.  The producer also arrives on tiss[s] when it
+// has issued a tail stage into slot s; a tail warp sleeps on it before it waits on full[s].  That
+// order matters: an mbarrier parity wait cannot tell phase p from p - 2, and a waiter that skips
+// stages could otherwise take the slot's previous, still pending phase for the one it wants --
+// once the stage is issued, its slot's previous phase has completed.  Warp t takes the fragments
+// q = t, t + 3, ... of the 2 MFW x nj grid (M fragment q / nj, tail n8 block q % nj; nj = 1 when
+// the tail is <= 8 columns wide); accumulators in shared memory, one double2 per lane per fragment
+// (tail stages are 1 / tail_ntn of the stages).  The CTA's partial goes to tp: element (tile row,
+// tail column c) at tp[row * 16 + c] (columns 8..15 only when nj = 2).
+template <int MFW, int NS>
+RS_DEVINL void kc_tail_warp(int t, int lane, int nt, int nk, int ntn, int nj, const unsigned char* sL, int l_bytes,
+                            const unsigned char* sT, double2* acc, uint64_t* full, uint64_t* empty, uint64_t* tiss,
+                            double* tp) {
+  const int r = lane >> 2, kk = lane & 3;
+  const int nq = 2 * MFW * nj;
+#pragma unroll 1
+  for (int q = t; q < nq; q += 3) acc[q * 32 + lane] = make_double2(0.0, 0.0);
+  unsigned tpar = 0;  // per slot: parity of its next tiss phase
+#pragma unroll 1
+  for (int it = nt; it < nk; it += ntn) {
+    const int s = it % NS;
+    mbar_wait_sleep(&tiss[s], (tpar >> s) & 1u);
+    tpar ^= 1u << s;
+    mbar_wait_sleep(&full[s], (it / NS) & 1);
+    const unsigned char* Ls = sL + s * l_bytes;
+    const unsigned char* Ts = sT + s * (16 * KT * 8);
+#pragma unroll 1
+    for (int q = t; q < nq; q += 3) {
+      const int mg = q / nj, j = q - mg * nj;
+      double2 c = acc[q * 32 + lane];
+#pragma unroll
+      for (int p = 0; p < 2; ++p) {
+        const double2 a2 = *reinterpret_cast<const double2*>(Ls + kc_pair_off(kc_row(mg >> 1, mg & 1, r), p, kk));
+        const double2 b2 = *reinterpret_cast<const double2*>(Ts + kc_pair_off(kc_row(0, j, r), p, kk));
+        dmma_8x8x4(c.x, c.y, a2.x, b2.x);
+        dmma_8x8x4(c.x, c.y, a2.y, b2.y);
+      }
+      acc[q * 32 + lane] = c;
+    }
+    ring_release_fenced(empty, s, lane);
+  }
+  // fragment element (r, 2kk + e) of n8 block j: tail column 8j + kk + 4e (kc_row of the B column)
+#pragma unroll 1
+  for (int q = t; q < nq; q += 3) {
+    const int mg = q / nj, j = q - mg * nj;
+    const double2 c = acc[q * 32 + lane];
+    double* row = tp + kc_row(mg >> 1, mg & 1, r) * 16 + 8 * j + kk;
+    row[0] = c.x;
+    row[4] = c.y;
   }
 }
 
@@ -229,18 +293,22 @@ __global__ void __launch_bounds__(GEMM_THREADS, 1)
 constexpr int KCP_THREADS = GEMM_THREADS + 128;
 constexpr int MCP_PROD_REGS = 40;
 constexpr int MCP_MMA_REGS = 232;  // 4*32*40 + 8*32*232 = 64512 <= 65536
-template <int MFW>
+template <int MFW, bool TAIL = false>
 __global__ void __launch_bounds__(KCP_THREADS, 1)
     kc_gemm_pwg_kernel(const __grid_constant__ CUtensorMap tmR, const __grid_constant__ CUtensorMap tmL,
-                       const GemmArgs a) {
-  using SM = KCSmem<MFW, false>;
+                       const __grid_constant__ CUtensorMap tmT, const GemmArgs a) {
+  using SM = KCSmem<MFW, false, TAIL>;
   constexpr int MT = SM::MT;
+  constexpr int TAILW = TAIL ? 3 : 0;  // tail warps (kc_tail_warp), counted by every slot release
   extern __shared__ unsigned char smem_raw[];
   unsigned char* smem = align1024(smem_raw);
   unsigned char* sR = smem;
   unsigned char* sL = sR + SM::NS * SM::R_BYTES;
-  uint64_t* full = reinterpret_cast<uint64_t*>(sL + SM::NS * SM::L_BYTES);
+  unsigned char* sT = sL + SM::NS * SM::L_BYTES;  // tail-fold stages (TAIL only)
+  double2* sAcc = reinterpret_cast<double2*>(sT + SM::NS * SM::T_BYTES);
+  uint64_t* full = reinterpret_cast<uint64_t*>(sT + SM::NS * SM::T_BYTES + SM::ACC_BYTES);
   uint64_t* empty = full + SM::NS;
+  uint64_t* tiss = empty + SM::NS;  // tail stage issued into slot s (TAIL only)
 
   const int warp = threadIdx.x >> 5, lane = threadIdx.x & 31;
   const int n0 = blockIdx.x * NT, m0 = blockIdx.y * MT;
@@ -252,7 +320,8 @@ __global__ void __launch_bounds__(KCP_THREADS, 1)
 #pragma unroll
     for (int s = 0; s < SM::NS; ++s) {
       mbar_init(&full[s], 1);
-      mbar_init(&empty[s], NCONS);
+      mbar_init(&empty[s], NCONS + TAILW);
+      if constexpr (TAIL) mbar_init(&tiss[s], 1);
     }
     fence_mbar_init();
   }
@@ -262,14 +331,31 @@ __global__ void __launch_bounds__(KCP_THREADS, 1)
     if (warp == NCONS && lane == 0) {
       tma_prefetch_desc(&tmR);
       tma_prefetch_desc(&tmL);
+      if constexpr (TAIL) tma_prefetch_desc(&tmT);
+      int nxt = blockIdx.x;  // next tail stage of this N tile
       for (int it = 0; it < nk; ++it) {
         const int s = it % SM::NS;
         if (it >= SM::NS) mbar_wait_sleep(&empty[s], ((it / SM::NS) - 1) & 1);
-        mbar_arrive_expect_tx(&full[s], SM::R_BYTES + SM::L_BYTES_TMA);
+        const bool tl = TAIL && it == nxt;
+        mbar_arrive_expect_tx(&full[s], SM::R_BYTES + SM::L_BYTES_TMA + (tl ? SM::T_BYTES : 0));
         const int kc = static_cast<int>(kb + static_cast<long long>(it) * KT);
         tma_load_2d(sR + s * SM::R_BYTES, &tmR, &full[s], kc, n0);
         tma_load_2d(sL + s * SM::L_BYTES, &tmL, &full[s], kc, m0);
+        if constexpr (TAIL) {
+          if (tl) {
+            tma_load_2d(sT + s * SM::T_BYTES, &tmT, &full[s], kc, a.tail_n0);
+            mbar_arrive(&tiss[s]);
+            nxt += a.tail_ntn;
+          } else {
+            mbar_arrive_cnt(&empty[s], TAILW);  // on behalf of the tail warps, which skip this stage
+          }
+        }
       }
+    } else if (TAIL && warp > NCONS) {
+      const long long cta = (static_cast<long long>(blockIdx.z) * gridDim.y + blockIdx.y) * gridDim.x + blockIdx.x;
+      const int nj = a.N - a.tail_n0 > 8 ? 2 : 1;
+      kc_tail_warp<MFW, SM::NS>(warp - NCONS - 1, lane, blockIdx.x, nk, a.tail_ntn, nj, sL, SM::L_BYTES, sT, sAcc,
+                                full, empty, tiss, a.tail_p + cta * MT * 16);
     }
     return;
   }

@@ -18,7 +18,17 @@ struct GemmOutDesc {
   long long ld_m, ld_n, split_stride;
   int m_store, n_store;
   int mode = 0;  // 0: store, 1: subtract from the existing output
+  // KC tail fold (kc_tail_applies): workspace for the per-CTA tail partials (nullptr: no fold)
+  double* tail_ws = nullptr;
+  long long tail_cap = 0;  // doubles
 };
+
+// KC tail fold: when N % 128 is in [1, 16] (n = 5 000: 8; n = 10 000: 16) and the product is
+// DMMA-bound (M tile >= 64 rows), the last N % 128 columns get no 128-wide N tile of their own
+// (which would cost a whole tile's DMMAs for <= 16 useful columns: 2.4 % of the work at
+// n = 5 000); the full N tiles of each K split compute them on every (N / 128)-th K stage instead.
+bool kc_tail_applies(int M, int N);
+long long kc_tail_elems(int M, int N, int splits);  // tail partial doubles for `splits` K splits
 
 struct PhiloxDesc {
   bool enabled;
@@ -62,7 +72,8 @@ cudaError_t gemm_sample_ring(cudaStream_t st, int M, int N, long long K, const V
                              int* nsplit_out);
 int num_sms_cached();
 cudaError_t gemm_syrk(cudaStream_t st, int rows, long long K, const View2D& Xv, const GemmOutDesc& out, int splits);
-int gemm_choose_splits(int M, int N, long long K, int max_splits, int num_sms);
+// tail: the KC tail fold will be used (N tiles = N / 128)
+int gemm_choose_splits(int M, int N, long long K, int max_splits, int num_sms, bool tail = false);
 int gemm_nsplit(long long K, int splits);   // splits actually launched for a requested count
 int gemm_mtile(int M);   // rows per CTA tile used for M
 

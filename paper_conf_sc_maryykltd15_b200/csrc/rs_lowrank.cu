@@ -46,8 +46,9 @@ struct Layout {
   int smax;          // max split-K partial tiles of an l x n product
   long long part_elems;
   size_t off_B, off_B0, off_Bt, off_B1, off_C, off_C1, off_part, off_G, off_Rf, off_Linv, off_cholw, off_Rho, off_Rhat,
-      off_T, off_Q1, off_R1, off_R2, off_Rbar, off_perm, off_info, off_qr, off_gaps, off_ring;
-  size_t ring_bytes;  // Omega chunk ring of the sample GEMM (0: the cluster kernel generates in smem)
+      off_T, off_Q1, off_R1, off_R2, off_Rbar, off_perm, off_info, off_qr, off_gaps, off_ring, off_tail;
+  size_t ring_bytes;
+  long long tail_elems;  // KC tail-fold partials of the l x n products (kc_tail_applies), smax splits  // Omega chunk ring of the sample GEMM (0: the cluster kernel generates in smem)
   size_t total;
 };
 
@@ -98,6 +99,8 @@ Layout plan(long long m_local, long long n, int k, int p) {
   // cluster kernel if the ring does not fit)
   L.ring_bytes = sample_ring_bytes(L.lp, static_cast<int>(n), m_local, L.smax, 148);
   L.off_ring = take(L.ring_bytes);
+  L.tail_elems = kc_tail_elems(L.lp, static_cast<int>(n), L.smax);
+  L.off_tail = take(static_cast<size_t>(L.tail_elems) * 8);
   L.total = off + 1024;
   return L;
 }
@@ -120,6 +123,7 @@ struct rs_lowrank_s {
   Layout L;
   char* ws;
   void* ring;
+  double* tailp;  // KC tail-fold partials (L.tail_elems doubles)
   double *B, *B0, *Bt, *B1, *C, *C1, *part, *G, *Rf, *Linv, *cholw, *Rho, *Rhat, *T, *Q1, *R1, *R2, *Rbar, *gaps;
   int64_t* perm;
   int* info;
@@ -433,6 +437,8 @@ rs_status_t enqueue_sample(rs_lowrank_t h, const double* A, long long lda) {
       Scope sc(h, "gemm_sample", 2.0 * h->ell * static_cast<double>(h->m_local) * h->n);
       View2D Av{A, h->m_local, h->n, lda};
       GemmOutDesc out{h->part, 1, L.lp, lxn, L.lp, static_cast<int>(h->n)};
+      out.tail_ws = h->tailp;
+      out.tail_cap = L.tail_elems;
       PhiloxDesc phx{true, h->seed, 0u, h->row_offset, h->ell};
       // Omega generated once per K split into an L2 ring shared by all N tiles; the cluster kernel
       // (Omega generated in shared memory per pair of N tiles) when the ring does not apply
@@ -461,13 +467,15 @@ rs_status_t gemm_b(rs_lowrank_t h, const double* A, long long lda, const double*
   const long long ml = h->m_local, n = h->n;
   const long long lxn = static_cast<long long>(L.lp) * n;
   if (ml > 0) {
-    const int splits = gemm_choose_splits(L.lp, static_cast<int>(n), ml, max_splits_for(h, lxn), h->sms);
+    const int splits = gemm_choose_splits(L.lp, static_cast<int>(n), ml, max_splits_for(h, lxn), h->sms, true);
     const int ns = gemm_nsplit(ml, splits);
     {
       Scope sc(h, "gemm_power_b", 2.0 * h->ell * static_cast<double>(ml) * n);
       View2D Cv{Csrc, ml, L.lp, L.ldc};
       View2D Av{A, ml, n, lda};
       GemmOutDesc out{h->part, 1, L.lp, lxn, L.lp, static_cast<int>(n)};
+      out.tail_ws = h->tailp;
+      out.tail_cap = L.tail_elems;
       PhiloxDesc nophx{false, 0, 0, 0, 0};
       RS_CUDA(h, gemm_kc(h->st, L.lp, static_cast<int>(n), ml, Cv, Av, nophx, out, splits));
     }
@@ -828,6 +836,7 @@ rs_status_t rs_lowrank_create(rs_lowrank_t* out, int64_t m_global, int64_t m_loc
   h->B = D(L.off_B);
   h->B0 = D(L.off_B0);
   h->ring = base + L.off_ring;
+  h->tailp = reinterpret_cast<double*>(base + L.off_tail);
   h->Bt = D(L.off_Bt);
   h->B1 = D(L.off_B1);
   h->C = D(L.off_C);

@@ -98,6 +98,25 @@ def test_sample_ring_shapes(m, n, k, p):
     assert rel(B, OPL.sample(A, k + p, SEED)) <= 1e-13
 
 
+@pytest.mark.parametrize("m,n,k,p", [
+    (60000, 1032, 100, 10),   # n % 128 = 8 (cfg2/cfg4's tail width), l = 110: 8 full N tiles share it
+    (50000, 1036, 60, 4),     # tail of 12 columns: the second tail n8 block is ragged; l = 64 (MFW 4)
+    (40000, 1040, 120, 8),    # tail of 16 (cfg3's width), l = 128 (MFW 8)
+    (3000, 1288, 100, 10),    # K = 3 000 rows: units with fewer K stages than N tiles (some get no tail stage)
+])
+def test_sample_narrow_last_tile(m, n, k, p):
+    """Ring sample GEMM with a last N tile of 8 / 12 / 16 columns (the widths the KC tail fold takes
+    in B := C~ A; the ring kernel keeps its own narrow tile) -- B = Omega A against the oracle."""
+    rng = np.random.default_rng(m + 7 * n)
+    A = np.asfortranarray(rng.standard_normal((m, n)))
+    B = _sample_gpu(A, k, p)
+    Bo = OPL.sample(A, k + p, SEED)
+    assert rel(B, Bo) <= 1e-13
+    # the tail columns on their own (an error confined to them would hide in the global norm)
+    t0 = (n // 128) * 128
+    assert rel(B[:, t0:], Bo[:, t0:]) <= 1e-13
+
+
 def _sample_gpu(A, k, p):
     m, n = A.shape
     h = rs.create(m, m, 0, n, k, p, SEED)
@@ -256,6 +275,12 @@ def test_pipeline_cfg1(q):
     (4000, 500, 150, 10, 0, "exp-k"),     # l = 160 > 128: two M tiles, k > 128
     (6000, 900, 400, 10, 1, "exp-k"),     # cfg5's largest k: l = 410, four M tiles, Cholesky n > 128
     (8000, 1000, 200, 20, 2, "power"),    # cfg3 law and (k, p, q) at reduced m, n
+    # KC tail fold in B := C~ A (n % 128 = 8 / 12 / 16: the last N % 128 columns computed by the
+    # producer warpgroup's tail warps on every (n / 128)-th K stage); the last with few K stages
+    # per split (N tiles without a tail stage)
+    (30000, 1032, 100, 10, 1, "exp-k"),
+    (20000, 1292, 50, 14, 2, "power"),
+    (2500, 1040, 100, 10, 1, "exp-k"),
     # m / 128 >= 8 x 148 tiles: the short-K applies (C1 = L^-1 C, Q1 = X R^-1) run on the persistent
     # MC kernel (resident operand, balanced triangular fragment / box sets)
     (160000, 300, 50, 10, 1, "exp-k"),

@@ -36,6 +36,10 @@ def test_sanitizer_clean(tool):
             "50", "--p", "10", "--q", "1"]
     r = subprocess.run(cmd, capture_output=True, text=True, timeout=1500, cwd=ROOT)
     out = r.stdout + r.stderr
+    if r.returncode == 86 and "closed" in out:
+        # the GPU pool's compute-sanitizer wrapper refuses to run (operator decision); the r02
+        # runs of this test before the closure are in profiles/r02_summary.md
+        pytest.skip("compute-sanitizer is closed on this GPU pool: " + out.strip().splitlines()[0][:200])
     assert r.returncode == 0, out[-4000:]
     assert "ok " in out, out[-2000:]
     m = re.search(r"(ERROR|RACECHECK) SUMMARY: (\d+)", out)
