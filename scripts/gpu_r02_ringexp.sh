@@ -1,8 +1,8 @@
 #!/bin/bash
-# r02 experiment: does the ring sample kernel get faster with N / 128 units per split (tail columns
-# dropped -- timing only) ?  Same box A/B, cfg4 and cfg2, several split counts.
+# r02 experiment: ring sample kernel time against its split count (rounds of the persistent grid),
+# with the narrow 40th tile (default) and with it dropped (-DRS_DEV_RING_DROP_TAIL: timing only)
 mkdir -p gpurun_out
-for flags in "" "-DRS_DEV_RING_DROP_TAIL" "-DRS_DEV_RING_DROP_TAIL -DRS_DEV_RING_S=34" "-DRS_DEV_RING_DROP_TAIL -DRS_DEV_RING_S=15" ""; do
+for flags in "" "-DRS_DEV_RING_S=11" "-DRS_DEV_RING_S=22" "-DRS_DEV_RING_S=7" "-DRS_DEV_RING_DROP_TAIL -DRS_DEV_RING_S=11" "-DRS_DEV_RING_DROP_TAIL -DRS_DEV_RING_S=15" "-DRS_DEV_RING_DROP_TAIL -DRS_DEV_RING_S=30" ""; do
   export RS_EXTRA_NVCC_FLAGS="$flags"
   python __graft_entry__.py build > gpurun_out/build.log 2>&1 || { tail -30 gpurun_out/build.log; exit 1; }
   for c in cfg4 cfg2; do
