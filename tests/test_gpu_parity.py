@@ -421,6 +421,43 @@ def test_pipeline_is_bitwise_deterministic():
     np.testing.assert_array_equal(g1["perm"], g2["perm"])
 
 
+@pytest.mark.parametrize("m,n,k,p,q", [(20000, 1032, 60, 10, 1), (3000, 600, 40, 10, 2)])
+def test_power_of_two_scaling_is_exact(m, n, k, p, q):
+    """SURVEY 8(c) invariance: A -> 4 A gives B -> 4 B, R -> 4 R bit for bit and Q, T, perm
+    unchanged -- every step (split-K and tail-fold sums, CholQR2, QRCP, TRSM) is homogeneous and
+    scaling by a power of two is exact in IEEE arithmetic (sqrt of 16^s exact, no over/underflow
+    here), so any stray constant, mis-scaled shift or wrong term in a kernel would show."""
+    A, _ = make_matrix(m, n, "exp-k", k, seed=m + n)
+    g1 = _run_gpu(A, k, p, q)
+    g4 = _run_gpu(np.asfortranarray(4.0 * A), k, p, q)
+    np.testing.assert_array_equal(g4["perm"], g1["perm"])
+    np.testing.assert_array_equal(g4["B"], 4.0 * g1["B"])
+    np.testing.assert_array_equal(g4["R"], 4.0 * g1["R"])
+    np.testing.assert_array_equal(g4["Q"], g1["Q"])
+    np.testing.assert_array_equal(g4["T"], g1["T"])
+
+
+def test_column_permutation_permutes_pivots():
+    """SURVEY 8(c) invariance: A -> A Pi (tie-free) selects the same columns, in Pi's labels, with
+    the same R up to rounding (columns moved into / out of the 8-column KC tail fold are summed in
+    another order, so the comparison is normwise, not bitwise)."""
+    m, n, k, p, q = 20000, 1032, 60, 10, 1
+    A, _ = make_matrix(m, n, "exp-k", k, seed=77)
+    pi = np.random.default_rng(3).permutation(n)
+    g1 = _run_gpu(A, k, p, q)
+    g2 = _run_gpu(np.asfortranarray(A[:, pi]), k, p, q)
+    np.testing.assert_array_equal(pi[g2["perm"][:k]], g1["perm"][:k])
+    # R's first k columns (the pivot columns) in pivot order; the rest compared after undoing pi
+    assert rel(g2["R"][:, :k], g1["R"][:, :k]) <= 1e-12
+    inv = np.empty(n, dtype=np.int64)
+    inv[pi] = np.arange(n)
+    R1 = np.zeros_like(g1["R"])
+    R2 = np.zeros_like(g2["R"])
+    R1[:, g1["perm"]] = g1["R"]
+    R2[:, pi[g2["perm"]]] = g2["R"]
+    assert rel(R2, R1) <= 1e-12
+
+
 def test_omega_identity_special_case_is_truncated_qp3():
     """set_sample(B := A) with l = m, q = 0: pivots = LAPACK dgeqp3's; |R| rows = QP3's."""
     import scipy.linalg as sla
