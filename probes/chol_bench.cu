@@ -7,6 +7,17 @@
 
 namespace rs {
 void count_launch() {}
+// chol.cu's 2 x 2 block path (n > 128) calls these; the probe only times n <= 128
+cudaError_t small_gemm(cudaStream_t, int, int, int, const double*, long long, long long, const double*, long long,
+                       long long, double*, long long, long long, bool, double) {
+  return cudaErrorNotSupported;
+}
+cudaError_t copy_2d(cudaStream_t, const double*, long long, double*, long long, long long, long long) {
+  return cudaErrorNotSupported;
+}
+cudaError_t ensure_func_attr(const void* fn, cudaFuncAttribute attr, int value) {
+  return cudaFuncSetAttribute(fn, attr, value);
+}
 }  // namespace rs
 
 int main() {
@@ -36,20 +47,22 @@ int main() {
     const int np = (n + 3) / 4 * 4;
     const size_t smem = rs::ct_smem_doubles(np) * 8;
     for (auto fn : {rs::chol_tile_kernel<1, 256>, rs::chol_tile_kernel<1, 512>, rs::chol_tile_kernel<1, 832>,
-                    rs::chol_tile_kernel<1, 1024>})
+                    rs::chol_tile_kernel<1, 1024>, rs::chol_tile_kernel<2, 416>, rs::chol_tile_kernel<2, 512>})
       cudaFuncSetAttribute(fn, cudaFuncAttributeMaxDynamicSharedMemorySize, rs::ct_smem_doubles(128) * 8);
     const int tiles = (np / 4) * (np / 4 + 1);
-    for (int nthr : {256, 512, 832, 1024}) {
-      if (tiles > nthr) continue;
+    for (int nthr : {256, 512, 832, 1024, -416, -512}) {  // negative: two tiles per thread
+      if (tiles > (nthr < 0 ? -2 * nthr : nthr)) continue;
       cudaEvent_t e0, e1;
       cudaEventCreate(&e0);
       cudaEventCreate(&e1);
       const int reps = 200;
       auto launch = [&] {
-        if (nthr == 256) rs::chol_tile_kernel<1, 256><<<1, 256, smem>>>(dG, n, n, dR, npad, dL, npad, info, 5, npad);
-        else if (nthr == 512) rs::chol_tile_kernel<1, 512><<<1, 512, smem>>>(dG, n, n, dR, npad, dL, npad, info, 5, npad);
-        else if (nthr == 832) rs::chol_tile_kernel<1, 832><<<1, 832, smem>>>(dG, n, n, dR, npad, dL, npad, info, 5, npad);
-        else rs::chol_tile_kernel<1, 1024><<<1, 1024, smem>>>(dG, n, n, dR, npad, dL, npad, info, 5, npad);
+        if (nthr == 256) rs::chol_tile_kernel<1, 256><<<1, 256, smem>>>(dG, n, n, dR, npad, dL, npad, info, 5, npad, 0);
+        else if (nthr == 512) rs::chol_tile_kernel<1, 512><<<1, 512, smem>>>(dG, n, n, dR, npad, dL, npad, info, 5, npad, 0);
+        else if (nthr == 832) rs::chol_tile_kernel<1, 832><<<1, 832, smem>>>(dG, n, n, dR, npad, dL, npad, info, 5, npad, 0);
+        else if (nthr == 1024) rs::chol_tile_kernel<1, 1024><<<1, 1024, smem>>>(dG, n, n, dR, npad, dL, npad, info, 5, npad, 0);
+        else if (nthr == -416) rs::chol_tile_kernel<2, 416><<<1, 416, smem>>>(dG, n, n, dR, npad, dL, npad, info, 5, npad, 0);
+        else rs::chol_tile_kernel<2, 512><<<1, 512, smem>>>(dG, n, n, dR, npad, dL, npad, info, 5, npad, 0);
       };
       for (int r = 0; r < 10; ++r) launch();
       cudaEventRecord(e0);
