@@ -76,8 +76,9 @@ typedef int (*rs_allreduce_fn)(void* ctx, double* buf, int64_t count, void* cuda
 
 /* Bytes of device workspace rs_lowrank_create needs for these sizes (no device access): the
  * sample B and its copies, C and C1 (l x m_local), split-K partials (<= 1 GiB), the small factors,
- * QRCP work, Q1 (m_local x k) and -- for l <= 128 and m_local >= 2048 -- the ring of Omega chunks
- * of the sample GEMM (~43 MB at m = 1e6, n = 5 000, l = 110).  cfg4: 2.96 GB.                 */
+ * QRCP work, Q1 (m_local x k), -- for l <= 128 and m_local >= 2048 -- the ring of Omega chunks
+ * of the sample GEMM (~43 MB at m = 1e6, n = 5 000, l = 110) and -- when n mod 128 is 1..16 --
+ * the per-tile partials of the KC tail fold (~36 MB at cfg4).  cfg4: 2.99 GB.                  */
 RS_API size_t rs_lowrank_workspace_bytes(int64_t m_local, int64_t n, int32_t k, int32_t p, int32_t nranks);
 
 /* Create a handle.
