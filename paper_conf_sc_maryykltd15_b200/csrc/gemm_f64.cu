@@ -307,6 +307,29 @@ int gemm_choose_splits(int M, int N, long long K, int max_splits, int num_sms, b
   if (tail && kc_tail_applies(M, N)) return std::min(max_splits, RS_DEV_KC_S);  // A/B experiments only
 #endif
   if (tiles >= 2LL * num_sms || max_splits <= 1) return 1;
+#ifndef RS_DEV_KC_SPLITS_OLD
+  if (tail && kc_tail_applies(M, N)) {
+    // B := C~ A with the tail fold: a time model in K rows per CTA, fitted to the measured split
+    // sweeps (cfg4: S = 15 / 34 / 53 -> 31.37 / 31.15 / 31.10 ms; cfg2: 1.625 / 1.643 / 1.673 ms):
+    // waves * (rows per split + ~48 rows of per-CTA start-up and epilogue) + the split-K reduce
+    // (one l x N partial per split, ~N / 800 rows' worth of time each)
+    int bs = 1;
+    double bc = 1e300;
+    for (int s = 1; s <= max_splits; ++s) {
+      const long long chunk = ((K + s - 1) / s + KT - 1) / KT * KT;
+      if (chunk < 8 * KT && s > 1) break;
+      const long long real_s = (K + chunk - 1) / chunk;
+      const long long waves = (tiles * real_s + num_sms - 1) / num_sms;
+      const double cost = static_cast<double>(waves) * static_cast<double>(chunk + 48) +
+                          static_cast<double>(real_s) * static_cast<double>(N) / 800.0;
+      if (cost < bc - 1e-9) {
+        bc = cost;
+        bs = static_cast<int>(real_s);
+      }
+    }
+    return bs;
+  }
+#endif
   int best = 1;
   double best_score = -1.0;
   for (int s = 1; s <= max_splits; ++s) {
