@@ -574,9 +574,6 @@ cudaError_t gemm_tsa(cudaStream_t st, long long m, int k, const View2D& Xv, cons
 SampleRingPlan sample_ring_plan(int N, long long K, int max_splits, int G) {
   SampleRingPlan p{};
   p.ntn = (N + NT - 1) / NT;
-#ifdef RS_DEV_RING_DROP_TAIL
-  if (N > NT && N % NT <= 16) p.ntn = N / NT;  // timing experiment only: the last N % 128 columns are NOT computed
-#endif
   double best = -1.0;
   for (int s = 1; s <= max_splits; ++s) {
 #ifdef RS_DEV_RING_S

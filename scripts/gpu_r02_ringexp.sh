@@ -1,6 +1,8 @@
 #!/bin/bash
 # r02 experiment: ring sample kernel time against its split count (rounds of the persistent grid),
-# with the narrow 40th tile (default) and with it dropped (-DRS_DEV_RING_DROP_TAIL: timing only)
+# with the narrow 40th tile (default) and with it dropped (-DRS_DEV_RING_DROP_TAIL, a timing-only
+# switch that skipped the tail columns; removed from the library after the experiment, see
+# profiles/r02_ring_splits.jsonl)
 mkdir -p gpurun_out
 for flags in "" "-DRS_DEV_RING_S=11" "-DRS_DEV_RING_S=22" "-DRS_DEV_RING_S=7" "-DRS_DEV_RING_DROP_TAIL -DRS_DEV_RING_S=11" "-DRS_DEV_RING_DROP_TAIL -DRS_DEV_RING_S=15" "-DRS_DEV_RING_DROP_TAIL -DRS_DEV_RING_S=30" ""; do
   export RS_EXTRA_NVCC_FLAGS="$flags"
